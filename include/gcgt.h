@@ -1,0 +1,138 @@
+/*
+ * gcgt.h — C ABI of the B200-native GCGT hot path (Sha, Li, Tan, "GPU-based Graph Traversal on Compressed
+ * Graphs", SIGMOD '19).  Library: paper_conf_sigmod_shalt19_b200/libgcgt.so (sm_100a CUDA + host C++).
+ *
+ * The boundary follows the paper's problem statement (§3.2, Fig. 3): the CPU compresses the
+ * graph into the compressed graph representation (CGR), the CGR is moved to device memory without being
+ * decompressed there, and the CPU issues traversal queries that run on the CGR.  Application outputs are
+ * per-vertex labels (§6 :1137-1286, Fig. 7).  The exact bit layout is FORMAT.md (rules R1-R19).
+ *
+ * Conventions (every entry point):
+ *  - Plain C types only; no C++ or torch types cross the boundary; no exception escapes.
+ *  - Ownership: the caller owns every buffer it passes in or out.  The library owns gcgt_cgr / gcgt_graph
+ *    objects until gcgt_cgr_free / gcgt_unload.
+ *  - Errors: a gcgt_status is returned; on anything but GCGT_OK, gcgt_last_error() returns a thread-local
+ *    message.  Inputs are validated before any allocation; on error no output buffer is partially trusted.
+ *  - Synchronisation: every call is synchronous with respect to the graph's stream on return (outputs are
+ *    complete and visible to the host or the device).
+ *  - Vertex ids are uint32 (n <= 2^32 - 1); bit offsets and arc counts are uint64.
+ *  - There is no CPU fallback: gcgt_load / gcgt_bfs / gcgt_cc / gcgt_bc fail with GCGT_ECUDA when no CUDA
+ *    device is usable.
+ */
+#ifndef GCGT_H
+#define GCGT_H
+
+#include <stdint.h>
+
+#ifdef __cplusplus
+extern "C" {
+#endif
+
+typedef enum {
+    GCGT_OK = 0,
+    GCGT_EINVAL = -1,     /* bad argument / parameter (e.g. min_interval_len == 1, zeta_k outside 1..5)      */
+    GCGT_EUNSORTED = -2,  /* a CSR row is not strictly increasing (FORMAT.md R6)                              */
+    GCGT_ERANGE = -3,     /* a column id or a source >= n                                                     */
+    GCGT_ESEGLEN = -4,    /* a residual segment cannot hold even one residual (FORMAT.md R19)                */
+    GCGT_ENOMEM = -5,     /* host or device allocation failed                                                 */
+    GCGT_ECUDA = -6,      /* CUDA runtime error, or no usable device                                          */
+    GCGT_ENCCL = -7,      /* NCCL error (multi-GPU)                                                            */
+    GCGT_EFORMAT = -8     /* corrupt or inconsistent CGR (file or view)                                        */
+} gcgt_status;
+
+/* Input graph in CSR (Fig. 1): out-arcs of u are cols[row_offsets[u] .. row_offsets[u+1]).
+ * Host memory, caller-owned.  m = row_offsets[n].  Rows must be strictly increasing with ids < n. */
+typedef struct {
+    uint64_t n;
+    const uint64_t* row_offsets; /* n + 1 entries */
+    const uint32_t* cols;        /* row_offsets[n] entries */
+} gcgt_csr;
+
+/* CGR parameters (Table 2; App. D sweeps them). */
+typedef struct {
+    uint32_t min_interval_len;     /* 0 = no intervals ("inf", Fig. 12); otherwise >= 2.  Paper default 4.          */
+    uint32_t residual_segment_len; /* residual segment length in BYTES (FORMAT.md R15); 0 = unsegmented ("inf").
+                                      Paper default 32.                                                               */
+    uint32_t zeta_k;               /* 1 = gamma code, 2..5 = the paper's zeta_k (App. B, Table 3).  Paper default 3. */
+} gcgt_params;
+
+/* Per-call statistics (optional; pass NULL to skip). */
+typedef struct {
+    uint32_t iterations;        /* BFS: levels expanded; CC: hook iterations; BC: sources processed             */
+    uint32_t reserved;
+    uint64_t vertices_expanded; /* frontier vertices whose CGR record was decoded (summed over passes)         */
+    uint64_t arcs_decoded;      /* neighbour ids produced by decoding (summed over passes)                     */
+    uint64_t cgr_bits_decoded;  /* CGR bits of the records decoded (algorithmic CGR traffic)     */
+    double device_ms;           /* device time of the call (CUDA events on the graph's stream)                 */
+} gcgt_stats;
+
+typedef struct gcgt_cgr gcgt_cgr;     /* host CGR: canonical bytes + bit_offsets + params; library-owned     */
+typedef struct gcgt_graph gcgt_graph; /* device-resident CGR and work buffers; library-owned                  */
+
+/* ---- Graph Compression Module (CPU; §3.1 :353-411, App. C :2097-2112, §5.2 :1092-1136, Fig. 3) ------------------
+ * gcgt_encode: CSR -> CGR, bit-exact with FORMAT.md.  Multi-threaded (OpenMP).  *out receives a new object.
+ * Errors: EINVAL (params), EUNSORTED / ERANGE (input rows), ESEGLEN (segment too short), ENOMEM. */
+gcgt_status gcgt_encode(const gcgt_csr* csr, const gcgt_params* params, gcgt_cgr** out);
+
+/* Read-only view of a CGR: bytes (ceil(nbits/8), MSB-first, R1), nbits, bit_offsets (n + 1 entries, R2),
+ * n, params.  Pointers stay valid until gcgt_cgr_free.  Any output pointer may be NULL. */
+gcgt_status gcgt_cgr_view(const gcgt_cgr* cgr, const uint8_t** bytes, uint64_t* nbits,
+                          const uint64_t** bit_offsets, uint64_t* n, gcgt_params* params);
+
+/* Builds a CGR object by copying caller arrays (e.g. a CGR produced elsewhere).  Checks bit_offsets is
+ * non-decreasing with bit_offsets[n] == nbits; returns EFORMAT otherwise. */
+gcgt_status gcgt_cgr_from_arrays(uint64_t n, const uint8_t* bytes, uint64_t nbits, const uint64_t* bit_offsets,
+                                 const gcgt_params* params, gcgt_cgr** out);
+
+/* Checkpoint / resume of the offline artefact (the CGR is the only persistent state, Fig. 3 :438-454). */
+gcgt_status gcgt_cgr_save(const gcgt_cgr* cgr, const char* path);
+gcgt_status gcgt_cgr_open(const char* path, gcgt_cgr** out);
+void gcgt_cgr_free(gcgt_cgr* cgr);
+
+/* ---- Device residency (§3.2 :469-479: "directly move the compressed adjacency lists to GPUs") -------------------- */
+typedef struct {
+    int device;        /* CUDA device ordinal                                                                       */
+    void* stream;      /* cudaStream_t to run on; NULL = a library-created non-blocking stream                      */
+    int rank, nranks;  /* 1-D vertex-range partition (multi-GPU).  nranks <= 1: single GPU (rank ignored)           */
+    void* nccl_comm;   /* ncclComm_t for nranks > 1 (created by the caller, e.g. from a unique id broadcast over
+                          torch.distributed); NULL for a single GPU                                                 */
+} gcgt_load_opts;
+
+/* Copies the CGR (bytes + bit_offsets) to the device and allocates the traversal work buffers.  With nranks > 1
+ * each rank keeps only the records of its owned vertex range (balanced by CGR bits; records are self-contained,
+ * so slicing is a bit copy) plus replicated n-bit bitmaps.  opts may be NULL (device 0, own stream). */
+gcgt_status gcgt_load(const gcgt_cgr* cgr, const gcgt_load_opts* opts, gcgt_graph** out);
+void gcgt_unload(gcgt_graph* g);
+
+/* Owned vertex range [*lo, *hi) of this rank (whole [0, n) on a single GPU). */
+gcgt_status gcgt_graph_range(const gcgt_graph* g, uint64_t* lo, uint64_t* hi);
+
+/* ---- Traversal queries (§4-§6; Fig. 7) ------------------------------------------------------------------------ */
+/* Output placement flag for the query calls below. */
+#define GCGT_OUT_HOST 0   /* output pointer is host memory (pageable or pinned); the library copies D2H       */
+#define GCGT_OUT_DEVICE 1 /* output pointer is device memory on the graph's device                             */
+
+/* BFS from `source` over out-arcs (Fig. 7(b)).  levels[v] = hop distance, -1 if unreached; n entries.
+ * Errors: ERANGE (source >= n), ECUDA, ENCCL. */
+gcgt_status gcgt_bfs(gcgt_graph* g, uint32_t source, int32_t* levels, int out_placement, gcgt_stats* stats);
+
+/* Weakly connected components (Fig. 7(c): hooking + pointer jumping, Soman et al. [42]).  labels[v] = the
+ * minimum vertex id in v's component (every arc joins both endpoints); n entries. */
+gcgt_status gcgt_cc(gcgt_graph* g, uint32_t* labels, int out_placement, gcgt_stats* stats);
+
+/* Betweenness centrality from k sources (host array; duplicates counted), Brandes' dependency accumulation
+ * (Fig. 7(d), §6 :1272-1284): bc[v] = sum_s delta_s(v), v != s; unnormalised, fp64; n entries.
+ * Errors: ERANGE (a source >= n). */
+gcgt_status gcgt_bc(gcgt_graph* g, const uint32_t* sources, uint32_t k, double* bc, int out_placement,
+                    gcgt_stats* stats);
+
+/* Thread-local message for the last non-OK status returned on this thread ("" if none). */
+const char* gcgt_last_error(void);
+
+/* Library / build identification string (compile target, e.g. "gcgt sm_100a"). */
+const char* gcgt_version(void);
+
+#ifdef __cplusplus
+}
+#endif
+#endif /* GCGT_H */

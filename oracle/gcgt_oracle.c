@@ -179,21 +179,29 @@ static int encode_vertex(bitbuf *bb, uint64_t u, const uint32_t *adj, uint64_t d
         }
         return ORC_OK;
     }
-    /* R18 packing: first decide every segment, then write segNum and the segments (R14, R16). */
+    /* R18 packing: first decide every segment, then write segNum and the segments (R14, R16).
+     * L(rest from i) = len(VLC(cnt+1)) + len(VLC(sm(r_i - u)+1)) + sum of the gap codes after r_i; the gap-code
+     * sum is a suffix sum G[i] so that each test is O(1) (hub lists have millions of residuals). */
     uint64_t segBits = 8ull * segLen;
     uint64_t nseg = 0, placed = 0;
     uint64_t *segcnt = (uint64_t *)malloc(sizeof(uint64_t) * (nres + 1));
-    if (!segcnt) return ORC_ENOMEM;
+    uint64_t *G = (uint64_t *)malloc(sizeof(uint64_t) * (nres + 1));
+    if (!segcnt || !G) { free(segcnt); free(G); return ORC_ENOMEM; }
+    if (nres) G[nres - 1] = 0;
+    for (uint64_t t = nres - 1; nres && t-- > 0;) G[t] = G[t + 1] + orc_vlc_len(k, (uint64_t)(res[t + 1] - res[t]));
     while (placed < nres) {
         uint64_t rest = nres - placed;
-        if (seg_body_len(k, u, res + placed, rest) <= 2 * segBits) {   /* last segment, unpadded */
+        uint64_t Lrest = orc_vlc_len(k, rest + 1) + orc_vlc_len(k, sm((int64_t)res[placed] - (int64_t)u) + 1) +
+                         G[placed];
+        if (Lrest <= 2 * segBits) {                                    /* last segment, unpadded */
             segcnt[nseg++] = rest; placed = nres; break;
         }
         uint64_t c = 0;                                                /* longest prefix fitting segBits */
         while (c + 1 <= rest && seg_body_len(k, u, res + placed, c + 1) <= segBits) c++;
-        if (c == 0) { free(segcnt); return ORC_ESEGLEN; }              /* R19 */
+        if (c == 0) { free(segcnt); free(G); return ORC_ESEGLEN; }     /* R19 */
         segcnt[nseg++] = c; placed += c;
     }
+    free(G);
     vlc_put(bb, k, nseg + 1);                                          /* R14: segNum (+1) */
     placed = 0;
     for (uint64_t s = 0; s < nseg; s++) {
