@@ -1,0 +1,319 @@
+"""bench.py — BFS GTEPS on the compressed graph (BASELINE.json metric) for the B200 GCGT path.
+
+    python bench.py [--gpus N] [--steps K] [--warmup W] [--config c2] [--impl gcgt|reference]
+    torchrun --nproc-per-node N bench.py --gpus N ...      (one process per GPU)
+
+A step is one BFS query (the whole §8(a) path: frontier management, header / interval / residual-segment decode,
+filter, contraction) from a seeded root over the device-resident CGR of the configuration's synthetic graph.
+Default workload = BASELINE.json configs[1] (uk-2002-like web graph, 18.5M vertices) on 1 B200.
+With N > 1 ranks every rank runs its own stream of BFS queries on a full replica ("weak" scaling over independent
+queries; no data-path collective); value = all ranks' traversed edges / max-over-ranks time.
+`--impl reference` times the oracle (oracle/, plain C, 1 thread) on the same workload (rank 0 only).
+Prints ONE JSON line on rank 0.
+"""
+from __future__ import annotations
+
+import argparse
+import json
+import os
+import subprocess
+import sys
+import time
+
+import numpy as np
+
+ROOT = os.path.dirname(os.path.abspath(__file__))
+sys.path.insert(0, ROOT)
+
+METRIC = "BFS GTEPS on compressed graph (1/2/4/8 B200); % HBM roofline on CGR bytes"
+PEAKS_PATH = os.path.join(ROOT, "MEASURED_PEAKS.json")
+FALLBACK_HBM_GBS = 6650.0  # B200_PROFILING.md fallback, used only if MEASURED_PEAKS.json is absent
+
+
+def parse():
+    ap = argparse.ArgumentParser()
+    ap.add_argument("--gpus", type=int, default=1)
+    ap.add_argument("--steps", type=int, default=16)
+    ap.add_argument("--warmup", type=int, default=3)
+    ap.add_argument("--config", default="c2")
+    ap.add_argument("--impl", default="gcgt", choices=["gcgt", "reference"])
+    ap.add_argument("--roots", type=int, default=16)
+    ap.add_argument("--no-cpu-baseline", action="store_true")
+    ap.add_argument("--no-e2e", action="store_true")
+    return ap.parse_args()
+
+
+def hbm_peak():
+    try:
+        with open(PEAKS_PATH) as f:
+            pk = json.load(f)
+        return float(pk["hbm_gbs"]), "measured (MEASURED_PEAKS.json hbm_gbs, copy read+write)"
+    except Exception:
+        return FALLBACK_HBM_GBS, "fallback (B200_PROFILING.md)"
+
+
+class ClockSampler:
+    """nvidia-smi clocks + throttle reasons sampled during the timed region."""
+
+    Q = ("index,clocks.sm,clocks.max.sm,power.draw,clocks_event_reasons.active,clocks_event_reasons.hw_slowdown,"
+         "clocks_event_reasons.hw_thermal_slowdown,clocks_event_reasons.sw_thermal_slowdown,"
+         "clocks_event_reasons.sw_power_cap")
+
+    def __init__(self, device_index: int):
+        self.dev = device_index
+        self.p = None
+
+    def start(self):
+        try:
+            self.p = subprocess.Popen(["nvidia-smi", "-i", str(self.dev), f"--query-gpu={self.Q}",
+                                       "--format=csv,noheader,nounits", "-lms", "100"],
+                                      stdout=subprocess.PIPE, stderr=subprocess.DEVNULL, text=True)
+        except Exception:
+            self.p = None
+
+    def stop(self):
+        if not self.p:
+            return {"sm_mhz": None, "sm_max_mhz": None, "reasons": ["nvidia-smi unavailable"]}
+        self.p.terminate()
+        try:
+            out, _ = self.p.communicate(timeout=5)
+        except Exception:
+            self.p.kill()
+            out = ""
+        sm, mx, reasons = [], [], set()
+        names = ["hw_slowdown", "hw_thermal_slowdown", "sw_thermal_slowdown", "sw_power_cap"]
+        for line in out.strip().splitlines():
+            f = [x.strip() for x in line.split(",")]
+            if len(f) < 9:
+                continue
+            try:
+                sm.append(float(f[1]))
+                mx.append(float(f[2]))
+            except ValueError:
+                continue
+            for nm, v in zip(names, f[5:9]):
+                if v.lower() == "active":
+                    reasons.add(nm)
+        return {"sm_mhz": float(np.median(sm)) if sm else None, "sm_max_mhz": max(mx) if mx else None,
+                "reasons": sorted(reasons), "samples": len(sm)}
+
+
+def dist_env():
+    ws = int(os.environ.get("WORLD_SIZE", "1"))
+    rank = int(os.environ.get("RANK", "0"))
+    local = int(os.environ.get("LOCAL_RANK", "0"))
+    return ws, rank, local
+
+
+def make_graph(cfg):
+    t0 = time.time()
+    ro, co = cfg.make()
+    return ro, co, time.time() - t0
+
+
+def edges_of(cfg, arcs):
+    """TEPS numerator: sum of out-degrees of reached vertices; halved on symmetrised R-MAT."""
+    return arcs / 2 if cfg.symmetric else arcs
+
+
+def choose_roots(ro, count, seed=20190630):
+    import synth
+    return synth.pick_roots(ro, count, seed)
+
+
+def run_reference(args, cfg, ws, rank):
+    """Oracle arm: oracle/ as it stands (plain C, one thread), BFS over the oracle's own CGR."""
+    if rank != 0:
+        return
+    import oracle as O
+    ro, co, tgen = make_graph(cfg)
+    ob, onb, ooffs = O.encode(ro, co, cfg.min_interval_len, cfg.residual_segment_len, cfg.zeta_k)
+    roots = choose_roots(ro, args.roots)
+    for i in range(args.warmup):
+        O.bfs_cgr(ob, ooffs, cfg.min_interval_len, cfg.residual_segment_len, cfg.zeta_k, roots[i % len(roots)])
+    tot_e, tot_t = 0.0, 0.0
+    for i in range(args.steps):
+        r = roots[(args.warmup + i) % len(roots)]
+        t0 = time.perf_counter()
+        _, arcs = O.bfs_cgr(ob, ooffs, cfg.min_interval_len, cfg.residual_segment_len, cfg.zeta_k, r)
+        tot_t += time.perf_counter() - t0
+        tot_e += edges_of(cfg, arcs)
+    v = tot_e / tot_t / 1e9
+    line = {"metric": METRIC, "value": v, "unit": "GTEPS", "n_gpus": ws, "steps": args.steps,
+            "warmup": args.warmup, "ms_per_step": tot_t * 1e3 / args.steps, "higher_is_better": True,
+            "scaling": "weak", "vs_baseline": None, "dtype": "u32", "data": "synthetic", "impl": "reference",
+            "config": {"workload": cfg.name + ": " + cfg.desc, "n": int(ro.size - 1), "m": int(ro[-1]),
+                       "min_interval_len": cfg.min_interval_len, "residual_segment_len": cfg.residual_segment_len,
+                       "zeta_k": cfg.zeta_k},
+            "cpu_baseline": {"value": v, "unit": "GTEPS", "cores": 1, "kind": "oracle",
+                             "sample": f"{args.steps} full BFS queries (oracle bfs_cgr over the oracle's CGR)"},
+            "e2e": {"value": v, "unit": "GTEPS", "h2d_bytes_per_step": 0, "d2h_bytes_per_step": 0}}
+    print(json.dumps(line), flush=True)
+
+
+def cpu_baseline(cfg, ro, co, root):
+    """The oracle as it stands, 1 thread, one full BFS over its own CGR from the first bench root (~10 s on c2)."""
+    import oracle as O
+    ob, onb, ooffs = O.encode(ro, co, cfg.min_interval_len, cfg.residual_segment_len, cfg.zeta_k)
+    t0 = time.perf_counter()
+    _, arcs = O.bfs_cgr(ob, ooffs, cfg.min_interval_len, cfg.residual_segment_len, cfg.zeta_k, root)
+    dt = time.perf_counter() - t0
+    return {"value": edges_of(cfg, arcs) / dt / 1e9, "unit": "GTEPS", "cores": 1, "kind": "oracle",
+            "sample": f"1 full BFS from root {root} over the oracle's own CGR of the same graph ({dt:.1f} s)"}
+
+
+def main():
+    args = parse()
+    import synth
+    cfg = synth.CONFIGS[args.config]
+    ws, rank, local = dist_env()
+    if args.impl == "reference":
+        return run_reference(args, cfg, ws, rank)
+
+    import torch
+    import torch.distributed as dist
+    import paper_conf_sigmod_shalt19_b200 as G
+
+    if ws > 1:
+        os.environ.setdefault("MASTER_ADDR", "127.0.0.1")
+        torch.cuda.set_device(local)
+        dist.init_process_group("nccl", device_id=torch.device("cuda", local))
+    else:
+        torch.cuda.set_device(local)
+    dev = torch.device("cuda", local)
+
+    ro, co, tgen = make_graph(cfg)
+    t0 = time.time()
+    cgr = G.encode(ro, co, cfg.min_interval_len, cfg.residual_segment_len, cfg.zeta_k)
+    tenc = time.time() - t0
+    _, nbits, _, n, _ = cgr.view()
+    g = G.load(cgr, device=local, stream="torch")
+    stream = torch.cuda.current_stream(dev)
+    roots_all = choose_roots(ro, args.roots * max(ws, 1))
+    roots = roots_all[rank::max(ws, 1)]
+    levels = torch.empty(n, dtype=torch.int32, device=dev)
+    # L2 flush buffer (> 126 MB L2), written between timed steps, outside the per-step events
+    flush = torch.empty(256 << 20, dtype=torch.uint8, device=dev)
+
+    for i in range(args.warmup):
+        g.bfs(roots[i % len(roots)], out=levels)
+    torch.cuda.synchronize()
+
+    g.profile(True)
+    evs = [(torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)) for _ in range(args.steps)]
+    clocks = ClockSampler(torch.cuda.current_device() if "CUDA_VISIBLE_DEVICES" not in os.environ else local)
+    tot = {"arcs": 0, "bits": 0, "vertices": 0, "levels": 0, "kms": 0.0, "klaunch": 0}
+    if ws > 1:
+        dist.barrier()
+    torch.cuda.synchronize()
+    clocks.start()
+    for i in range(args.steps):
+        flush.fill_(i & 0xFF)
+        evs[i][0].record(stream)
+        g.bfs(roots[(args.warmup + i) % len(roots)], out=levels)
+        evs[i][1].record(stream)
+        st = g.last_stats
+        tot["arcs"] += st["arcs_decoded"]
+        tot["bits"] += st["cgr_bits_decoded"]
+        tot["vertices"] += st["vertices_expanded"]
+        tot["levels"] += st["iterations"]
+        tot["kms"] += st["kernel_ms"]
+        tot["klaunch"] += st["kernel_launches"]
+    torch.cuda.synchronize()
+    if ws > 1:
+        dist.barrier()
+    ck = clocks.stop()
+    g.profile(False)
+    t_ms = sum(a.elapsed_time(b) for a, b in evs)
+    edges = edges_of(cfg, tot["arcs"])
+    if ws > 1:
+        tt = torch.tensor([t_ms], dtype=torch.float64, device=dev)
+        dist.all_reduce(tt, op=dist.ReduceOp.MAX)
+        ee = torch.tensor([edges], dtype=torch.float64, device=dev)
+        dist.all_reduce(ee, op=dist.ReduceOp.SUM)
+        t_ms, edges_all = float(tt.item()), float(ee.item())
+    else:
+        edges_all = edges
+    value = edges_all / (t_ms * 1e-3) / 1e9
+
+    # roofline of the dominant kernel (bfs_expand): algorithmic bytes per launch =
+    # CGR bytes of the expanded records + 8 B bit offset + 4 B level write per expanded vertex
+    peak, peak_src = hbm_peak()
+    alg_bytes = tot["bits"] / 8 + 12 * tot["vertices"]
+    k_s = tot["kms"] * 1e-3
+    achieved = alg_bytes / k_s / 1e9 if k_s > 0 else 0.0
+    cgr_gbs = tot["bits"] / 8 / k_s / 1e9 if k_s > 0 else 0.0
+    launches_per_step = 2 * tot["levels"] / args.steps + 1  # expand + commit per level, + seed
+
+    e2e = None
+    if not args.no_e2e:
+        e2e = measure_e2e(G, cgr, roots, cfg, n, nbits, dev, local, steps=min(args.steps, 3))
+
+    cpu = None
+    if rank == 0 and ws == 1 and not args.no_cpu_baseline:
+        cpu = cpu_baseline(cfg, ro, co, roots[0])
+
+    if rank == 0:
+        line = {"metric": METRIC, "value": value, "unit": "GTEPS", "n_gpus": ws, "steps": args.steps,
+                "warmup": args.warmup, "ms_per_step": t_ms / args.steps, "higher_is_better": True,
+                "scaling": "weak", "vs_baseline": None, "dtype": "u32", "data": "synthetic",
+                "config": {"workload": cfg.name + ": " + cfg.desc, "n": int(n), "m": int(ro[-1]),
+                           "bits_per_arc": nbits / max(1, int(ro[-1])), "cgr_mb": nbits / 8e6,
+                           "min_interval_len": cfg.min_interval_len, "residual_segment_len": cfg.residual_segment_len,
+                           "zeta_k": cfg.zeta_k, "roots_per_rank": len(roots), "levels_per_bfs": tot["levels"] / args.steps,
+                           "edges_per_bfs": edges / args.steps,
+                           "l2": "flushed between steps (256 MiB fill, outside the per-step CUDA events)",
+                           "parallelism": f"{ws} x independent BFS queries (replicas)" if ws > 1 else "1 GPU",
+                           "gen_s": round(tgen, 1), "encode_s": round(tenc, 1)},
+                "roofline": {"bound": "hbm", "achieved": achieved, "peak": peak, "unit": "GB/s",
+                             "frac": achieved / peak, "traffic": None, "kernel": "bfs_expand",
+                             "peak_source": peak_src, "cgr_only_gbs": cgr_gbs, "cgr_only_frac": cgr_gbs / peak,
+                             "kernel_share_of_step": tot["kms"] / t_ms if t_ms else None,
+                             "launches": tot["klaunch"]},
+                "cpu_baseline": cpu, "e2e": e2e, "gpu_launches": int(round(launches_per_step * args.steps)),
+                "clocks": ck}
+        print(json.dumps(line), flush=True)
+    g.unload()
+    if ws > 1:
+        dist.destroy_process_group()
+
+
+def measure_e2e(G, cgr, roots, cfg, n, nbits, dev, local, steps=3):
+    """Same metric through the public API with HOST buffers: per step gcgt_load (H2D of the CGR bytes and bit
+    offsets from pinned host memory) + gcgt_bfs into a pinned host levels array (D2H) + gcgt_unload."""
+    import torch
+    cudart = torch.cuda.cudart()
+    b, nb, offs, _, _ = cgr.view()
+    # re-wrap into a CGR whose arrays we can pin: the library copies into its own (pageable) vectors, so pin those
+    import ctypes as C
+    L = G.lib()
+    bp, op = C.c_void_p(), C.c_void_p()
+    L.gcgt_cgr_view(cgr.handle, C.byref(bp), None, C.byref(op), None, None)
+    nbytes_words = ((nbits + 63) // 64 + 2) * 8
+    reg = [(bp.value, nbytes_words), (op.value, (n + 1) * 8)]
+    for ptr, size in reg:
+        cudart.cudaHostRegister(ptr, size, 0)
+    levels = torch.empty(n, dtype=torch.int32).pin_memory()
+    tot_e, tot_t = 0.0, 0.0
+    try:
+        for i in range(steps):
+            torch.cuda.synchronize()
+            t0 = time.perf_counter()
+            g = G.load(cgr, device=local, stream="torch")
+            g.bfs(roots[i % len(roots)], out=levels)
+            arcs = g.last_stats["arcs_decoded"]
+            g.unload()
+            torch.cuda.synchronize()
+            tot_t += time.perf_counter() - t0
+            tot_e += edges_of(cfg, arcs)
+    finally:
+        for ptr, _ in reg:
+            cudart.cudaHostUnregister(ptr)
+    return {"value": tot_e / tot_t / 1e9, "unit": "GTEPS", "h2d_bytes_per_step": int(nbytes_words + (n + 1) * 8),
+            "d2h_bytes_per_step": int(4 * n),
+            "note": "per step: gcgt_load (CGR + bit offsets H2D from pinned host memory, device allocation) + "
+                    "gcgt_bfs with a pinned host levels array + gcgt_unload; host wall clock"}
+
+
+if __name__ == "__main__":
+    main()

@@ -64,6 +64,9 @@ typedef struct {
     uint64_t arcs_decoded;      /* neighbour ids produced by decoding (summed over passes)                     */
     uint64_t cgr_bits_decoded;  /* CGR bits of the records decoded (algorithmic CGR traffic)     */
     double device_ms;           /* device time of the call (CUDA events on the graph's stream)                 */
+    double kernel_ms;           /* with gcgt_profile(g, 1): summed CUDA-event time of the call's dominant kernel
+                                   (BFS/BC: frontier expansion; CC: hooking), else 0                              */
+    uint64_t kernel_launches;   /* launches of that kernel in the call (0 unless profiling)                      */
 } gcgt_stats;
 
 typedef struct gcgt_cgr gcgt_cgr;     /* host CGR: canonical bytes + bit_offsets + params; library-owned     */
@@ -103,6 +106,10 @@ typedef struct {
  * so slicing is a bit copy) plus replicated n-bit bitmaps.  opts may be NULL (device 0, own stream). */
 gcgt_status gcgt_load(const gcgt_cgr* cgr, const gcgt_load_opts* opts, gcgt_graph** out);
 void gcgt_unload(gcgt_graph* g);
+
+/* Enables (1) / disables (0) per-launch CUDA-event timing of the dominant kernel (fills gcgt_stats.kernel_ms).
+ * Adds one event pair per launch; results are unchanged. */
+gcgt_status gcgt_profile(gcgt_graph* g, int enable);
 
 /* Owned vertex range [*lo, *hi) of this rank (whole [0, n) on a single GPU). */
 gcgt_status gcgt_graph_range(const gcgt_graph* g, uint64_t* lo, uint64_t* hi);

@@ -1,0 +1,253 @@
+"""paper_conf_sigmod_shalt19_b200 — thin Python binding over libgcgt.so (include/gcgt.h).
+
+Argument marshalling only: every step of the hot path runs in the library (host C++ encoder + sm_100a kernels).
+There is no CPU fallback: if libgcgt.so is missing or no CUDA device is usable, calls raise ``GcgtError``.
+PyTorch is used (optionally) for device memory and streams: output tensors on ``cuda`` are written in place via
+``GCGT_OUT_DEVICE``; the graph runs on the caller's current torch stream when ``stream="torch"``.
+"""
+from __future__ import annotations
+
+import ctypes as C
+import os
+
+import numpy as np
+
+_HERE = os.path.dirname(os.path.abspath(__file__))
+LIB_PATH = os.path.join(_HERE, "libgcgt.so")
+
+OK, EINVAL, EUNSORTED, ERANGE, ESEGLEN, ENOMEM, ECUDA, ENCCL, EFORMAT = 0, -1, -2, -3, -4, -5, -6, -7, -8
+STATUS_NAMES = {0: "OK", -1: "EINVAL", -2: "EUNSORTED", -3: "ERANGE", -4: "ESEGLEN", -5: "ENOMEM", -6: "ECUDA",
+                -7: "ENCCL", -8: "EFORMAT"}
+OUT_HOST, OUT_DEVICE = 0, 1
+
+# public symbols of include/gcgt.h (tests check the library exports every one)
+ABI_SYMBOLS = ["gcgt_encode", "gcgt_cgr_view", "gcgt_cgr_from_arrays", "gcgt_cgr_save", "gcgt_cgr_open",
+               "gcgt_cgr_free", "gcgt_load", "gcgt_unload", "gcgt_profile", "gcgt_graph_range", "gcgt_bfs", "gcgt_cc", "gcgt_bc",
+               "gcgt_last_error", "gcgt_version"]
+
+
+class GcgtError(RuntimeError):
+    def __init__(self, status: int, what: str, msg: str = ""):
+        super().__init__(f"{what}: {STATUS_NAMES.get(status, status)} {msg}".strip())
+        self.status = status
+
+
+class Params(C.Structure):
+    _fields_ = [("min_interval_len", C.c_uint32), ("residual_segment_len", C.c_uint32), ("zeta_k", C.c_uint32)]
+
+
+class Csr(C.Structure):
+    _fields_ = [("n", C.c_uint64), ("row_offsets", C.c_void_p), ("cols", C.c_void_p)]
+
+
+class Stats(C.Structure):
+    _fields_ = [("iterations", C.c_uint32), ("reserved", C.c_uint32), ("vertices_expanded", C.c_uint64),
+                ("arcs_decoded", C.c_uint64), ("cgr_bits_decoded", C.c_uint64), ("device_ms", C.c_double),
+                ("kernel_ms", C.c_double), ("kernel_launches", C.c_uint64)]
+
+    def as_dict(self):
+        return {k: getattr(self, k) for k, _ in self._fields_ if k != "reserved"}
+
+
+class LoadOpts(C.Structure):
+    _fields_ = [("device", C.c_int), ("stream", C.c_void_p), ("rank", C.c_int), ("nranks", C.c_int),
+                ("nccl_comm", C.c_void_p)]
+
+
+_lib = None
+
+
+def lib():
+    """Loads libgcgt.so (built by build.py / __graft_entry__.build()).  Fails loudly if it is missing."""
+    global _lib
+    if _lib is None:
+        if not os.path.exists(LIB_PATH):
+            raise GcgtError(ECUDA, "libgcgt.so not built", f"({LIB_PATH}); run __graft_entry__.build()")
+        L = C.CDLL(LIB_PATH)
+        p, u32, u64, i32 = C.c_void_p, C.c_uint32, C.c_uint64, C.c_int
+        L.gcgt_encode.argtypes = [C.POINTER(Csr), C.POINTER(Params), C.POINTER(p)]
+        L.gcgt_cgr_view.argtypes = [p, C.POINTER(p), C.POINTER(u64), C.POINTER(p), C.POINTER(u64), C.POINTER(Params)]
+        L.gcgt_cgr_from_arrays.argtypes = [u64, p, u64, p, C.POINTER(Params), C.POINTER(p)]
+        L.gcgt_cgr_save.argtypes = [p, C.c_char_p]
+        L.gcgt_cgr_open.argtypes = [C.c_char_p, C.POINTER(p)]
+        L.gcgt_cgr_free.argtypes = [p]
+        L.gcgt_cgr_free.restype = None
+        L.gcgt_load.argtypes = [p, C.POINTER(LoadOpts), C.POINTER(p)]
+        L.gcgt_unload.argtypes = [p]
+        L.gcgt_unload.restype = None
+        L.gcgt_profile.argtypes = [p, i32]
+        L.gcgt_graph_range.argtypes = [p, C.POINTER(u64), C.POINTER(u64)]
+        L.gcgt_bfs.argtypes = [p, u32, p, i32, C.POINTER(Stats)]
+        L.gcgt_cc.argtypes = [p, p, i32, C.POINTER(Stats)]
+        L.gcgt_bc.argtypes = [p, p, u32, p, i32, C.POINTER(Stats)]
+        L.gcgt_last_error.restype = C.c_char_p
+        L.gcgt_version.restype = C.c_char_p
+        _lib = L
+    return _lib
+
+
+def _check(st: int, what: str):
+    if st != OK:
+        raise GcgtError(st, what, lib().gcgt_last_error().decode(errors="replace"))
+
+
+def _np_ptr(a: np.ndarray):
+    return C.c_void_p(a.ctypes.data)
+
+
+class CGR:
+    """Host CGR (library-owned).  Build with ``encode`` / ``from_arrays`` / ``open``."""
+
+    def __init__(self, handle: C.c_void_p):
+        self._h = handle
+
+    @property
+    def handle(self):
+        return self._h
+
+    def view(self):
+        """(bytes u8[ceil(nbits/8)], nbits, bit_offsets u64[n+1], n, (min_interval_len, residual_segment_len, zeta_k));
+        numpy arrays are copies."""
+        b, off = C.c_void_p(), C.c_void_p()
+        nbits, n = C.c_uint64(), C.c_uint64()
+        P = Params()
+        _check(lib().gcgt_cgr_view(self._h, C.byref(b), C.byref(nbits), C.byref(off), C.byref(n), C.byref(P)),
+               "gcgt_cgr_view")
+        nbytes = (nbits.value + 7) // 8
+        by = np.ctypeslib.as_array((C.c_uint8 * max(nbytes, 1)).from_address(b.value))[:nbytes].copy()
+        bo = np.ctypeslib.as_array((C.c_uint64 * (n.value + 1)).from_address(off.value)).copy()
+        return by, int(nbits.value), bo, int(n.value), (P.min_interval_len, P.residual_segment_len, P.zeta_k)
+
+    def save(self, path: str):
+        _check(lib().gcgt_cgr_save(self._h, path.encode()), "gcgt_cgr_save")
+
+    def free(self):
+        if self._h:
+            lib().gcgt_cgr_free(self._h)
+            self._h = None
+
+    def __del__(self):
+        try:
+            self.free()
+        except Exception:
+            pass
+
+
+def encode(row_offsets: np.ndarray, cols: np.ndarray, min_interval_len: int = 4, residual_segment_len: int = 32,
+           zeta_k: int = 3) -> CGR:
+    ro = np.ascontiguousarray(row_offsets, dtype=np.uint64)
+    co = np.ascontiguousarray(cols, dtype=np.uint32)
+    if co.size == 0:
+        co = np.zeros(1, dtype=np.uint32)
+    csr = Csr(ro.size - 1, ro.ctypes.data, co.ctypes.data)
+    P = Params(min_interval_len, residual_segment_len, zeta_k)
+    h = C.c_void_p()
+    _check(lib().gcgt_encode(C.byref(csr), C.byref(P), C.byref(h)), "gcgt_encode")
+    return CGR(h)
+
+
+def from_arrays(bytes_: np.ndarray, nbits: int, bit_offsets: np.ndarray, min_interval_len: int,
+                residual_segment_len: int, zeta_k: int) -> CGR:
+    b = np.ascontiguousarray(bytes_, dtype=np.uint8)
+    if b.size == 0:
+        b = np.zeros(1, dtype=np.uint8)
+    bo = np.ascontiguousarray(bit_offsets, dtype=np.uint64)
+    P = Params(min_interval_len, residual_segment_len, zeta_k)
+    h = C.c_void_p()
+    _check(lib().gcgt_cgr_from_arrays(bo.size - 1, _np_ptr(b), nbits, _np_ptr(bo), C.byref(P), C.byref(h)),
+           "gcgt_cgr_from_arrays")
+    return CGR(h)
+
+
+def open_cgr(path: str) -> CGR:
+    h = C.c_void_p()
+    _check(lib().gcgt_cgr_open(path.encode(), C.byref(h)), "gcgt_cgr_open")
+    return CGR(h)
+
+
+def _out(out, n, np_dtype, torch_dtype_name):
+    """Returns (pointer, placement, result_object)."""
+    if out is None:
+        a = np.empty(n, dtype=np_dtype)
+        return _np_ptr(a), OUT_HOST, a
+    if isinstance(out, np.ndarray):
+        if out.dtype != np_dtype or out.size != n or not out.flags.c_contiguous:
+            raise GcgtError(EINVAL, "output array", f"need contiguous {np_dtype} of size {n}")
+        return _np_ptr(out), OUT_HOST, out
+    # torch tensor
+    import torch
+    if out.dtype != getattr(torch, torch_dtype_name) or out.numel() != n or not out.is_contiguous():
+        raise GcgtError(EINVAL, "output tensor", f"need contiguous {torch_dtype_name} of size {n}")
+    return C.c_void_p(out.data_ptr()), (OUT_DEVICE if out.is_cuda else OUT_HOST), out
+
+
+class Graph:
+    """Device-resident CGR (gcgt_load)."""
+
+    def __init__(self, cgr: CGR, device: int = 0, stream=None, rank: int = 0, nranks: int = 1, nccl_comm=None):
+        if stream == "torch":
+            import torch
+            stream = torch.cuda.current_stream(device).cuda_stream
+        opts = LoadOpts(device, C.c_void_p(stream) if stream else None, rank, nranks,
+                        C.c_void_p(nccl_comm) if nccl_comm else None)
+        h = C.c_void_p()
+        _check(lib().gcgt_load(cgr.handle, C.byref(opts), C.byref(h)), "gcgt_load")
+        self._h = h
+        self.n = cgr_n(cgr)
+        self.last_stats: dict = {}
+
+    def profile(self, enable: bool = True):
+        _check(lib().gcgt_profile(self._h, 1 if enable else 0), "gcgt_profile")
+
+    def range(self):
+        lo, hi = C.c_uint64(), C.c_uint64()
+        _check(lib().gcgt_graph_range(self._h, C.byref(lo), C.byref(hi)), "gcgt_graph_range")
+        return int(lo.value), int(hi.value)
+
+    def bfs(self, source: int, out=None):
+        ptr, where, res = _out(out, self.n, np.int32, "int32")
+        st = Stats()
+        _check(lib().gcgt_bfs(self._h, source, ptr, where, C.byref(st)), "gcgt_bfs")
+        self.last_stats = st.as_dict()
+        return res
+
+    def cc(self, out=None):
+        ptr, where, res = _out(out, self.n, np.uint32, "int32")
+        st = Stats()
+        _check(lib().gcgt_cc(self._h, ptr, where, C.byref(st)), "gcgt_cc")
+        self.last_stats = st.as_dict()
+        return res
+
+    def bc(self, sources, out=None):
+        src = np.ascontiguousarray(sources, dtype=np.uint32)
+        ptr, where, res = _out(out, self.n, np.float64, "float64")
+        st = Stats()
+        _check(lib().gcgt_bc(self._h, _np_ptr(src) if src.size else None, src.size, ptr, where, C.byref(st)),
+               "gcgt_bc")
+        self.last_stats = st.as_dict()
+        return res
+
+    def unload(self):
+        if self._h:
+            lib().gcgt_unload(self._h)
+            self._h = None
+
+    def __del__(self):
+        try:
+            self.unload()
+        except Exception:
+            pass
+
+
+def cgr_n(cgr: CGR) -> int:
+    n = C.c_uint64()
+    _check(lib().gcgt_cgr_view(cgr.handle, None, None, None, C.byref(n), None), "gcgt_cgr_view")
+    return int(n.value)
+
+
+def load(cgr: CGR, device: int = 0, stream=None, **kw) -> Graph:
+    return Graph(cgr, device, stream, **kw)
+
+
+def version() -> str:
+    return lib().gcgt_version().decode()
