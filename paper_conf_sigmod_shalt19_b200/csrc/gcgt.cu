@@ -56,6 +56,12 @@ struct Stats {  // device-side counters
     unsigned long long vertices, arcs, bits;
 };
 
+struct HubEntry {
+    uint64_t base;     // bit position of the vertex's first residual segment
+    uint32_t u;        // vertex
+    uint32_t seg_off;  // first flattened segment index of this entry (entries are ordered by seg_off)
+};
+
 struct gcgt_graph {
     int device = 0;
     cudaStream_t stream = nullptr;
@@ -71,7 +77,9 @@ struct gcgt_graph {
     uint32_t* q = nullptr;      // word queue storage (BFS: 2 x nw ping-pong; BC: all levels, nw + n)
     uint32_t* qbits = nullptr;  // BC: frontier bits per queue entry
     uint64_t qcap = 0;
-    uint32_t* ctr = nullptr;    // device counters [4]
+    uint32_t* ctr = nullptr;    // device counters [8]
+    HubEntry* hubq = nullptr;   // per-level hub queue (capacity = hub vertices + 1)
+    unsigned long long* hub_ctr = nullptr;
     Stats* stats = nullptr;
     int32_t* levels = nullptr;
     uint32_t* parent = nullptr;
@@ -91,52 +99,100 @@ namespace {
 
 constexpr int kBlock = 256;
 constexpr int kWarps = kBlock / 32;
+// A vertex with more residual segments than this is not expanded by its own warp: its segments go to the
+// level's hub queue and are spread over the whole grid (segment-level work stealing, the B200 analogue of the
+// paper's Task Stealing + Residual Segmentation, §4.3 :884-930, §5.2 :1092-1136).
+constexpr uint32_t kHubSegs = 32;
 
 __device__ __forceinline__ uint32_t lane_id() { return threadIdx.x & 31; }
+__device__ __forceinline__ uint32_t lanemask_lt() { uint32_t m; asm("mov.u32 %0, %%lanemask_lt;" : "=r"(m)); return m; }
 
-// Appends word index w to the queue; aggregated over the currently converged lanes (one atomic per group).
-__device__ __forceinline__ void enqueue_word(uint32_t* __restrict__ qn, uint32_t* __restrict__ qn_len, uint32_t w) {
-    cg::coalesced_group g = cg::coalesced_threads();
-    uint32_t base = 0;
-    if (g.thread_rank() == 0) base = atomicAdd(qn_len, g.size());
-    base = g.shfl(base, 0);
-    qn[base + g.thread_rank()] = w;
-}
+// Kernel-constant view of the device CGR plus the per-level hub queue.
+struct Ctx {
+    const uint64_t* __restrict__ W;
+    const uint64_t* __restrict__ offs;
+    uint32_t min_len;
+    uint32_t seg_bits;
+    HubEntry* hubq;
+    unsigned long long* hub_ctr;  // (entries << 32) | segments
+    Stats* st;
+};
 
 __device__ __forceinline__ void add_stats(Stats* st, uint64_t v, uint64_t a, uint64_t b) {
-    // warp-reduce then one atomic per warp
-    for (int o = 16; o; o >>= 1) {
+    for (int o = 16; o; o >>= 1) {  // warp reduce (call with the full warp), one atomic per warp
         v += __shfl_xor_sync(0xffffffffu, v, o);
         a += __shfl_xor_sync(0xffffffffu, a, o);
         b += __shfl_xor_sync(0xffffffffu, b, o);
     }
-    if (lane_id() == 0 && v) {
-        atomicAdd(&st->vertices, (unsigned long long)v);
-        atomicAdd(&st->arcs, (unsigned long long)a);
-        atomicAdd(&st->bits, (unsigned long long)b);
+    if (lane_id() == 0 && (v | a | b)) {
+        if (v) atomicAdd(&st->vertices, (unsigned long long)v);
+        if (a) atomicAdd(&st->arcs, (unsigned long long)a);
+        if (b) atomicAdd(&st->bits, (unsigned long long)b);
     }
 }
 
-// ---- frontier iteration -------------------------------------------------------------------------------------------
-// Each warp takes `wpb` queue words at a time, expands their set bits into a compact list in shared memory and
-// hands one frontier vertex to each lane.  fn(u, lane_active) is called warp-uniformly (lanes without a vertex
-// pass active = false), so fn may use warp collectives.
-template <class Fn>
-__device__ __forceinline__ void for_each_frontier_vertex(const uint32_t* __restrict__ q, uint32_t qlen,
-                                                         uint32_t* __restrict__ Fbits, const uint32_t* qbits,
-                                                         uint32_t wpb, Fn&& fn) {
+// ---- frontier sources ------------------------------------------------------------------------------------------------
+// Queue of frontier words (BFS / BC): entry i is word q[i]; its bits come from qbits[i] (BC keeps them per level)
+// or from F[w], which is read and cleared (BFS).
+struct QueueFront {
+    const uint32_t* __restrict__ q;
+    const uint32_t* __restrict__ qlen_p;
+    uint32_t* __restrict__ F;
+    const uint32_t* __restrict__ qbits;
+    __device__ __forceinline__ uint64_t size() const { return *qlen_p; }
+    __device__ __forceinline__ void get(uint64_t i, uint32_t& w, uint32_t& bits) const {
+        w = q[i];
+        if (qbits) bits = qbits[i];
+        else { bits = F[w]; F[w] = 0; }
+    }
+};
+
+// Every vertex of [lo, hi) (CC's hooking pass).
+struct DenseFront {
+    uint64_t lo, hi;
+    __device__ __forceinline__ uint64_t size() const { return hi > lo ? ((hi + 31) >> 5) - (lo >> 5) : 0; }
+    __device__ __forceinline__ void get(uint64_t i, uint32_t& w, uint32_t& bits) const {
+        w = (uint32_t)((lo >> 5) + i);
+        const uint64_t v0 = (uint64_t)w * 32;
+        bits = 0xffffffffu;
+        if (v0 < lo) bits &= 0xffffffffu << (lo - v0);
+        if (v0 + 32 > hi) bits &= (hi - v0 >= 32) ? 0xffffffffu : ((1u << (hi - v0)) - 1);
+    }
+};
+
+// ---- decode helpers ---------------------------------------------------------------------------------------------------
+// One residual segment (FORMAT.md R17): count, first residual anchored at u, then gaps.  Returns the count.
+template <int K, class T>
+__device__ __forceinline__ uint32_t decode_segment(const uint64_t* __restrict__ W, uint64_t q, uint32_t u, T& t) {
+    const uint32_t cnt = (uint32_t)(decode<K>(W, q) - 1);
+    int64_t cur = unmap_first(u, decode<K>(W, q));
+    t.one((uint32_t)cur);
+    for (uint32_t i = 1; i < cnt; i++) {
+        cur += (int64_t)decode<K>(W, q);
+        t.one((uint32_t)cur);
+    }
+    return cnt;
+}
+
+// ---- the expansion engine -----------------------------------------------------------------------------------------
+// Phase A (lane per frontier vertex): App::vertex, then the record header and interval area (decoded serially,
+// each interval handed over as a range), then segNum.  Unsegmented records are decoded completely here.
+// Phase B (segmented format): the warp's segments are flattened with a warp scan and decoded one segment per lane
+// (each segment is self-contained, R17), so the lanes' work is bounded by 2 segBits bits regardless of degree.
+// Vertices with more than kHubSegs segments go to the hub queue (hub_kernel).
+template <int K, bool SEG, class App, class Front>
+__global__ void __launch_bounds__(kBlock) expand_kernel(Ctx c, Front fr, App app, uint32_t wpb) {
     __shared__ uint32_t s_w[kWarps][32], s_b[kWarps][32], s_pre[kWarps][33];
+    __shared__ uint32_t s_u[kWarps][32], s_spre[kWarps][33];
+    __shared__ uint64_t s_base[kWarps][32];
     const uint32_t wid = threadIdx.x >> 5, lane = lane_id();
     const uint64_t gw = (uint64_t)blockIdx.x * kWarps + wid, nwarps = (uint64_t)gridDim.x * kWarps;
+    const uint64_t qlen = fr.size();
+    uint64_t nv = 0, na = 0, nb = 0;
     for (uint64_t base = gw * wpb; base < qlen; base += nwarps * wpb) {
         uint32_t w = 0, bits = 0;
-        if (lane < wpb && base + lane < qlen) {
-            w = q[base + lane];
-            if (qbits) bits = qbits[base + lane];
-            else { bits = Fbits[w]; Fbits[w] = 0; }
-        }
-        const uint32_t c = __popc(bits);
-        uint32_t incl = c;
+        if (lane < wpb && base + lane < qlen) fr.get(base + lane, w, bits);
+        uint32_t incl = __popc(bits);
         for (int o = 1; o < 32; o <<= 1) {
             const uint32_t t = __shfl_up_sync(0xffffffffu, incl, o);
             if (lane >= (uint32_t)o) incl += t;
@@ -147,101 +203,204 @@ __device__ __forceinline__ void for_each_frontier_vertex(const uint32_t* __restr
         if (lane == 0) s_pre[wid][0] = 0;
         __syncwarp();
         const uint32_t total = s_pre[wid][32];
-        for (uint32_t t = 0; t < total; t += 32) {
-            const uint32_t j = t + lane;
-            uint32_t u = 0;
-            const bool act = j < total;
-            if (act) {
-                uint32_t lo = 0, hi = 31;  // owner: largest o with s_pre[o] <= j
+        for (uint32_t t0 = 0; t0 < total; t0 += 32) {
+            // ---- phase A
+            const uint32_t j = t0 + lane;
+            uint32_t nseg = 0, u = 0;
+            uint64_t segbase = 0;
+            if (j < total) {
+                uint32_t lo = 0, hi = 31;  // owner lane: largest o with s_pre[o] <= j
                 while (lo < hi) {
                     const uint32_t mid = (lo + hi + 1) >> 1;
                     if (s_pre[wid][mid] <= j) lo = mid; else hi = mid - 1;
                 }
-                const uint32_t r = j - s_pre[wid][lo];
-                const uint32_t pos = __fns(s_b[wid][lo], 0, (int)r + 1);
-                u = s_w[wid][lo] * 32 + pos;
+                u = s_w[wid][lo] * 32 + __fns(s_b[wid][lo], 0, (int)(j - s_pre[wid][lo]) + 1);
+                uint64_t p = ldg64(c.offs + u);
+                nb += ldg64(c.offs + u + 1) - p;
+                nv++;
+                App t = app;
+                t.begin(u);
+                t.vertex(u);
+                uint64_t deg = 0;
+                if (!SEG) deg = decode<K>(c.W, p) - 1;
+                const uint64_t itv = decode<K>(c.W, p) - 1;
+                int64_t prev_end = 0;
+                uint64_t in_itv = 0;
+                for (uint64_t i = 0; i < itv; i++) {
+                    const uint64_t g = decode<K>(c.W, p);
+                    const uint64_t len = decode<K>(c.W, p) - 1 + c.min_len;
+                    const int64_t start = i == 0 ? unmap_first(u, g) : prev_end + (int64_t)g;
+                    t.range((uint32_t)start, (uint32_t)len);
+                    prev_end = start + (int64_t)len - 1;
+                    in_itv += len;
+                }
+                na += in_itv;
+                if (!SEG) {
+                    const uint64_t nres = deg - in_itv;
+                    int64_t cur = 0;
+                    for (uint64_t i = 0; i < nres; i++) {
+                        const uint64_t cd = decode<K>(c.W, p);
+                        cur = i == 0 ? unmap_first(u, cd) : cur + (int64_t)cd;
+                        t.one((uint32_t)cur);
+                    }
+                    na += nres;
+                } else {
+                    nseg = (uint32_t)(decode<K>(c.W, p) - 1);
+                    segbase = p;
+                    if (nseg > kHubSegs) {  // hub: hand the segments to the whole grid
+                        const unsigned long long old = atomicAdd(c.hub_ctr, (1ull << 32) | (unsigned long long)nseg);
+                        c.hubq[old >> 32] = HubEntry{segbase, u, (uint32_t)(old & 0xffffffffu)};
+                        nseg = 0;
+                    }
+                }
+                t.end();
             }
-            fn(u, act);
+            if (SEG) {
+                // ---- phase B: flatten the warp's segments and decode one per lane
+                uint32_t sincl = nseg;
+                for (int o = 1; o < 32; o <<= 1) {
+                    const uint32_t tt = __shfl_up_sync(0xffffffffu, sincl, o);
+                    if (lane >= (uint32_t)o) sincl += tt;
+                }
+                s_u[wid][lane] = u;
+                s_base[wid][lane] = segbase;
+                s_spre[wid][lane + 1] = sincl;
+                if (lane == 0) s_spre[wid][0] = 0;
+                __syncwarp();
+                const uint32_t stotal = s_spre[wid][32];
+                for (uint32_t k0 = 0; k0 < stotal; k0 += 32) {
+                    const uint32_t sj = k0 + lane;
+                    if (sj < stotal) {
+                        uint32_t lo = 0, hi = 31;
+                        while (lo < hi) {
+                            const uint32_t mid = (lo + hi + 1) >> 1;
+                            if (s_spre[wid][mid] <= sj) lo = mid; else hi = mid - 1;
+                        }
+                        const uint32_t su = s_u[wid][lo];
+                        App t = app;
+                        t.begin(su);
+                        na += decode_segment<K>(c.W, s_base[wid][lo] + (uint64_t)(sj - s_spre[wid][lo]) * c.seg_bits,
+                                                su, t);
+                        t.end();
+                    }
+                }
+                __syncwarp();
+            }
         }
         __syncwarp();
     }
+    add_stats(c.st, nv, na, nb);
 }
 
-// ---- BFS ------------------------------------------------------------------------------------------------------------
-struct BfsVisitor {
+// Hub segments of the level, flattened over the whole grid (one segment per thread at a time).
+template <int K, class App>
+__global__ void __launch_bounds__(kBlock) hub_kernel(Ctx c, App app) {
+    const unsigned long long hc = *c.hub_ctr;
+    const uint32_t nh = (uint32_t)(hc >> 32), S = (uint32_t)(hc & 0xffffffffu);
+    uint64_t na = 0;
+    for (uint64_t j = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; j < S; j += (uint64_t)gridDim.x * blockDim.x) {
+        uint32_t lo = 0, hi = nh - 1;  // entry: largest e with seg_off <= j
+        while (lo < hi) {
+            const uint32_t mid = (lo + hi + 1) >> 1;
+            if (c.hubq[mid].seg_off <= j) lo = mid; else hi = mid - 1;
+        }
+        const HubEntry e = c.hubq[lo];
+        App t = app;
+        t.begin(e.u);
+        na += decode_segment<K>(c.W, e.base + (j - e.seg_off) * (uint64_t)c.seg_bits, e.u, t);
+        t.end();
+    }
+    add_stats(c.st, 0, na, 0);
+}
+
+// ---- applications (filters, Fig. 7) -------------------------------------------------------------------------------
+// BFS (Fig. 7(b)).  V (visited, levels <= d) is immutable during a level, so it is read through the read-only path;
+// a new vertex is claimed with a fire-and-forget atomicOr on the next-frontier bitmap N (no returned value on the
+// critical path).  An interval is claimed 32 ids per atomic.
+struct BfsApp {
     const uint32_t* __restrict__ V;
     uint32_t* __restrict__ N;
-    uint32_t* __restrict__ qn;
-    uint32_t* __restrict__ qn_len;
+    int32_t* __restrict__ levels;
+    int32_t level;
+    __device__ __forceinline__ void begin(uint32_t) {}
+    __device__ __forceinline__ void end() {}
+    __device__ __forceinline__ void vertex(uint32_t u) { levels[u] = level; }
     __device__ __forceinline__ void claim(uint32_t w, uint32_t mask) {
         const uint32_t cand = mask & ~__ldg(V + w);
-        if (!cand) return;
-        const uint32_t old = atomicOr(N + w, cand);
-        if (old == 0) enqueue_word(qn, qn_len, w);
+        if (cand) atomicOr(N + w, cand);
     }
     __device__ __forceinline__ void one(uint32_t v) { claim(v >> 5, 1u << (v & 31)); }
-    __device__ __forceinline__ void range(uint32_t s, uint32_t len) {  // interval: one claim per 32-id word
-        uint32_t e = s + len;                                           // exclusive
+    __device__ __forceinline__ void range(uint32_t s, uint32_t len) {
+        const uint32_t e = s + len;
         while (s < e) {
-            const uint32_t w = s >> 5, b0 = s & 31;
-            const uint32_t nb = min(32u - b0, e - s);
-            const uint32_t mask = (nb == 32 ? 0xffffffffu : ((1u << nb) - 1)) << b0;
-            claim(w, mask);
+            const uint32_t b0 = s & 31, nb = min(32u - b0, e - s);
+            claim(s >> 5, (nb == 32 ? 0xffffffffu : ((1u << nb) - 1)) << b0);
             s += nb;
         }
     }
 };
 
-template <int K, bool SEG>
-__global__ void __launch_bounds__(kBlock) bfs_expand(const uint64_t* __restrict__ W, const uint64_t* __restrict__ offs,
-                                                     uint32_t min_len, uint32_t seg_bits, int32_t level,
-                                                     const uint32_t* __restrict__ q, const uint32_t* __restrict__ qlen_p,
-                                                     uint32_t* __restrict__ F, const uint32_t* __restrict__ V,
-                                                     uint32_t* __restrict__ N, uint32_t* __restrict__ qn,
-                                                     uint32_t* __restrict__ qn_len, int32_t* __restrict__ levels,
-                                                     uint32_t wpb, Stats* st) {
-    const uint32_t qlen = *qlen_p;
-    BfsVisitor vis{V, N, qn, qn_len};
-    uint64_t nv = 0, na = 0, nb = 0;
-    for_each_frontier_vertex(q, qlen, F, nullptr, wpb, [&](uint32_t u, bool act) {
-        if (!act) return;
-        levels[u] = level;
-        const uint64_t p0 = ldg64(offs + u), p1 = ldg64(offs + u + 1);
-        na += walk_record<K, SEG>(W, p0, u, min_len, seg_bits, vis);
-        nv += 1;
-        nb += p1 - p0;
-    });
-    add_stats(st, nv, na, nb);
-}
-
-// Folds the next frontier into V and F: for every queued word, V |= N, F = N, N = 0.
-__global__ void bfs_commit(const uint32_t* __restrict__ qn, const uint32_t* __restrict__ qn_len,
-                           uint32_t* __restrict__ V, uint32_t* __restrict__ F, uint32_t* __restrict__ N,
-                           uint32_t* __restrict__ qbits_out, uint32_t* __restrict__ reset_ctr) {
-    const uint32_t len = *qn_len;
-    for (uint64_t i = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; i < len; i += (uint64_t)gridDim.x * blockDim.x) {
-        const uint32_t w = qn[i];
-        const uint32_t b = N[w];
-        N[w] = 0;
-        V[w] |= b;
-        if (qbits_out) qbits_out[i] = b;
-        else F[w] = b;
+// BC forward (Fig. 7(d), Brandes [9]): an arc u->v with v not in V (levels <= d) has level(v) = d+1, so
+// sigma(v) += sigma(u); N collects level d+1.
+struct BcFwdApp {
+    const uint32_t* __restrict__ V;
+    uint32_t* __restrict__ N;
+    int32_t* __restrict__ levels;
+    double* __restrict__ sigma;
+    int32_t level;
+    double su;
+    __device__ __forceinline__ void begin(uint32_t u) { su = sigma[u]; }
+    __device__ __forceinline__ void end() {}
+    __device__ __forceinline__ void vertex(uint32_t u) { levels[u] = level; }
+    __device__ __forceinline__ void claim(uint32_t w, uint32_t mask) {
+        const uint32_t cand = mask & ~__ldg(V + w);
+        if (!cand) return;
+        atomicOr(N + w, cand);
+        uint32_t cb = cand;
+        while (cb) {
+            const int b = __ffs(cb) - 1;
+            cb &= cb - 1;
+            atomicAdd(sigma + (uint64_t)w * 32 + b, su);
+        }
     }
-    if (reset_ctr && blockIdx.x == 0 && threadIdx.x == 0) *reset_ctr = 0;
-}
+    __device__ __forceinline__ void one(uint32_t v) { claim(v >> 5, 1u << (v & 31)); }
+    __device__ __forceinline__ void range(uint32_t s, uint32_t len) {
+        const uint32_t e = s + len;
+        while (s < e) {
+            const uint32_t b0 = s & 31, nb = min(32u - b0, e - s);
+            claim(s >> 5, (nb == 32 ? 0xffffffffu : ((1u << nb) - 1)) << b0);
+            s += nb;
+        }
+    }
+};
 
-__global__ void bfs_seed(uint32_t s, uint32_t* V, uint32_t* F, uint32_t* q, uint32_t* qlen, uint32_t* qbits) {
-    V[s >> 5] = 1u << (s & 31);
-    if (F) F[s >> 5] = 1u << (s & 31);
-    q[0] = s >> 5;
-    if (qbits) qbits[0] = 1u << (s & 31);
-    *qlen = 1;
-}
-
-__global__ void bswap_words(uint64_t* w, uint64_t n) {
-    for (uint64_t i = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; i < n; i += (uint64_t)gridDim.x * blockDim.x)
-        w[i] = __byte_perm((uint32_t)(w[i] >> 32), 0, 0x0123) | ((uint64_t)__byte_perm((uint32_t)w[i], 0, 0x0123) << 32);
-}
+// BC backward: delta(u) = sum_{w in out(u), d(w) = d(u)+1} sigma(u)/sigma(w) (1 + delta(w))  (Fig. 7(d)).
+// A vertex's arcs are split over tasks (interval area + segments), so each task adds its partial sum to delta(u)
+// and bc(u) (u != source); delta is zeroed per source.  Zero partials are skipped, so exact zeros stay exact.
+struct BcBwdApp {
+    const int32_t* __restrict__ levels;
+    const double* __restrict__ sigma;
+    double* __restrict__ delta;
+    double* __restrict__ bc;
+    int32_t next;
+    uint32_t source;
+    uint32_t u;
+    double sv, acc;
+    __device__ __forceinline__ void begin(uint32_t uu) { u = uu; sv = sigma[uu]; acc = 0.0; }
+    __device__ __forceinline__ void vertex(uint32_t) {}
+    __device__ __forceinline__ void one(uint32_t w) {
+        if (levels[w] == next) acc += sv / sigma[w] * (1.0 + delta[w]);
+    }
+    __device__ __forceinline__ void range(uint32_t s, uint32_t len) {
+        for (uint32_t t = 0; t < len; t++) one(s + t);
+    }
+    __device__ __forceinline__ void end() {
+        if (acc != 0.0) {
+            atomicAdd(delta + u, acc);
+            if (u != source) atomicAdd(bc + u, acc);
+        }
+    }
+};
 
 // ---- CC -------------------------------------------------------------------------------------------------------------
 // Hooking (Fig. 7(c), Soman et al. [42]) as a lock-free union-find: a root hi is hooked under lo < hi only by
@@ -260,15 +419,17 @@ __device__ __forceinline__ uint32_t cc_find(uint32_t* parent, uint32_t x) {  // 
     return x;
 }
 
-struct CcVisitor {
+struct CcApp {
     uint32_t* parent;
     uint32_t ru;
-    uint32_t hooks;
+    __device__ __forceinline__ void begin(uint32_t u) { ru = cc_find(parent, u); }
+    __device__ __forceinline__ void end() {}
+    __device__ __forceinline__ void vertex(uint32_t) {}
     __device__ __forceinline__ void one(uint32_t v) {
         uint32_t rv = cc_find(parent, v);
         while (ru != rv) {
             const uint32_t hi = max(ru, rv), lo = min(ru, rv);
-            if (atomicCAS(parent + hi, hi, lo) == hi) { hooks++; break; }
+            if (atomicCAS(parent + hi, hi, lo) == hi) break;
             ru = cc_find(parent, ru);  // hi stopped being a root: re-find both
             rv = cc_find(parent, rv);
         }
@@ -277,25 +438,6 @@ struct CcVisitor {
         for (uint32_t t = 0; t < len; t++) one(s + t);
     }
 };
-
-template <int K, bool SEG>
-__global__ void __launch_bounds__(kBlock) cc_hook(const uint64_t* __restrict__ W, const uint64_t* __restrict__ offs,
-                                                  uint32_t min_len, uint32_t seg_bits, uint64_t lo, uint64_t hi,
-                                                  uint32_t* parent, uint32_t* hooks, Stats* st) {
-    uint64_t nv = 0, na = 0, nb = 0, nh = 0;
-    for (uint64_t u = lo + (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; u < hi;
-         u += (uint64_t)gridDim.x * blockDim.x) {
-        CcVisitor vis{parent, cc_find(parent, (uint32_t)u), 0};
-        const uint64_t p0 = ldg64(offs + u), p1 = ldg64(offs + u + 1);
-        na += walk_record<K, SEG>(W, p0, u, min_len, seg_bits, vis);
-        nv++;
-        nb += p1 - p0;
-        nh += vis.hooks;
-    }
-    add_stats(st, nv, na, nb);
-    for (int o = 16; o; o >>= 1) nh += __shfl_xor_sync(0xffffffffu, nh, o);
-    if (lane_id() == 0 && nh) atomicAdd(hooks, (uint32_t)nh);
-}
 
 __global__ void cc_jump(uint32_t* parent, uint64_t n) {
     for (uint64_t v = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; v < n; v += (uint64_t)gridDim.x * blockDim.x) {
@@ -310,129 +452,122 @@ __global__ void cc_init(uint32_t* parent, uint64_t n) {
         parent[v] = (uint32_t)v;
 }
 
-// ---- BC -------------------------------------------------------------------------------------------------------------
-struct BcFwdVisitor {
-    const uint32_t* __restrict__ V;
-    uint32_t* __restrict__ N;
-    uint32_t* __restrict__ qn;
-    uint32_t* __restrict__ qn_len;
-    double* sigma;
-    double su;
-    __device__ __forceinline__ void claim(uint32_t w, uint32_t mask) {
-        const uint32_t cand = mask & ~__ldg(V + w);  // not at level <= d: level(v) = d + 1
-        if (!cand) return;
-        const uint32_t old = atomicOr(N + w, cand);
-        if (old == 0) enqueue_word(qn, qn_len, w);
-        uint32_t c = cand;
-        while (c) {
-            const int b = __ffs(c) - 1;
-            c &= c - 1;
-            atomicAdd(sigma + (uint64_t)w * 32 + b, su);
+// ---- contraction ---------------------------------------------------------------------------------------------------
+// Dense scan of N over words [w_lo, w_hi): every non-zero word is folded into V (and F), cleared, and appended to
+// the next queue (one atomic per warp).  Also resets the hub counter and the consumed queue's length.
+__global__ void commit_dense(uint32_t* __restrict__ V, uint32_t* __restrict__ F, uint32_t* __restrict__ N,
+                             uint64_t w_lo, uint64_t w_hi, uint32_t* __restrict__ qn, uint32_t* __restrict__ qn_len,
+                             uint32_t* __restrict__ qbits_out, uint32_t* __restrict__ reset_ctr,
+                             unsigned long long* __restrict__ hub_ctr) {
+    const uint32_t lane = lane_id();
+    const uint64_t gw = ((uint64_t)blockIdx.x * blockDim.x + threadIdx.x) >> 5;
+    const uint64_t nwarps = ((uint64_t)gridDim.x * blockDim.x) >> 5;
+    for (uint64_t base = w_lo + gw * 32; base < w_hi; base += nwarps * 32) {
+        const uint64_t w = base + lane;
+        uint32_t b = 0;
+        if (w < w_hi) {
+            b = N[w];
+            if (b) {
+                N[w] = 0;
+                V[w] |= b;
+                if (F) F[w] = b;
+            }
+        }
+        const uint32_t bal = __ballot_sync(0xffffffffu, b != 0);
+        if (bal) {
+            uint32_t pos = 0;
+            if (lane == 0) pos = atomicAdd(qn_len, __popc(bal));
+            pos = __shfl_sync(0xffffffffu, pos, 0) + __popc(bal & lanemask_lt());
+            if (b) {
+                qn[pos] = (uint32_t)w;
+                if (qbits_out) qbits_out[pos] = b;
+            }
         }
     }
-    __device__ __forceinline__ void one(uint32_t v) { claim(v >> 5, 1u << (v & 31)); }
-    __device__ __forceinline__ void range(uint32_t s, uint32_t len) {
-        uint32_t e = s + len;
-        while (s < e) {
-            const uint32_t w = s >> 5, b0 = s & 31;
-            const uint32_t nb = min(32u - b0, e - s);
-            claim(w, (nb == 32 ? 0xffffffffu : ((1u << nb) - 1)) << b0);
-            s += nb;
-        }
+    if (blockIdx.x == 0 && threadIdx.x == 0) {
+        if (reset_ctr) *reset_ctr = 0;
+        if (hub_ctr) *hub_ctr = 0;
     }
-};
-
-template <int K, bool SEG>
-__global__ void __launch_bounds__(kBlock) bc_forward(const uint64_t* __restrict__ W, const uint64_t* __restrict__ offs,
-                                                     uint32_t min_len, uint32_t seg_bits, int32_t level,
-                                                     const uint32_t* __restrict__ q, const uint32_t* __restrict__ qbits,
-                                                     const uint32_t* __restrict__ qlen_p, const uint32_t* __restrict__ V,
-                                                     uint32_t* __restrict__ N, uint32_t* __restrict__ qn,
-                                                     uint32_t* __restrict__ qn_len, int32_t* __restrict__ levels,
-                                                     double* sigma, uint32_t wpb, Stats* st) {
-    const uint32_t qlen = *qlen_p;
-    uint64_t nv = 0, na = 0, nb = 0;
-    for_each_frontier_vertex(q, qlen, nullptr, qbits, wpb, [&](uint32_t u, bool act) {
-        if (!act) return;
-        levels[u] = level;
-        BcFwdVisitor vis{V, N, qn, qn_len, sigma, sigma[u]};
-        const uint64_t p0 = ldg64(offs + u), p1 = ldg64(offs + u + 1);
-        na += walk_record<K, SEG>(W, p0, u, min_len, seg_bits, vis);
-        nv++;
-        nb += p1 - p0;
-    });
-    add_stats(st, nv, na, nb);
 }
 
-struct BcBwdVisitor {
-    const int32_t* __restrict__ levels;
-    const double* __restrict__ sigma;
-    const double* __restrict__ delta;
-    int32_t next;
-    double sv;
-    double acc;
-    __device__ __forceinline__ void one(uint32_t w) {
-        if (levels[w] == next) acc += sv / sigma[w] * (1.0 + delta[w]);
-    }
-    __device__ __forceinline__ void range(uint32_t s, uint32_t len) {
-        for (uint32_t t = 0; t < len; t++) one(s + t);
-    }
-};
+__global__ void bfs_seed(uint32_t s, uint32_t* V, uint32_t* F, uint32_t* q, uint32_t* qlen, uint32_t* qbits) {
+    V[s >> 5] = 1u << (s & 31);
+    if (F) F[s >> 5] = 1u << (s & 31);
+    q[0] = s >> 5;
+    if (qbits) qbits[0] = 1u << (s & 31);
+    *qlen = 1;
+}
 
-// delta(v) = sum_{w in out(v), d(w) = d(v)+1} sigma(v)/sigma(w) (1 + delta(w))  (Fig. 7(d), pull form)
-template <int K, bool SEG>
-__global__ void __launch_bounds__(kBlock) bc_backward(const uint64_t* __restrict__ W, const uint64_t* __restrict__ offs,
-                                                      uint32_t min_len, uint32_t seg_bits, int32_t level,
-                                                      const uint32_t* __restrict__ q, const uint32_t* __restrict__ qbits,
-                                                      uint32_t qlen, uint32_t source, const int32_t* __restrict__ levels,
-                                                      const double* __restrict__ sigma, double* __restrict__ delta,
-                                                      double* __restrict__ bc, uint32_t wpb, Stats* st) {
-    uint64_t nv = 0, na = 0, nb = 0;
-    for_each_frontier_vertex(q, qlen, nullptr, qbits, wpb, [&](uint32_t v, bool act) {
-        if (!act) return;
-        BcBwdVisitor vis{levels, sigma, delta, level + 1, sigma[v], 0.0};
-        const uint64_t p0 = ldg64(offs + v), p1 = ldg64(offs + v + 1);
-        na += walk_record<K, SEG>(W, p0, v, min_len, seg_bits, vis);
-        const double d = vis.acc;
-        delta[v] = d;
-        if (v != source) bc[v] += d;
-        nv++;
-        nb += p1 - p0;
-    });
-    add_stats(st, nv, na, nb);
+__global__ void bswap_words(uint64_t* w, uint64_t n) {
+    for (uint64_t i = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; i < n; i += (uint64_t)gridDim.x * blockDim.x)
+        w[i] = __byte_perm((uint32_t)(w[i] >> 32), 0, 0x0123) | ((uint64_t)__byte_perm((uint32_t)w[i], 0, 0x0123) << 32);
+}
+
+// Load-time pass: number of hub vertices (more than kHubSegs residual segments); sizes the hub queue.
+template <int K>
+__global__ void count_hubs(const uint64_t* __restrict__ W, const uint64_t* __restrict__ offs, uint32_t min_len,
+                           uint64_t n, unsigned long long* out) {
+    uint32_t cnt = 0;
+    for (uint64_t u = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; u < n; u += (uint64_t)gridDim.x * blockDim.x) {
+        uint64_t p = ldg64(offs + u);
+        const uint64_t itv = decode<K>(W, p) - 1;
+        for (uint64_t i = 0; i < 2 * itv; i++) decode<K>(W, p);
+        if (decode<K>(W, p) - 1 > kHubSegs) cnt++;
+    }
+    for (int o = 16; o; o >>= 1) cnt += __shfl_xor_sync(0xffffffffu, cnt, o);
+    if (lane_id() == 0 && cnt) atomicAdd(out, (unsigned long long)cnt);
 }
 
 // ---- dispatch -------------------------------------------------------------------------------------------------------
-#define GCGT_DISPATCH(P, KERNEL, GRID, BLOCK, STREAM, ...)                                                      \
-    do {                                                                                                        \
-        const bool seg_ = (P).residual_segment_len != 0;                                                        \
-        switch ((P).zeta_k) {                                                                                   \
-            case 1: if (seg_) KERNEL<1, true><<<GRID, BLOCK, 0, STREAM>>>(__VA_ARGS__);                         \
-                    else KERNEL<1, false><<<GRID, BLOCK, 0, STREAM>>>(__VA_ARGS__); break;                      \
-            case 2: if (seg_) KERNEL<2, true><<<GRID, BLOCK, 0, STREAM>>>(__VA_ARGS__);                         \
-                    else KERNEL<2, false><<<GRID, BLOCK, 0, STREAM>>>(__VA_ARGS__); break;                      \
-            case 3: if (seg_) KERNEL<3, true><<<GRID, BLOCK, 0, STREAM>>>(__VA_ARGS__);                         \
-                    else KERNEL<3, false><<<GRID, BLOCK, 0, STREAM>>>(__VA_ARGS__); break;                      \
-            case 4: if (seg_) KERNEL<4, true><<<GRID, BLOCK, 0, STREAM>>>(__VA_ARGS__);                         \
-                    else KERNEL<4, false><<<GRID, BLOCK, 0, STREAM>>>(__VA_ARGS__); break;                      \
-            default: if (seg_) KERNEL<5, true><<<GRID, BLOCK, 0, STREAM>>>(__VA_ARGS__);                        \
-                    else KERNEL<5, false><<<GRID, BLOCK, 0, STREAM>>>(__VA_ARGS__); break;                      \
-        }                                                                                                       \
-    } while (0)
+template <int K, bool SEG, class App, class Front>
+inline void launch_expand_k(int grid, cudaStream_t s, const Ctx& c, const Front& fr, const App& app, uint32_t wpb) {
+    expand_kernel<K, SEG, App, Front><<<grid, kBlock, 0, s>>>(c, fr, app, wpb);
+}
 
-// Grid for a frontier of qlen words: aim for ~1 word per lane when the queue is small, batches of 32 otherwise.
-inline void frontier_launch(const gcgt_graph* g, uint32_t qlen, int* grid, uint32_t* wpb) {
+template <class App, class Front>
+inline void launch_expand(const gcgt_params& P, int grid, cudaStream_t s, const Ctx& c, const Front& fr,
+                          const App& app, uint32_t wpb) {
+    const bool seg = P.residual_segment_len != 0;
+    switch (P.zeta_k) {
+        case 1: seg ? launch_expand_k<1, true>(grid, s, c, fr, app, wpb) : launch_expand_k<1, false>(grid, s, c, fr, app, wpb); break;
+        case 2: seg ? launch_expand_k<2, true>(grid, s, c, fr, app, wpb) : launch_expand_k<2, false>(grid, s, c, fr, app, wpb); break;
+        case 3: seg ? launch_expand_k<3, true>(grid, s, c, fr, app, wpb) : launch_expand_k<3, false>(grid, s, c, fr, app, wpb); break;
+        case 4: seg ? launch_expand_k<4, true>(grid, s, c, fr, app, wpb) : launch_expand_k<4, false>(grid, s, c, fr, app, wpb); break;
+        default: seg ? launch_expand_k<5, true>(grid, s, c, fr, app, wpb) : launch_expand_k<5, false>(grid, s, c, fr, app, wpb); break;
+    }
+}
+
+template <class App>
+inline void launch_hub(const gcgt_params& P, int grid, cudaStream_t s, const Ctx& c, const App& app) {
+    if (!P.residual_segment_len) return;
+    switch (P.zeta_k) {
+        case 1: hub_kernel<1, App><<<grid, kBlock, 0, s>>>(c, app); break;
+        case 2: hub_kernel<2, App><<<grid, kBlock, 0, s>>>(c, app); break;
+        case 3: hub_kernel<3, App><<<grid, kBlock, 0, s>>>(c, app); break;
+        case 4: hub_kernel<4, App><<<grid, kBlock, 0, s>>>(c, app); break;
+        default: hub_kernel<5, App><<<grid, kBlock, 0, s>>>(c, app); break;
+    }
+}
+
+// Grid for a frontier of qlen words: ~1 word per warp when the queue is small, up to 32 per warp batch otherwise.
+inline void frontier_launch(const gcgt_graph* g, uint64_t qlen, int* grid, uint32_t* wpb) {
     const uint64_t max_warps = (uint64_t)g->num_sms * 2048 / 32;  // one wave at full occupancy
     uint32_t b = 1;
-    while (b < 32 && (uint64_t)qlen > max_warps * b) b <<= 1;
-    uint64_t warps = ((uint64_t)qlen + b - 1) / b;
-    uint64_t blocks = std::max<uint64_t>(1, (warps + kWarps - 1) / kWarps);
+    while (b < 32 && qlen > max_warps * b) b <<= 1;
+    const uint64_t warps = (qlen + b - 1) / b;
+    const uint64_t blocks = std::max<uint64_t>(1, (warps + kWarps - 1) / kWarps);
     *grid = (int)std::min<uint64_t>(blocks, (uint64_t)g->num_sms * 8);
     *wpb = b;
 }
 
 inline int flat_grid(const gcgt_graph* g, uint64_t n) {
     return (int)std::max<uint64_t>(1, std::min<uint64_t>((n + kBlock - 1) / kBlock, (uint64_t)g->num_sms * 16));
+}
+
+inline int hub_grid(const gcgt_graph* g) { return g->num_sms * 4; }
+
+inline Ctx make_ctx(const gcgt_graph* g) {
+    return Ctx{g->W, g->offs, g->P.min_interval_len, 8 * g->P.residual_segment_len, g->hubq, g->hub_ctr, g->stats};
 }
 
 gcgt_status copy_out(gcgt_graph* g, void* dst, const void* src, size_t bytes, int placement) {
@@ -506,7 +641,7 @@ extern "C" void gcgt_unload(gcgt_graph* g) {
     cudaSetDevice(g->device);
     if (g->stream) cudaStreamSynchronize(g->stream);
     cudaFree(g->W); cudaFree(g->offs); cudaFree(g->V); cudaFree(g->F); cudaFree(g->N); cudaFree(g->q);
-    cudaFree(g->qbits); cudaFree(g->ctr); cudaFree(g->stats); cudaFree(g->levels); cudaFree(g->parent);
+    cudaFree(g->qbits); cudaFree(g->ctr); cudaFree(g->hubq); cudaFree(g->hub_ctr); cudaFree(g->stats); cudaFree(g->levels); cudaFree(g->parent);
     cudaFree(g->sigma); cudaFree(g->delta); cudaFree(g->bc);
     if (g->h_ctr) cudaFreeHost(g->h_ctr);
     if (g->h_stats) cudaFreeHost(g->h_stats);
@@ -563,6 +698,23 @@ extern "C" gcgt_status gcgt_load(const gcgt_cgr* c, const gcgt_load_opts* opts, 
                        g->stream));
     bswap_words<<<flat_grid(g.get(), nwords), kBlock, 0, g->stream>>>(g->W, nwords);
     CU(cudaMemsetAsync(g->N, 0, g->nw * 4, g->stream));
+    if ((st = dalloc(&g->hub_ctr, 1))) return st;
+    uint64_t nhubs = 0;
+    if (g->P.residual_segment_len) {
+        CU(cudaMemsetAsync(g->hub_ctr, 0, 8, g->stream));
+        const int gr = flat_grid(g.get(), g->n);
+        switch (g->P.zeta_k) {
+            case 1: count_hubs<1><<<gr, kBlock, 0, g->stream>>>(g->W, g->offs, g->P.min_interval_len, g->n, g->hub_ctr); break;
+            case 2: count_hubs<2><<<gr, kBlock, 0, g->stream>>>(g->W, g->offs, g->P.min_interval_len, g->n, g->hub_ctr); break;
+            case 3: count_hubs<3><<<gr, kBlock, 0, g->stream>>>(g->W, g->offs, g->P.min_interval_len, g->n, g->hub_ctr); break;
+            case 4: count_hubs<4><<<gr, kBlock, 0, g->stream>>>(g->W, g->offs, g->P.min_interval_len, g->n, g->hub_ctr); break;
+            default: count_hubs<5><<<gr, kBlock, 0, g->stream>>>(g->W, g->offs, g->P.min_interval_len, g->n, g->hub_ctr); break;
+        }
+        CU(cudaMemcpyAsync(&nhubs, g->hub_ctr, 8, cudaMemcpyDeviceToHost, g->stream));
+    }
+    CU(cudaStreamSynchronize(g->stream));
+    if ((st = dalloc(&g->hubq, nhubs + 1))) return st;
+    CU(cudaMemsetAsync(g->hub_ctr, 0, 8, g->stream));
     CU(cudaStreamSynchronize(g->stream));
     CU(cudaGetLastError());
     *out = g.release();
@@ -592,22 +744,25 @@ extern "C" gcgt_status gcgt_bfs(gcgt_graph* g, uint32_t source, int32_t* levels,
     CU(cudaMemsetAsync(g->F, 0, g->nw * 4, s));
     CU(cudaMemsetAsync(g->levels, 0xff, g->n * 4, s));
     CU(cudaMemsetAsync(g->ctr, 0, 8 * 4, s));
+    CU(cudaMemsetAsync(g->hub_ctr, 0, sizeof(unsigned long long), s));
     uint32_t* q[2] = {g->q, g->q + g->nw};
     bfs_seed<<<1, 1, 0, s>>>(source, g->V, g->F, q[0], g->ctr + 0, nullptr);
-    const uint32_t seg_bits = 8 * g->P.residual_segment_len;
-    uint32_t qlen = 1, level = 0;
+    const Ctx c = make_ctx(g);
+    uint64_t qlen = 1;
+    uint32_t level = 0;
     while (qlen) {
         const int cur = level & 1, nxt = cur ^ 1;
         int grid;
         uint32_t wpb;
         frontier_launch(g, qlen, &grid, &wpb);
+        const QueueFront fr{q[cur], g->ctr + cur, g->F, nullptr};
+        const BfsApp app{g->V, g->N, g->levels, (int32_t)level};
         if ((st = kprof_begin(g))) return st;
-        GCGT_DISPATCH(g->P, bfs_expand, grid, kBlock, s, g->W, g->offs, g->P.min_interval_len, seg_bits,
-                      (int32_t)level, q[cur], g->ctr + cur, g->F, g->V, g->N, q[nxt], g->ctr + nxt, g->levels, wpb,
-                      g->stats);
+        launch_expand(g->P, grid, s, c, fr, app, wpb);
         if ((st = kprof_end(g))) return st;
-        bfs_commit<<<flat_grid(g, g->nw), kBlock, 0, s>>>(q[nxt], g->ctr + nxt, g->V, g->F, g->N, nullptr,
-                                                           g->ctr + cur);
+        launch_hub(g->P, hub_grid(g), s, c, app);
+        commit_dense<<<flat_grid(g, g->nw), kBlock, 0, s>>>(g->V, g->F, g->N, 0, g->nw, q[nxt], g->ctr + nxt, nullptr,
+                                                             g->ctr + cur, g->hub_ctr);
         CU(cudaMemcpyAsync(g->h_ctr + nxt, g->ctr + nxt, 4, cudaMemcpyDeviceToHost, s));
         CU(cudaStreamSynchronize(s));
         if ((st = kprof_collect(g))) return st;
@@ -624,13 +779,18 @@ extern "C" gcgt_status gcgt_cc(gcgt_graph* g, uint32_t* labels, int placement, g
     if (!g->parent && (st = dalloc(&g->parent, g->n))) return st;
     if ((st = begin_call(g))) return st;
     cudaStream_t s = g->stream;
-    const uint32_t seg_bits = 8 * g->P.residual_segment_len;
+    CU(cudaMemsetAsync(g->hub_ctr, 0, sizeof(unsigned long long), s));
     cc_init<<<flat_grid(g, g->n), kBlock, 0, s>>>(g->parent, g->n);
-    CU(cudaMemsetAsync(g->ctr, 0, 4, s));
+    const Ctx c = make_ctx(g);
+    const DenseFront fr{g->lo, g->hi};
+    const CcApp app{g->parent, 0};
+    int grid;
+    uint32_t wpb;
+    frontier_launch(g, (g->hi - g->lo + 31) / 32 + 1, &grid, &wpb);
     if ((st = kprof_begin(g))) return st;
-    GCGT_DISPATCH(g->P, cc_hook, flat_grid(g, g->n), kBlock, s, g->W, g->offs, g->P.min_interval_len, seg_bits,
-                  (uint64_t)0, g->n, g->parent, g->ctr, g->stats);
+    launch_expand(g->P, grid, s, c, fr, app, wpb);
     if ((st = kprof_end(g))) return st;
+    launch_hub(g->P, hub_grid(g), s, c, app);
     cc_jump<<<flat_grid(g, g->n), kBlock, 0, s>>>(g->parent, g->n);
     if ((st = copy_out(g, labels, g->parent, g->n * 4, placement))) return st;
     CU(cudaStreamSynchronize(s));
@@ -656,54 +816,58 @@ extern "C" gcgt_status gcgt_bc(gcgt_graph* g, const uint32_t* sources, uint32_t 
     }
     if ((st = begin_call(g))) return st;
     cudaStream_t s = g->stream;
-    const uint32_t seg_bits = 8 * g->P.residual_segment_len;
+    const Ctx c = make_ctx(g);
     CU(cudaMemsetAsync(g->bc, 0, g->n * 8, s));
+    CU(cudaMemsetAsync(g->hub_ctr, 0, sizeof(unsigned long long), s));
     std::vector<uint32_t> lvl_off;
     for (uint32_t si = 0; si < k; si++) {
         const uint32_t src = sources[si];
         CU(cudaMemsetAsync(g->V, 0, g->nw * 4, s));
         CU(cudaMemsetAsync(g->levels, 0xff, g->n * 4, s));
         CU(cudaMemsetAsync(g->sigma, 0, g->n * 8, s));
+        CU(cudaMemsetAsync(g->delta, 0, g->n * 8, s));
         CU(cudaMemsetAsync(g->ctr, 0, 8 * 4, s));
-        double one = 1.0;
+        const double one = 1.0;
         CU(cudaMemcpyAsync(g->sigma + src, &one, 8, cudaMemcpyHostToDevice, s));
-        // level d occupies q[lvl_off[d] .. lvl_off[d+1]); ctr[0] = running total of queued words
-        bfs_seed<<<1, 1, 0, s>>>(src, g->V, nullptr, g->q, g->ctr + 0, g->qbits);
+        // level d occupies q[lvl_off[d] .. lvl_off[d+1]) (words) with qbits (their frontier bits)
+        bfs_seed<<<1, 1, 0, s>>>(src, g->V, nullptr, g->q, g->ctr + 2, g->qbits);
         lvl_off.assign(1, 0);
         uint32_t total = 1, level = 0;
-        // ctr[1] = length of the level being built; the kernels index q from lvl_off
-        while (true) {
+        for (;;) {
             const uint32_t off = lvl_off.back(), qlen = total - off;
             lvl_off.push_back(total);
             if (!qlen) break;
-            CU(cudaMemcpyAsync(g->ctr + 2, &qlen, 4, cudaMemcpyHostToDevice, s));
-            CU(cudaMemsetAsync(g->ctr + 1, 0, 4, s));
             int grid;
             uint32_t wpb;
             frontier_launch(g, qlen, &grid, &wpb);
+            // ctr[2] holds this level's length (seed or the previous commit), ctr[3] receives the next one
+            const QueueFront fr{g->q + off, g->ctr + 2 + (level & 1), nullptr, g->qbits + off};
+            const BcFwdApp app{g->V, g->N, g->levels, g->sigma, (int32_t)level, 0.0};
             if ((st = kprof_begin(g))) return st;
-            GCGT_DISPATCH(g->P, bc_forward, grid, kBlock, s, g->W, g->offs, g->P.min_interval_len, seg_bits,
-                          (int32_t)level, g->q + off, g->qbits + off, g->ctr + 2, g->V, g->N, g->q + total,
-                          g->ctr + 1, g->levels, g->sigma, wpb, g->stats);
+            launch_expand(g->P, grid, s, c, fr, app, wpb);
             if ((st = kprof_end(g))) return st;
-            bfs_commit<<<flat_grid(g, g->nw), kBlock, 0, s>>>(g->q + total, g->ctr + 1, g->V, nullptr, g->N,
-                                                               g->qbits + total, nullptr);
-            CU(cudaMemcpyAsync(g->h_ctr + 1, g->ctr + 1, 4, cudaMemcpyDeviceToHost, s));
+            launch_hub(g->P, hub_grid(g), s, c, app);
+            commit_dense<<<flat_grid(g, g->nw), kBlock, 0, s>>>(g->V, nullptr, g->N, 0, g->nw, g->q + total,
+                                                                 g->ctr + 2 + ((level + 1) & 1), g->qbits + total,
+                                                                 g->ctr + 2 + (level & 1), g->hub_ctr);
+            CU(cudaMemcpyAsync(g->h_ctr + 1, g->ctr + 2 + ((level + 1) & 1), 4, cudaMemcpyDeviceToHost, s));
             CU(cudaStreamSynchronize(s));
             if ((st = kprof_collect(g))) return st;
             total += g->h_ctr[1];
             level++;
         }
-        // lvl_off has D+2 entries: levels 0..D-1 plus the empty terminator
-        const int D = (int)lvl_off.size() - 2;
+        const int D = (int)lvl_off.size() - 2;  // levels 0..D-1
         for (int d = D - 1; d >= 0; d--) {
             const uint32_t off = lvl_off[d], qlen = lvl_off[d + 1] - off;
+            CU(cudaMemcpyAsync(g->ctr + 4, &qlen, 4, cudaMemcpyHostToDevice, s));
             int grid;
             uint32_t wpb;
             frontier_launch(g, qlen, &grid, &wpb);
-            GCGT_DISPATCH(g->P, bc_backward, grid, kBlock, s, g->W, g->offs, g->P.min_interval_len, seg_bits,
-                          (int32_t)d, g->q + off, g->qbits + off, qlen, src, g->levels, g->sigma, g->delta, g->bc, wpb,
-                          g->stats);
+            const QueueFront fr{g->q + off, g->ctr + 4, nullptr, g->qbits + off};
+            const BcBwdApp app{g->levels, g->sigma, g->delta, g->bc, d + 1, src, 0, 0.0, 0.0};
+            launch_expand(g->P, grid, s, c, fr, app, wpb);
+            launch_hub(g->P, hub_grid(g), s, c, app);
+            CU(cudaMemsetAsync(g->hub_ctr, 0, sizeof(unsigned long long), s));
         }
     }
     if ((st = copy_out(g, bc, g->bc, g->n * 8, placement))) return st;

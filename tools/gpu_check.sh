@@ -1,5 +1,6 @@
-set -x
-nproc; free -g | head -2; nvidia-smi --query-gpu=name,clocks.sm,clocks.max.sm --format=csv
-python -c "import __graft_entry__ as e; e.smoke()" 2>&1 | tail -5
-timeout 1500 python -m pytest tests -m gpu -x -q 2>&1 | tail -25
-timeout 900 python bench.py --steps 8 --warmup 3 > gpurun_out/bench1.json 2> gpurun_out/bench1.err; tail -3 gpurun_out/bench1.err; cat gpurun_out/bench1.json
+# usage: bash tools/gpu_check.sh [tag]   (run under gpurun from the repo root)
+TAG=${1:-run}
+mkdir -p gpurun_out
+python -c "import __graft_entry__ as e; e.smoke()" 2>&1 | tail -3
+timeout 1500 python -m pytest tests -m gpu -x -q 2>&1 | tail -15
+timeout 900 python bench.py --steps 8 --warmup 3 --no-cpu-baseline > gpurun_out/bench_$TAG.json 2> gpurun_out/bench_$TAG.err; tail -3 gpurun_out/bench_$TAG.err; cat gpurun_out/bench_$TAG.json
