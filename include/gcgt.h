@@ -133,6 +133,15 @@ gcgt_status gcgt_cc(gcgt_graph* g, uint32_t* labels, int out_placement, gcgt_sta
 gcgt_status gcgt_bc(gcgt_graph* g, const uint32_t* sources, uint32_t k, double* bc, int out_placement,
                     gcgt_stats* stats);
 
+/* ---- Test hook (parity pin of the warp decoder against Fig. 5 / Ex. 5.1) ------------------
+ * Runs the device warp-parallel decoder (Alg. 4 :901-919) on one warp over a caller bit array (host, MSB-first
+ * bytes, R1): vals[0..count-1] receive the first `count` codewords decoded from bit 0; the FIRST window step over
+ * `window` (16 or 32) lanes is traced: trace_pos / trace_flags (6 x 32 entries, row r = state after marking round
+ * r, row 0 = initial; 0xFFFFFFFF = Fig. 5's 'x') and *rounds = number of rows written.  Uses device 0. */
+gcgt_status gcgt_debug_warp_decode(const uint8_t* bytes, uint64_t nbits, uint32_t zeta_k, uint32_t window,
+                                   uint64_t count, uint64_t* vals, uint32_t* trace_pos, uint32_t* trace_flags,
+                                   uint32_t* rounds);
+
 /* Thread-local message for the last non-OK status returned on this thread ("" if none). */
 const char* gcgt_last_error(void);
 

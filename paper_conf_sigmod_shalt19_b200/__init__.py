@@ -23,7 +23,7 @@ OUT_HOST, OUT_DEVICE = 0, 1
 # public symbols of include/gcgt.h (tests check the library exports every one)
 ABI_SYMBOLS = ["gcgt_encode", "gcgt_cgr_view", "gcgt_cgr_from_arrays", "gcgt_cgr_save", "gcgt_cgr_open",
                "gcgt_cgr_free", "gcgt_load", "gcgt_unload", "gcgt_profile", "gcgt_graph_range", "gcgt_bfs", "gcgt_cc", "gcgt_bc",
-               "gcgt_last_error", "gcgt_version"]
+               "gcgt_debug_warp_decode", "gcgt_last_error", "gcgt_version"]
 
 
 class GcgtError(RuntimeError):
@@ -80,6 +80,7 @@ def lib():
         L.gcgt_bfs.argtypes = [p, u32, p, i32, C.POINTER(Stats)]
         L.gcgt_cc.argtypes = [p, p, i32, C.POINTER(Stats)]
         L.gcgt_bc.argtypes = [p, p, u32, p, i32, C.POINTER(Stats)]
+        L.gcgt_debug_warp_decode.argtypes = [p, u64, u32, u32, u64, p, p, p, C.POINTER(u32)]
         L.gcgt_last_error.restype = C.c_char_p
         L.gcgt_version.restype = C.c_char_p
         _lib = L
@@ -247,6 +248,22 @@ def cgr_n(cgr: CGR) -> int:
 
 def load(cgr: CGR, device: int = 0, stream=None, **kw) -> Graph:
     return Graph(cgr, device, stream, **kw)
+
+
+def debug_warp_decode(bytes_: np.ndarray, nbits: int, zeta_k: int, window: int, count: int):
+    """Test hook: (vals[count], trace_pos[rounds][window], trace_flags[rounds][window], rounds) from the device
+    warp decoder (gcgt_debug_warp_decode)."""
+    b = np.zeros(np.asarray(bytes_).size + 16, dtype=np.uint8)
+    b[: np.asarray(bytes_).size] = bytes_
+    vals = np.zeros(max(count, 1), dtype=np.uint64)
+    tp = np.zeros(6 * 32, dtype=np.uint32)
+    tf = np.zeros(6 * 32, dtype=np.uint32)
+    r = C.c_uint32(0)
+    _check(lib().gcgt_debug_warp_decode(_np_ptr(b), nbits, zeta_k, window, count, _np_ptr(vals), _np_ptr(tp),
+                                        _np_ptr(tf), C.byref(r)), "gcgt_debug_warp_decode")
+    n = r.value
+    return (vals[:count], tp.reshape(6, 32)[:n, :window].astype(np.int64), tf.reshape(6, 32)[:n, :window],
+            n)
 
 
 def version() -> str:

@@ -79,6 +79,7 @@ struct gcgt_graph {
     uint64_t qcap = 0;
     uint32_t* ctr = nullptr;    // device counters [8]
     HubEntry* hubq = nullptr;   // per-level hub queue (capacity = hub vertices + 1)
+    unsigned long long* cursor = nullptr;  // [0] work cursor, [1] finished-warp count (expand_kernel)
     unsigned long long* hub_ctr = nullptr;
     Stats* stats = nullptr;
     int32_t* levels = nullptr;
@@ -116,6 +117,7 @@ struct Ctx {
     HubEntry* hubq;
     unsigned long long* hub_ctr;  // (entries << 32) | segments
     Stats* st;
+    unsigned long long* cursor;   // work cursor over the frontier queue (reset per launch)
 };
 
 __device__ __forceinline__ void add_stats(Stats* st, uint64_t v, uint64_t a, uint64_t b) {
@@ -175,21 +177,111 @@ __device__ __forceinline__ uint32_t decode_segment(const uint64_t* __restrict__ 
 }
 
 // ---- the expansion engine -----------------------------------------------------------------------------------------
-// Phase A (lane per frontier vertex): App::vertex, then the record header and interval area (decoded serially,
-// each interval handed over as a range), then segNum.  Unsegmented records are decoded completely here.
-// Phase B (segmented format): the warp's segments are flattened with a warp scan and decoded one segment per lane
-// (each segment is self-contained, R17), so the lanes' work is bounded by 2 segBits bits regardless of degree.
-// Vertices with more than kHubSegs segments go to the hub queue (hub_kernel).
+// Work distribution: a persistent grid (one wave, sized by the occupancy calculator) whose warps grab `wpb` queue
+// words at a time from an atomic cursor (dynamic load balancing; no tail of idle SMs).  For each batch:
+// Phase A (lane per frontier vertex): App::vertex, the record header and the interval area (decoded serially, each
+//   interval handed over as a word-range claim), then segNum.  A vertex whose interval area (or unsegmented list)
+//   is long is deferred as "heavy".
+// Phase B (segmented format): the batch's segments are flattened with a warp scan and decoded one segment per
+//   lane (segments are self-contained, R17), so lane work is bounded by 2 segBits bits regardless of degree.
+//   Vertices with more than kHubSegs segments go to the hub queue (hub_kernel, whole grid).
+// Phase C: each heavy vertex is decoded by the whole warp with warp_decode (Alg. 4): intervals are paired and
+//   their starts recovered with a warp scan, residual ids likewise.
+constexpr uint32_t kHeavyItv = 8;    // interval count above which phase C takes the interval area
+constexpr uint32_t kHeavyRes = 64;   // unsegmented residual count above which phase C takes the list
+
+struct WarpSmem {
+    uint32_t w[32], b[32], pre[33];
+    uint32_t u[32], spre[33];
+    uint64_t base[32];
+    uint32_t hu[32], hitv[32], hdeg[32];
+    uint64_t hp[32];
+    uint64_t codes[64];
+};
+
+// Heavy vertex u (warp-uniform arguments), p = first bit after the itvNum field.
+template <int K, bool SEG, class App>
+__device__ __forceinline__ void heavy_vertex(const Ctx& c, const App& app, WarpSmem& sm, uint32_t u, uint64_t p,
+                                             uint64_t itv, uint64_t deg, uint64_t& na) {
+    const uint32_t lane = lane_id();
+    App t = app;
+    t.begin(u);
+    int64_t prev_end = 0;        // warp-uniform
+    uint64_t pairs_done = 0, in_itv = 0;
+    p = warp_decode<K>(c.W, p, 2 * itv, [&](uint64_t base, uint32_t take, uint64_t idx, uint64_t v, bool act) {
+        if (act) sm.codes[idx & 63] = v;
+        __syncwarp();
+        const uint64_t npairs = (base + take) / 2 - pairs_done;
+        if (npairs) {
+            const uint64_t j = pairs_done + lane;
+            const bool has = lane < npairs;
+            uint64_t len = 0;
+            int64_t a = 0;
+            if (has) {
+                const uint64_t g = sm.codes[(2 * j) & 63];
+                len = sm.codes[(2 * j + 1) & 63] - 1 + c.min_len;
+                a = j == 0 ? unmap_first(u, g) + (int64_t)len - 1 : (int64_t)g + (int64_t)len - 1;
+            }
+            int64_t incl = a;
+            for (int o = 1; o < 32; o <<= 1) {
+                const int64_t tt = __shfl_up_sync(0xffffffffu, incl, o);
+                if (lane >= (uint32_t)o) incl += tt;
+            }
+            if (has) {
+                const int64_t end = prev_end + incl;
+                t.range((uint32_t)(end - (int64_t)len + 1), (uint32_t)len);
+                in_itv += len;
+            }
+            prev_end += __shfl_sync(0xffffffffu, incl, (int)npairs - 1);
+            pairs_done += npairs;
+        }
+        __syncwarp();
+    });
+    na += in_itv;
+    if (SEG) {
+        uint64_t q = p;
+        const uint64_t nseg = decode<K>(c.W, q) - 1;  // every lane decodes the same field
+        if (nseg > kHubSegs) {
+            if (lane == 0) {
+                const unsigned long long old = atomicAdd(c.hub_ctr, (1ull << 32) | (unsigned long long)nseg);
+                c.hubq[old >> 32] = HubEntry{q, u, (uint32_t)(old & 0xffffffffu)};
+            }
+        } else if (lane < nseg) {
+            na += decode_segment<K>(c.W, q + (uint64_t)lane * c.seg_bits, u, t);
+        }
+    } else {
+        uint64_t tot_itv = in_itv;
+        for (int o = 16; o; o >>= 1) tot_itv += __shfl_xor_sync(0xffffffffu, tot_itv, o);
+        const uint64_t nres = deg - tot_itv;
+        int64_t cur = 0;  // warp-uniform: last residual id
+        warp_decode<K>(c.W, p, nres, [&](uint64_t base, uint32_t take, uint64_t idx, uint64_t v, bool act) {
+            int64_t a = 0;
+            if (act) a = idx == 0 ? unmap_first(u, v) : (int64_t)v;
+            int64_t incl = a;
+            for (int o = 1; o < 32; o <<= 1) {
+                const int64_t tt = __shfl_up_sync(0xffffffffu, incl, o);
+                if (lane >= (uint32_t)o) incl += tt;
+            }
+            if (act) t.one((uint32_t)(cur + incl));
+            cur += __shfl_sync(0xffffffffu, incl, 31);
+        });
+        if (lane == 0) na += nres;
+    }
+    t.end();
+}
+
 template <int K, bool SEG, class App, class Front>
 __global__ void __launch_bounds__(kBlock) expand_kernel(Ctx c, Front fr, App app, uint32_t wpb) {
-    __shared__ uint32_t s_w[kWarps][32], s_b[kWarps][32], s_pre[kWarps][33];
-    __shared__ uint32_t s_u[kWarps][32], s_spre[kWarps][33];
-    __shared__ uint64_t s_base[kWarps][32];
+    __shared__ WarpSmem smem[kWarps];
     const uint32_t wid = threadIdx.x >> 5, lane = lane_id();
-    const uint64_t gw = (uint64_t)blockIdx.x * kWarps + wid, nwarps = (uint64_t)gridDim.x * kWarps;
+    WarpSmem& sm = smem[wid];
     const uint64_t qlen = fr.size();
     uint64_t nv = 0, na = 0, nb = 0;
-    for (uint64_t base = gw * wpb; base < qlen; base += nwarps * wpb) {
+    for (;;) {
+        uint64_t base = 0;
+        if (lane == 0) base = atomicAdd(c.cursor, (unsigned long long)wpb);
+        base = __shfl_sync(0xffffffffu, base, 0);
+        if (base >= qlen) break;
         uint32_t w = 0, bits = 0;
         if (lane < wpb && base + lane < qlen) fr.get(base + lane, w, bits);
         uint32_t incl = __popc(bits);
@@ -197,24 +289,25 @@ __global__ void __launch_bounds__(kBlock) expand_kernel(Ctx c, Front fr, App app
             const uint32_t t = __shfl_up_sync(0xffffffffu, incl, o);
             if (lane >= (uint32_t)o) incl += t;
         }
-        s_w[wid][lane] = w;
-        s_b[wid][lane] = bits;
-        s_pre[wid][lane + 1] = incl;
-        if (lane == 0) s_pre[wid][0] = 0;
+        sm.w[lane] = w;
+        sm.b[lane] = bits;
+        sm.pre[lane + 1] = incl;
+        if (lane == 0) sm.pre[0] = 0;
         __syncwarp();
-        const uint32_t total = s_pre[wid][32];
+        const uint32_t total = sm.pre[32];
         for (uint32_t t0 = 0; t0 < total; t0 += 32) {
             // ---- phase A
             const uint32_t j = t0 + lane;
             uint32_t nseg = 0, u = 0;
-            uint64_t segbase = 0;
+            uint64_t segbase = 0, hp = 0, hitv = 0, hdeg = 0;
+            bool heavy = false;
             if (j < total) {
-                uint32_t lo = 0, hi = 31;  // owner lane: largest o with s_pre[o] <= j
+                uint32_t lo = 0, hi = 31;  // owner lane: largest o with pre[o] <= j
                 while (lo < hi) {
                     const uint32_t mid = (lo + hi + 1) >> 1;
-                    if (s_pre[wid][mid] <= j) lo = mid; else hi = mid - 1;
+                    if (sm.pre[mid] <= j) lo = mid; else hi = mid - 1;
                 }
-                u = s_w[wid][lo] * 32 + __fns(s_b[wid][lo], 0, (int)(j - s_pre[wid][lo]) + 1);
+                u = sm.w[lo] * 32 + __fns(sm.b[lo], 0, (int)(j - sm.pre[lo]) + 1);
                 uint64_t p = ldg64(c.offs + u);
                 nb += ldg64(c.offs + u + 1) - p;
                 nv++;
@@ -224,72 +317,100 @@ __global__ void __launch_bounds__(kBlock) expand_kernel(Ctx c, Front fr, App app
                 uint64_t deg = 0;
                 if (!SEG) deg = decode<K>(c.W, p) - 1;
                 const uint64_t itv = decode<K>(c.W, p) - 1;
-                int64_t prev_end = 0;
-                uint64_t in_itv = 0;
-                for (uint64_t i = 0; i < itv; i++) {
-                    const uint64_t g = decode<K>(c.W, p);
-                    const uint64_t len = decode<K>(c.W, p) - 1 + c.min_len;
-                    const int64_t start = i == 0 ? unmap_first(u, g) : prev_end + (int64_t)g;
-                    t.range((uint32_t)start, (uint32_t)len);
-                    prev_end = start + (int64_t)len - 1;
-                    in_itv += len;
-                }
-                na += in_itv;
-                if (!SEG) {
-                    const uint64_t nres = deg - in_itv;
-                    int64_t cur = 0;
-                    for (uint64_t i = 0; i < nres; i++) {
-                        const uint64_t cd = decode<K>(c.W, p);
-                        cur = i == 0 ? unmap_first(u, cd) : cur + (int64_t)cd;
-                        t.one((uint32_t)cur);
-                    }
-                    na += nres;
+                if (itv > kHeavyItv || (!SEG && deg > kHeavyRes)) {
+                    heavy = true;
+                    hp = p;
+                    hitv = itv;
+                    hdeg = deg;
                 } else {
-                    nseg = (uint32_t)(decode<K>(c.W, p) - 1);
-                    segbase = p;
-                    if (nseg > kHubSegs) {  // hub: hand the segments to the whole grid
-                        const unsigned long long old = atomicAdd(c.hub_ctr, (1ull << 32) | (unsigned long long)nseg);
-                        c.hubq[old >> 32] = HubEntry{segbase, u, (uint32_t)(old & 0xffffffffu)};
-                        nseg = 0;
+                    int64_t prev_end = 0;
+                    uint64_t in_itv = 0;
+                    for (uint64_t i = 0; i < itv; i++) {
+                        const uint64_t g = decode<K>(c.W, p);
+                        const uint64_t len = decode<K>(c.W, p) - 1 + c.min_len;
+                        const int64_t start = i == 0 ? unmap_first(u, g) : prev_end + (int64_t)g;
+                        t.range((uint32_t)start, (uint32_t)len);
+                        prev_end = start + (int64_t)len - 1;
+                        in_itv += len;
                     }
+                    na += in_itv;
+                    if (!SEG) {
+                        const uint64_t nres = deg - in_itv;
+                        int64_t cur = 0;
+                        for (uint64_t i = 0; i < nres; i++) {
+                            const uint64_t cd = decode<K>(c.W, p);
+                            cur = i == 0 ? unmap_first(u, cd) : cur + (int64_t)cd;
+                            t.one((uint32_t)cur);
+                        }
+                        na += nres;
+                    } else {
+                        nseg = (uint32_t)(decode<K>(c.W, p) - 1);
+                        segbase = p;
+                        if (nseg > kHubSegs) {  // hub: hand the segments to the whole grid
+                            const unsigned long long old =
+                                atomicAdd(c.hub_ctr, (1ull << 32) | (unsigned long long)nseg);
+                            c.hubq[old >> 32] = HubEntry{segbase, u, (uint32_t)(old & 0xffffffffu)};
+                            nseg = 0;
+                        }
+                    }
+                    t.end();
                 }
-                t.end();
+            }
+            const uint32_t hbal = __ballot_sync(0xffffffffu, heavy);
+            if (heavy) {
+                const uint32_t r = __popc(hbal & lanemask_lt());
+                sm.hu[r] = u;
+                sm.hp[r] = hp;
+                sm.hitv[r] = (uint32_t)hitv;
+                sm.hdeg[r] = (uint32_t)hdeg;
             }
             if (SEG) {
-                // ---- phase B: flatten the warp's segments and decode one per lane
+                // ---- phase B: flatten the batch's segments and decode one per lane
                 uint32_t sincl = nseg;
                 for (int o = 1; o < 32; o <<= 1) {
                     const uint32_t tt = __shfl_up_sync(0xffffffffu, sincl, o);
                     if (lane >= (uint32_t)o) sincl += tt;
                 }
-                s_u[wid][lane] = u;
-                s_base[wid][lane] = segbase;
-                s_spre[wid][lane + 1] = sincl;
-                if (lane == 0) s_spre[wid][0] = 0;
+                sm.u[lane] = u;
+                sm.base[lane] = segbase;
+                sm.spre[lane + 1] = sincl;
+                if (lane == 0) sm.spre[0] = 0;
                 __syncwarp();
-                const uint32_t stotal = s_spre[wid][32];
+                const uint32_t stotal = sm.spre[32];
                 for (uint32_t k0 = 0; k0 < stotal; k0 += 32) {
                     const uint32_t sj = k0 + lane;
                     if (sj < stotal) {
                         uint32_t lo = 0, hi = 31;
                         while (lo < hi) {
                             const uint32_t mid = (lo + hi + 1) >> 1;
-                            if (s_spre[wid][mid] <= sj) lo = mid; else hi = mid - 1;
+                            if (sm.spre[mid] <= sj) lo = mid; else hi = mid - 1;
                         }
-                        const uint32_t su = s_u[wid][lo];
+                        const uint32_t su = sm.u[lo];
                         App t = app;
                         t.begin(su);
-                        na += decode_segment<K>(c.W, s_base[wid][lo] + (uint64_t)(sj - s_spre[wid][lo]) * c.seg_bits,
-                                                su, t);
+                        na += decode_segment<K>(c.W, sm.base[lo] + (uint64_t)(sj - sm.spre[lo]) * c.seg_bits, su, t);
                         t.end();
                     }
                 }
-                __syncwarp();
             }
+            __syncwarp();
+            // ---- phase C: heavy vertices, one at a time, whole warp
+            const uint32_t nh = __popc(hbal);
+            for (uint32_t h = 0; h < nh; h++)
+                heavy_vertex<K, SEG>(c, app, sm, sm.hu[h], sm.hp[h], sm.hitv[h], sm.hdeg[h], na);
+            __syncwarp();
         }
         __syncwarp();
     }
     add_stats(c.st, nv, na, nb);
+    // the last warp out resets the work cursor for the next launch
+    if (lane == 0) {
+        const unsigned long long nw = (unsigned long long)gridDim.x * kWarps;
+        if (atomicAdd(c.cursor + 1, 1ull) == nw - 1) {
+            c.cursor[0] = 0;
+            c.cursor[1] = 0;
+        }
+    }
 }
 
 // Hub segments of the level, flattened over the whole grid (one segment per thread at a time).
@@ -519,8 +640,19 @@ __global__ void count_hubs(const uint64_t* __restrict__ W, const uint64_t* __res
 }
 
 // ---- dispatch -------------------------------------------------------------------------------------------------------
+// Persistent launch: at most one wave (occupancy calculator), never more blocks than the work needs.
 template <int K, bool SEG, class App, class Front>
 inline void launch_expand_k(int grid, cudaStream_t s, const Ctx& c, const Front& fr, const App& app, uint32_t wpb) {
+    static int per_sm = 0;
+    static int sms = 0;
+    if (!per_sm) {
+        int dev = 0;
+        cudaGetDevice(&dev);
+        cudaDeviceGetAttribute(&sms, cudaDevAttrMultiProcessorCount, dev);
+        cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per_sm, expand_kernel<K, SEG, App, Front>, kBlock, 0);
+        if (per_sm < 1) per_sm = 1;
+    }
+    grid = std::max(1, std::min(grid, per_sm * sms));
     expand_kernel<K, SEG, App, Front><<<grid, kBlock, 0, s>>>(c, fr, app, wpb);
 }
 
@@ -549,15 +681,15 @@ inline void launch_hub(const gcgt_params& P, int grid, cudaStream_t s, const Ctx
     }
 }
 
-// Grid for a frontier of qlen words: ~1 word per warp when the queue is small, up to 32 per warp batch otherwise.
+// Work granularity for a frontier of qlen words: every resident warp should take several batches (dynamic
+// balancing); small frontiers get one word per batch and only as many blocks as there are words.
 inline void frontier_launch(const gcgt_graph* g, uint64_t qlen, int* grid, uint32_t* wpb) {
-    const uint64_t max_warps = (uint64_t)g->num_sms * 2048 / 32;  // one wave at full occupancy
-    uint32_t b = 1;
-    while (b < 32 && qlen > max_warps * b) b <<= 1;
+    const uint64_t resident_warps = (uint64_t)g->num_sms * 48;
+    uint64_t b = qlen / (resident_warps * 4);
+    b = std::max<uint64_t>(1, std::min<uint64_t>(b, 16));
     const uint64_t warps = (qlen + b - 1) / b;
-    const uint64_t blocks = std::max<uint64_t>(1, (warps + kWarps - 1) / kWarps);
-    *grid = (int)std::min<uint64_t>(blocks, (uint64_t)g->num_sms * 8);
-    *wpb = b;
+    *grid = (int)std::max<uint64_t>(1, std::min<uint64_t>((warps + kWarps - 1) / kWarps, (uint64_t)g->num_sms * 32));
+    *wpb = (uint32_t)b;
 }
 
 inline int flat_grid(const gcgt_graph* g, uint64_t n) {
@@ -567,7 +699,8 @@ inline int flat_grid(const gcgt_graph* g, uint64_t n) {
 inline int hub_grid(const gcgt_graph* g) { return g->num_sms * 4; }
 
 inline Ctx make_ctx(const gcgt_graph* g) {
-    return Ctx{g->W, g->offs, g->P.min_interval_len, 8 * g->P.residual_segment_len, g->hubq, g->hub_ctr, g->stats};
+    return Ctx{g->W,     g->offs,     g->P.min_interval_len, 8 * g->P.residual_segment_len,
+               g->hubq, g->hub_ctr, g->stats,              g->cursor};
 }
 
 gcgt_status copy_out(gcgt_graph* g, void* dst, const void* src, size_t bytes, int placement) {
@@ -641,7 +774,7 @@ extern "C" void gcgt_unload(gcgt_graph* g) {
     cudaSetDevice(g->device);
     if (g->stream) cudaStreamSynchronize(g->stream);
     cudaFree(g->W); cudaFree(g->offs); cudaFree(g->V); cudaFree(g->F); cudaFree(g->N); cudaFree(g->q);
-    cudaFree(g->qbits); cudaFree(g->ctr); cudaFree(g->hubq); cudaFree(g->hub_ctr); cudaFree(g->stats); cudaFree(g->levels); cudaFree(g->parent);
+    cudaFree(g->qbits); cudaFree(g->ctr); cudaFree(g->hubq); cudaFree(g->hub_ctr); cudaFree(g->cursor); cudaFree(g->stats); cudaFree(g->levels); cudaFree(g->parent);
     cudaFree(g->sigma); cudaFree(g->delta); cudaFree(g->bc);
     if (g->h_ctr) cudaFreeHost(g->h_ctr);
     if (g->h_stats) cudaFreeHost(g->h_stats);
@@ -698,7 +831,8 @@ extern "C" gcgt_status gcgt_load(const gcgt_cgr* c, const gcgt_load_opts* opts, 
                        g->stream));
     bswap_words<<<flat_grid(g.get(), nwords), kBlock, 0, g->stream>>>(g->W, nwords);
     CU(cudaMemsetAsync(g->N, 0, g->nw * 4, g->stream));
-    if ((st = dalloc(&g->hub_ctr, 1))) return st;
+    if ((st = dalloc(&g->hub_ctr, 1)) || (st = dalloc(&g->cursor, 2))) return st;
+    CU(cudaMemsetAsync(g->cursor, 0, 16, g->stream));
     uint64_t nhubs = 0;
     if (g->P.residual_segment_len) {
         CU(cudaMemsetAsync(g->hub_ctr, 0, 8, g->stream));
@@ -718,6 +852,69 @@ extern "C" gcgt_status gcgt_load(const gcgt_cgr* c, const gcgt_load_opts* opts, 
     CU(cudaStreamSynchronize(g->stream));
     CU(cudaGetLastError());
     *out = g.release();
+    return GCGT_OK;
+}
+
+// ---- test hook: the warp decoder on a caller bit array (Fig. 5 pin) --------------------------------------------------
+namespace {
+template <int K, int WIN>
+__global__ void debug_warp_decode_kernel(const uint64_t* W, uint64_t count, uint64_t* vals, uint32_t* tpos,
+                                         uint32_t* tflags, uint32_t* rounds) {
+    uint64_t v;
+    uint32_t len;
+    window_step<K, WIN, true>(W, 0, v, len, tpos, tflags, rounds);
+    warp_decode<K>(W, 0, count, [&](uint64_t, uint32_t, uint64_t idx, uint64_t val, bool act) {
+        if (act) vals[idx] = val;
+    });
+}
+
+template <int K>
+void launch_debug(uint32_t win, const uint64_t* W, uint64_t count, uint64_t* vals, uint32_t* tp, uint32_t* tf,
+                  uint32_t* r) {
+    if (win == 16) debug_warp_decode_kernel<K, 16><<<1, 32>>>(W, count, vals, tp, tf, r);
+    else debug_warp_decode_kernel<K, 32><<<1, 32>>>(W, count, vals, tp, tf, r);
+}
+}  // namespace
+
+extern "C" gcgt_status gcgt_debug_warp_decode(const uint8_t* bytes, uint64_t nbits, uint32_t zeta_k, uint32_t window,
+                                              uint64_t count, uint64_t* vals, uint32_t* trace_pos,
+                                              uint32_t* trace_flags, uint32_t* rounds) {
+    gcgt_internal::clear_error();
+    if (!bytes || !vals || !trace_pos || !trace_flags || !rounds) return fail(GCGT_EINVAL, "null argument");
+    if (zeta_k < 1 || zeta_k > 5 || (window != 16 && window != 32)) return fail(GCGT_EINVAL, "bad zeta_k / window");
+    int ndev = 0;
+    if (cudaGetDeviceCount(&ndev) != cudaSuccess || ndev == 0) return fail(GCGT_ECUDA, "no CUDA device");
+    const uint64_t nwords = (nbits + 63) / 64 + 4;
+    std::vector<uint64_t> h(nwords, 0);
+    memcpy(h.data(), bytes, (nbits + 7) / 8);
+    for (auto& x : h) x = __builtin_bswap64(x);
+    uint64_t *dW = nullptr, *dv = nullptr;
+    uint32_t *dp = nullptr, *df = nullptr, *dr = nullptr;
+    gcgt_status st = GCGT_OK;
+    if ((st = dalloc(&dW, nwords)) || (st = dalloc(&dv, count + 1)) || (st = dalloc(&dp, 6 * 32)) ||
+        (st = dalloc(&df, 6 * 32)) || (st = dalloc(&dr, 1))) {
+        cudaFree(dW); cudaFree(dv); cudaFree(dp); cudaFree(df); cudaFree(dr);
+        return st;
+    }
+    cudaMemcpy(dW, h.data(), nwords * 8, cudaMemcpyHostToDevice);
+    cudaMemset(dp, 0xff, 6 * 32 * 4);
+    cudaMemset(df, 0, 6 * 32 * 4);
+    switch (zeta_k) {
+        case 1: launch_debug<1>(window, dW, count, dv, dp, df, dr); break;
+        case 2: launch_debug<2>(window, dW, count, dv, dp, df, dr); break;
+        case 3: launch_debug<3>(window, dW, count, dv, dp, df, dr); break;
+        case 4: launch_debug<4>(window, dW, count, dv, dp, df, dr); break;
+        default: launch_debug<5>(window, dW, count, dv, dp, df, dr); break;
+    }
+    cudaError_t e = cudaDeviceSynchronize();
+    if (e == cudaSuccess) {
+        cudaMemcpy(vals, dv, count * 8, cudaMemcpyDeviceToHost);
+        cudaMemcpy(trace_pos, dp, 6 * 32 * 4, cudaMemcpyDeviceToHost);
+        cudaMemcpy(trace_flags, df, 6 * 32 * 4, cudaMemcpyDeviceToHost);
+        e = cudaMemcpy(rounds, dr, 4, cudaMemcpyDeviceToHost);
+    }
+    cudaFree(dW); cudaFree(dv); cudaFree(dp); cudaFree(df); cudaFree(dr);
+    if (e != cudaSuccess) return fail(GCGT_ECUDA, cudaGetErrorString(e));
     return GCGT_OK;
 }
 

@@ -164,3 +164,33 @@ def test_c2_full_size_bench_launch():
     for r in synth.pick_roots(ro, 2):
         assert np.array_equal(g.bfs(r), O.bfs(ro, co, r)), r
     assert np.array_equal(g.cc(), O.cc(ro, co))
+
+
+# ---------------------------------------------------------------------------------------------------------------------
+# The device warp decoder (Alg. 4 analogue) pinned against the paper's Fig. 5 and against serial decoding
+# ---------------------------------------------------------------------------------------------------------------------
+def test_warp_decoder_fig5_trace(golden):
+    """Fig. 5: 16 threads, gamma, bit array of 1..5.  The device trace must reproduce every
+    printed poss / flags row and the decoded values 1..5."""
+    g = golden("fig5.txt")
+    b, nb = O.bits_to_bytes(g["bits"][0])
+    vals, tpos, tflags, rounds = G.debug_warp_decode(b, nb, 1, 16, 5)
+    assert list(vals) == [1, 2, 3, 4, 5]
+    assert rounds == 4
+    X = 0xFFFFFFFF
+    for r in range(4):
+        exp = [X if t == "x" else int(t) for t in g[f"poss{r}"]]
+        assert [int(x) for x in tpos[r]] == exp, r
+        assert [int(x) for x in tflags[r]] == [int(t) for t in g[f"flags{r}"]], r
+
+
+@pytest.mark.parametrize("k", [1, 2, 3, 4, 5])
+def test_warp_decoder_random_streams(k):
+    rng = np.random.default_rng(77 + k)
+    for trial in range(6):
+        hi = [2, 8, 1 << 10, 1 << 20, 1 << 33, 1 << 40][trial]
+        xs = [int(x) for x in rng.integers(1, hi, size=500)]
+        bits = "".join(O.vlc_string(k, x) for x in xs)
+        b, nb = O.bits_to_bytes(bits)
+        vals, _, _, _ = G.debug_warp_decode(b, nb, k, 32, len(xs))
+        assert [int(v) for v in vals] == xs, (k, trial)
