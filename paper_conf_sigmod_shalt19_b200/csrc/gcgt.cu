@@ -62,6 +62,13 @@ struct HubEntry {
     uint32_t seg_off;  // first flattened segment index of this entry (entries are ordered by seg_off)
 };
 
+struct HeavyEntry {
+    uint64_t p;    // first bit after the itvNum field
+    uint32_t u;
+    uint32_t itv;  // interval count
+    uint64_t deg;  // unsegmented records: degree (else 0)
+};
+
 struct gcgt_graph {
     int device = 0;
     cudaStream_t stream = nullptr;
@@ -80,6 +87,8 @@ struct gcgt_graph {
     uint32_t* ctr = nullptr;    // device counters [8]
     HubEntry* hubq = nullptr;   // per-level hub queue (capacity = hub vertices + 1)
     unsigned long long* cursor = nullptr;  // [0] work cursor, [1] finished-warp count (expand_kernel)
+    HeavyEntry* heavyq = nullptr;          // per-level heavy-vertex queue (capacity = heavy vertices + 1)
+    uint32_t* heavy_len = nullptr;
     unsigned long long* hub_ctr = nullptr;
     Stats* stats = nullptr;
     int32_t* levels = nullptr;
@@ -118,6 +127,8 @@ struct Ctx {
     unsigned long long* hub_ctr;  // (entries << 32) | segments
     Stats* st;
     unsigned long long* cursor;   // work cursor over the frontier queue (reset per launch)
+    HeavyEntry* heavyq;           // per-level heavy-vertex queue
+    uint32_t* heavy_len;
 };
 
 __device__ __forceinline__ void add_stats(Stats* st, uint64_t v, uint64_t a, uint64_t b) {
@@ -185,23 +196,25 @@ __device__ __forceinline__ uint32_t decode_segment(const uint64_t* __restrict__ 
 // Phase B (segmented format): the batch's segments are flattened with a warp scan and decoded one segment per
 //   lane (segments are self-contained, R17), so lane work is bounded by 2 segBits bits regardless of degree.
 //   Vertices with more than kHubSegs segments go to the hub queue (hub_kernel, whole grid).
-// Phase C: each heavy vertex is decoded by the whole warp with warp_decode (Alg. 4): intervals are paired and
-//   their starts recovered with a warp scan, residual ids likewise.
-constexpr uint32_t kHeavyItv = 8;    // interval count above which phase C takes the interval area
-constexpr uint32_t kHeavyRes = 64;   // unsegmented residual count above which phase C takes the list
+// Heavy vertices (long interval area, or long unsegmented list) go to the level's heavy queue; heavy_kernel then
+//   decodes each with a whole warp via warp_decode (Alg. 4): intervals are paired and their starts recovered
+//   with a warp scan, residual ids likewise.
+constexpr uint32_t kHeavyItv = 16;   // interval count above which the heavy kernel takes the interval area
+constexpr uint32_t kHeavyRes = 64;   // unsegmented residual count above which the heavy kernel takes the list
 
 struct WarpSmem {
     uint32_t w[32], b[32], pre[33];
     uint32_t u[32], spre[33];
     uint64_t base[32];
-    uint32_t hu[32], hitv[32], hdeg[32];
-    uint64_t hp[32];
+};
+
+struct HeavySmem {
     uint64_t codes[64];
 };
 
 // Heavy vertex u (warp-uniform arguments), p = first bit after the itvNum field.
 template <int K, bool SEG, class App>
-__device__ __forceinline__ void heavy_vertex(const Ctx& c, const App& app, WarpSmem& sm, uint32_t u, uint64_t p,
+__device__ __forceinline__ void heavy_vertex(const Ctx& c, const App& app, HeavySmem& sm, uint32_t u, uint64_t p,
                                              uint64_t itv, uint64_t deg, uint64_t& na) {
     const uint32_t lane = lane_id();
     App t = app;
@@ -271,7 +284,7 @@ __device__ __forceinline__ void heavy_vertex(const Ctx& c, const App& app, WarpS
 }
 
 template <int K, bool SEG, class App, class Front>
-__global__ void __launch_bounds__(kBlock) expand_kernel(Ctx c, Front fr, App app, uint32_t wpb) {
+__global__ void __launch_bounds__(kBlock, 6) expand_kernel(Ctx c, Front fr, App app, uint32_t wpb) {
     __shared__ WarpSmem smem[kWarps];
     const uint32_t wid = threadIdx.x >> 5, lane = lane_id();
     WarpSmem& sm = smem[wid];
@@ -299,8 +312,7 @@ __global__ void __launch_bounds__(kBlock) expand_kernel(Ctx c, Front fr, App app
             // ---- phase A
             const uint32_t j = t0 + lane;
             uint32_t nseg = 0, u = 0;
-            uint64_t segbase = 0, hp = 0, hitv = 0, hdeg = 0;
-            bool heavy = false;
+            uint64_t segbase = 0;
             if (j < total) {
                 uint32_t lo = 0, hi = 31;  // owner lane: largest o with pre[o] <= j
                 while (lo < hi) {
@@ -317,11 +329,12 @@ __global__ void __launch_bounds__(kBlock) expand_kernel(Ctx c, Front fr, App app
                 uint64_t deg = 0;
                 if (!SEG) deg = decode<K>(c.W, p) - 1;
                 const uint64_t itv = decode<K>(c.W, p) - 1;
-                if (itv > kHeavyItv || (!SEG && deg > kHeavyRes)) {
-                    heavy = true;
-                    hp = p;
-                    hitv = itv;
-                    hdeg = deg;
+                if (itv > kHeavyItv || (!SEG && deg > kHeavyRes)) {  // heavy: the whole grid takes it later
+                    cg::coalesced_group grp = cg::coalesced_threads();
+                    uint32_t slot = 0;
+                    if (grp.thread_rank() == 0) slot = atomicAdd(c.heavy_len, grp.size());
+                    slot = grp.shfl(slot, 0) + grp.thread_rank();
+                    c.heavyq[slot] = HeavyEntry{p, u, (uint32_t)itv, deg};
                 } else {
                     int64_t prev_end = 0;
                     uint64_t in_itv = 0;
@@ -356,14 +369,6 @@ __global__ void __launch_bounds__(kBlock) expand_kernel(Ctx c, Front fr, App app
                     t.end();
                 }
             }
-            const uint32_t hbal = __ballot_sync(0xffffffffu, heavy);
-            if (heavy) {
-                const uint32_t r = __popc(hbal & lanemask_lt());
-                sm.hu[r] = u;
-                sm.hp[r] = hp;
-                sm.hitv[r] = (uint32_t)hitv;
-                sm.hdeg[r] = (uint32_t)hdeg;
-            }
             if (SEG) {
                 // ---- phase B: flatten the batch's segments and decode one per lane
                 uint32_t sincl = nseg;
@@ -394,11 +399,6 @@ __global__ void __launch_bounds__(kBlock) expand_kernel(Ctx c, Front fr, App app
                 }
             }
             __syncwarp();
-            // ---- phase C: heavy vertices, one at a time, whole warp
-            const uint32_t nh = __popc(hbal);
-            for (uint32_t h = 0; h < nh; h++)
-                heavy_vertex<K, SEG>(c, app, sm, sm.hu[h], sm.hp[h], sm.hitv[h], sm.hdeg[h], na);
-            __syncwarp();
         }
         __syncwarp();
     }
@@ -411,6 +411,20 @@ __global__ void __launch_bounds__(kBlock) expand_kernel(Ctx c, Front fr, App app
             c.cursor[1] = 0;
         }
     }
+}
+
+// Heavy vertices of the level: one warp per vertex (warp_decode), warps strided over the queue.
+template <int K, bool SEG, class App>
+__global__ void __launch_bounds__(kBlock) heavy_kernel(Ctx c, App app) {
+    __shared__ HeavySmem smem[kWarps];
+    const uint32_t nh = *c.heavy_len;
+    uint64_t na = 0;
+    for (uint64_t h = ((uint64_t)blockIdx.x * blockDim.x + threadIdx.x) >> 5; h < nh;
+         h += ((uint64_t)gridDim.x * blockDim.x) >> 5) {
+        const HeavyEntry e = c.heavyq[h];
+        heavy_vertex<K, SEG>(c, app, smem[threadIdx.x >> 5], e.u, e.p, e.itv, e.deg, na);
+    }
+    add_stats(c.st, 0, na, 0);
 }
 
 // Hub segments of the level, flattened over the whole grid (one segment per thread at a time).
@@ -579,7 +593,7 @@ __global__ void cc_init(uint32_t* parent, uint64_t n) {
 __global__ void commit_dense(uint32_t* __restrict__ V, uint32_t* __restrict__ F, uint32_t* __restrict__ N,
                              uint64_t w_lo, uint64_t w_hi, uint32_t* __restrict__ qn, uint32_t* __restrict__ qn_len,
                              uint32_t* __restrict__ qbits_out, uint32_t* __restrict__ reset_ctr,
-                             unsigned long long* __restrict__ hub_ctr) {
+                             unsigned long long* __restrict__ hub_ctr, uint32_t* __restrict__ heavy_len) {
     const uint32_t lane = lane_id();
     const uint64_t gw = ((uint64_t)blockIdx.x * blockDim.x + threadIdx.x) >> 5;
     const uint64_t nwarps = ((uint64_t)gridDim.x * blockDim.x) >> 5;
@@ -608,6 +622,7 @@ __global__ void commit_dense(uint32_t* __restrict__ V, uint32_t* __restrict__ F,
     if (blockIdx.x == 0 && threadIdx.x == 0) {
         if (reset_ctr) *reset_ctr = 0;
         if (hub_ctr) *hub_ctr = 0;
+        if (heavy_len) *heavy_len = 0;
     }
 }
 
@@ -624,19 +639,31 @@ __global__ void bswap_words(uint64_t* w, uint64_t n) {
         w[i] = __byte_perm((uint32_t)(w[i] >> 32), 0, 0x0123) | ((uint64_t)__byte_perm((uint32_t)w[i], 0, 0x0123) << 32);
 }
 
-// Load-time pass: number of hub vertices (more than kHubSegs residual segments); sizes the hub queue.
-template <int K>
-__global__ void count_hubs(const uint64_t* __restrict__ W, const uint64_t* __restrict__ offs, uint32_t min_len,
-                           uint64_t n, unsigned long long* out) {
-    uint32_t cnt = 0;
+// Load-time pass: number of hub vertices (more than kHubSegs residual segments) and heavy vertices (long
+// interval area / unsegmented list); sizes the per-level hub and heavy queues.
+template <int K, bool SEG>
+__global__ void count_special(const uint64_t* __restrict__ W, const uint64_t* __restrict__ offs, uint64_t n,
+                              unsigned long long* out) {
+    uint32_t hubs = 0, heavy = 0;
     for (uint64_t u = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; u < n; u += (uint64_t)gridDim.x * blockDim.x) {
         uint64_t p = ldg64(offs + u);
+        uint64_t deg = 0;
+        if (!SEG) deg = decode<K>(W, p) - 1;
         const uint64_t itv = decode<K>(W, p) - 1;
-        for (uint64_t i = 0; i < 2 * itv; i++) decode<K>(W, p);
-        if (decode<K>(W, p) - 1 > kHubSegs) cnt++;
+        if (itv > kHeavyItv || (!SEG && deg > kHeavyRes)) heavy++;
+        if (SEG) {
+            for (uint64_t i = 0; i < 2 * itv; i++) decode<K>(W, p);
+            if (decode<K>(W, p) - 1 > kHubSegs) hubs++;
+        }
     }
-    for (int o = 16; o; o >>= 1) cnt += __shfl_xor_sync(0xffffffffu, cnt, o);
-    if (lane_id() == 0 && cnt) atomicAdd(out, (unsigned long long)cnt);
+    for (int o = 16; o; o >>= 1) {
+        hubs += __shfl_xor_sync(0xffffffffu, hubs, o);
+        heavy += __shfl_xor_sync(0xffffffffu, heavy, o);
+    }
+    if (lane_id() == 0) {
+        if (hubs) atomicAdd(out, (unsigned long long)hubs);
+        if (heavy) atomicAdd(out + 1, (unsigned long long)heavy);
+    }
 }
 
 // ---- dispatch -------------------------------------------------------------------------------------------------------
@@ -670,6 +697,18 @@ inline void launch_expand(const gcgt_params& P, int grid, cudaStream_t s, const 
 }
 
 template <class App>
+inline void launch_heavy(const gcgt_params& P, int grid, cudaStream_t s, const Ctx& c, const App& app) {
+    const bool seg = P.residual_segment_len != 0;
+    switch (P.zeta_k) {
+        case 1: seg ? heavy_kernel<1, true, App><<<grid, kBlock, 0, s>>>(c, app) : heavy_kernel<1, false, App><<<grid, kBlock, 0, s>>>(c, app); break;
+        case 2: seg ? heavy_kernel<2, true, App><<<grid, kBlock, 0, s>>>(c, app) : heavy_kernel<2, false, App><<<grid, kBlock, 0, s>>>(c, app); break;
+        case 3: seg ? heavy_kernel<3, true, App><<<grid, kBlock, 0, s>>>(c, app) : heavy_kernel<3, false, App><<<grid, kBlock, 0, s>>>(c, app); break;
+        case 4: seg ? heavy_kernel<4, true, App><<<grid, kBlock, 0, s>>>(c, app) : heavy_kernel<4, false, App><<<grid, kBlock, 0, s>>>(c, app); break;
+        default: seg ? heavy_kernel<5, true, App><<<grid, kBlock, 0, s>>>(c, app) : heavy_kernel<5, false, App><<<grid, kBlock, 0, s>>>(c, app); break;
+    }
+}
+
+template <class App>
 inline void launch_hub(const gcgt_params& P, int grid, cudaStream_t s, const Ctx& c, const App& app) {
     if (!P.residual_segment_len) return;
     switch (P.zeta_k) {
@@ -686,7 +725,7 @@ inline void launch_hub(const gcgt_params& P, int grid, cudaStream_t s, const Ctx
 inline void frontier_launch(const gcgt_graph* g, uint64_t qlen, int* grid, uint32_t* wpb) {
     const uint64_t resident_warps = (uint64_t)g->num_sms * 48;
     uint64_t b = qlen / (resident_warps * 4);
-    b = std::max<uint64_t>(1, std::min<uint64_t>(b, 16));
+    b = std::max<uint64_t>(1, std::min<uint64_t>(b, 4));
     const uint64_t warps = (qlen + b - 1) / b;
     *grid = (int)std::max<uint64_t>(1, std::min<uint64_t>((warps + kWarps - 1) / kWarps, (uint64_t)g->num_sms * 32));
     *wpb = (uint32_t)b;
@@ -700,7 +739,8 @@ inline int hub_grid(const gcgt_graph* g) { return g->num_sms * 4; }
 
 inline Ctx make_ctx(const gcgt_graph* g) {
     return Ctx{g->W,     g->offs,     g->P.min_interval_len, 8 * g->P.residual_segment_len,
-               g->hubq, g->hub_ctr, g->stats,              g->cursor};
+               g->hubq, g->hub_ctr, g->stats,              g->cursor,
+               g->heavyq, g->heavy_len};
 }
 
 gcgt_status copy_out(gcgt_graph* g, void* dst, const void* src, size_t bytes, int placement) {
@@ -774,7 +814,8 @@ extern "C" void gcgt_unload(gcgt_graph* g) {
     cudaSetDevice(g->device);
     if (g->stream) cudaStreamSynchronize(g->stream);
     cudaFree(g->W); cudaFree(g->offs); cudaFree(g->V); cudaFree(g->F); cudaFree(g->N); cudaFree(g->q);
-    cudaFree(g->qbits); cudaFree(g->ctr); cudaFree(g->hubq); cudaFree(g->hub_ctr); cudaFree(g->cursor); cudaFree(g->stats); cudaFree(g->levels); cudaFree(g->parent);
+    cudaFree(g->qbits); cudaFree(g->ctr); cudaFree(g->hubq); cudaFree(g->hub_ctr); cudaFree(g->cursor);
+    cudaFree(g->heavyq); cudaFree(g->heavy_len); cudaFree(g->stats); cudaFree(g->levels); cudaFree(g->parent);
     cudaFree(g->sigma); cudaFree(g->delta); cudaFree(g->bc);
     if (g->h_ctr) cudaFreeHost(g->h_ctr);
     if (g->h_stats) cudaFreeHost(g->h_stats);
@@ -833,20 +874,28 @@ extern "C" gcgt_status gcgt_load(const gcgt_cgr* c, const gcgt_load_opts* opts, 
     CU(cudaMemsetAsync(g->N, 0, g->nw * 4, g->stream));
     if ((st = dalloc(&g->hub_ctr, 1)) || (st = dalloc(&g->cursor, 2))) return st;
     CU(cudaMemsetAsync(g->cursor, 0, 16, g->stream));
-    uint64_t nhubs = 0;
-    if (g->P.residual_segment_len) {
-        CU(cudaMemsetAsync(g->hub_ctr, 0, 8, g->stream));
+    unsigned long long* dcount = nullptr;
+    if ((st = dalloc(&dcount, 2))) return st;
+    CU(cudaMemsetAsync(dcount, 0, 16, g->stream));
+    {
         const int gr = flat_grid(g.get(), g->n);
+        const bool seg = g->P.residual_segment_len != 0;
+        cudaStream_t s = g->stream;
         switch (g->P.zeta_k) {
-            case 1: count_hubs<1><<<gr, kBlock, 0, g->stream>>>(g->W, g->offs, g->P.min_interval_len, g->n, g->hub_ctr); break;
-            case 2: count_hubs<2><<<gr, kBlock, 0, g->stream>>>(g->W, g->offs, g->P.min_interval_len, g->n, g->hub_ctr); break;
-            case 3: count_hubs<3><<<gr, kBlock, 0, g->stream>>>(g->W, g->offs, g->P.min_interval_len, g->n, g->hub_ctr); break;
-            case 4: count_hubs<4><<<gr, kBlock, 0, g->stream>>>(g->W, g->offs, g->P.min_interval_len, g->n, g->hub_ctr); break;
-            default: count_hubs<5><<<gr, kBlock, 0, g->stream>>>(g->W, g->offs, g->P.min_interval_len, g->n, g->hub_ctr); break;
+            case 1: seg ? count_special<1, true><<<gr, kBlock, 0, s>>>(g->W, g->offs, g->n, dcount) : count_special<1, false><<<gr, kBlock, 0, s>>>(g->W, g->offs, g->n, dcount); break;
+            case 2: seg ? count_special<2, true><<<gr, kBlock, 0, s>>>(g->W, g->offs, g->n, dcount) : count_special<2, false><<<gr, kBlock, 0, s>>>(g->W, g->offs, g->n, dcount); break;
+            case 3: seg ? count_special<3, true><<<gr, kBlock, 0, s>>>(g->W, g->offs, g->n, dcount) : count_special<3, false><<<gr, kBlock, 0, s>>>(g->W, g->offs, g->n, dcount); break;
+            case 4: seg ? count_special<4, true><<<gr, kBlock, 0, s>>>(g->W, g->offs, g->n, dcount) : count_special<4, false><<<gr, kBlock, 0, s>>>(g->W, g->offs, g->n, dcount); break;
+            default: seg ? count_special<5, true><<<gr, kBlock, 0, s>>>(g->W, g->offs, g->n, dcount) : count_special<5, false><<<gr, kBlock, 0, s>>>(g->W, g->offs, g->n, dcount); break;
         }
-        CU(cudaMemcpyAsync(&nhubs, g->hub_ctr, 8, cudaMemcpyDeviceToHost, g->stream));
     }
+    unsigned long long counts[2] = {0, 0};
+    CU(cudaMemcpyAsync(counts, dcount, 16, cudaMemcpyDeviceToHost, g->stream));
     CU(cudaStreamSynchronize(g->stream));
+    cudaFree(dcount);
+    const uint64_t nhubs = counts[0], nheavy = counts[1];
+    if ((st = dalloc(&g->heavyq, nheavy + 1)) || (st = dalloc(&g->heavy_len, 1))) return st;
+    CU(cudaMemsetAsync(g->heavy_len, 0, 4, g->stream));
     if ((st = dalloc(&g->hubq, nhubs + 1))) return st;
     CU(cudaMemsetAsync(g->hub_ctr, 0, 8, g->stream));
     CU(cudaStreamSynchronize(g->stream));
@@ -942,6 +991,7 @@ extern "C" gcgt_status gcgt_bfs(gcgt_graph* g, uint32_t source, int32_t* levels,
     CU(cudaMemsetAsync(g->levels, 0xff, g->n * 4, s));
     CU(cudaMemsetAsync(g->ctr, 0, 8 * 4, s));
     CU(cudaMemsetAsync(g->hub_ctr, 0, sizeof(unsigned long long), s));
+    CU(cudaMemsetAsync(g->heavy_len, 0, 4, s));
     uint32_t* q[2] = {g->q, g->q + g->nw};
     bfs_seed<<<1, 1, 0, s>>>(source, g->V, g->F, q[0], g->ctr + 0, nullptr);
     const Ctx c = make_ctx(g);
@@ -957,9 +1007,10 @@ extern "C" gcgt_status gcgt_bfs(gcgt_graph* g, uint32_t source, int32_t* levels,
         if ((st = kprof_begin(g))) return st;
         launch_expand(g->P, grid, s, c, fr, app, wpb);
         if ((st = kprof_end(g))) return st;
+        launch_heavy(g->P, hub_grid(g), s, c, app);
         launch_hub(g->P, hub_grid(g), s, c, app);
         commit_dense<<<flat_grid(g, g->nw), kBlock, 0, s>>>(g->V, g->F, g->N, 0, g->nw, q[nxt], g->ctr + nxt, nullptr,
-                                                             g->ctr + cur, g->hub_ctr);
+                                                             g->ctr + cur, g->hub_ctr, g->heavy_len);
         CU(cudaMemcpyAsync(g->h_ctr + nxt, g->ctr + nxt, 4, cudaMemcpyDeviceToHost, s));
         CU(cudaStreamSynchronize(s));
         if ((st = kprof_collect(g))) return st;
@@ -977,6 +1028,7 @@ extern "C" gcgt_status gcgt_cc(gcgt_graph* g, uint32_t* labels, int placement, g
     if ((st = begin_call(g))) return st;
     cudaStream_t s = g->stream;
     CU(cudaMemsetAsync(g->hub_ctr, 0, sizeof(unsigned long long), s));
+    CU(cudaMemsetAsync(g->heavy_len, 0, 4, s));
     cc_init<<<flat_grid(g, g->n), kBlock, 0, s>>>(g->parent, g->n);
     const Ctx c = make_ctx(g);
     const DenseFront fr{g->lo, g->hi};
@@ -987,6 +1039,7 @@ extern "C" gcgt_status gcgt_cc(gcgt_graph* g, uint32_t* labels, int placement, g
     if ((st = kprof_begin(g))) return st;
     launch_expand(g->P, grid, s, c, fr, app, wpb);
     if ((st = kprof_end(g))) return st;
+    launch_heavy(g->P, hub_grid(g), s, c, app);
     launch_hub(g->P, hub_grid(g), s, c, app);
     cc_jump<<<flat_grid(g, g->n), kBlock, 0, s>>>(g->parent, g->n);
     if ((st = copy_out(g, labels, g->parent, g->n * 4, placement))) return st;
@@ -1016,6 +1069,7 @@ extern "C" gcgt_status gcgt_bc(gcgt_graph* g, const uint32_t* sources, uint32_t 
     const Ctx c = make_ctx(g);
     CU(cudaMemsetAsync(g->bc, 0, g->n * 8, s));
     CU(cudaMemsetAsync(g->hub_ctr, 0, sizeof(unsigned long long), s));
+    CU(cudaMemsetAsync(g->heavy_len, 0, 4, s));
     std::vector<uint32_t> lvl_off;
     for (uint32_t si = 0; si < k; si++) {
         const uint32_t src = sources[si];
@@ -1043,10 +1097,12 @@ extern "C" gcgt_status gcgt_bc(gcgt_graph* g, const uint32_t* sources, uint32_t 
             if ((st = kprof_begin(g))) return st;
             launch_expand(g->P, grid, s, c, fr, app, wpb);
             if ((st = kprof_end(g))) return st;
+            launch_heavy(g->P, hub_grid(g), s, c, app);
             launch_hub(g->P, hub_grid(g), s, c, app);
             commit_dense<<<flat_grid(g, g->nw), kBlock, 0, s>>>(g->V, nullptr, g->N, 0, g->nw, g->q + total,
                                                                  g->ctr + 2 + ((level + 1) & 1), g->qbits + total,
-                                                                 g->ctr + 2 + (level & 1), g->hub_ctr);
+                                                                 g->ctr + 2 + (level & 1), g->hub_ctr,
+                                                                 g->heavy_len);
             CU(cudaMemcpyAsync(g->h_ctr + 1, g->ctr + 2 + ((level + 1) & 1), 4, cudaMemcpyDeviceToHost, s));
             CU(cudaStreamSynchronize(s));
             if ((st = kprof_collect(g))) return st;
@@ -1063,8 +1119,10 @@ extern "C" gcgt_status gcgt_bc(gcgt_graph* g, const uint32_t* sources, uint32_t 
             const QueueFront fr{g->q + off, g->ctr + 4, nullptr, g->qbits + off};
             const BcBwdApp app{g->levels, g->sigma, g->delta, g->bc, d + 1, src, 0, 0.0, 0.0};
             launch_expand(g->P, grid, s, c, fr, app, wpb);
+            launch_heavy(g->P, hub_grid(g), s, c, app);
             launch_hub(g->P, hub_grid(g), s, c, app);
             CU(cudaMemsetAsync(g->hub_ctr, 0, sizeof(unsigned long long), s));
+            CU(cudaMemsetAsync(g->heavy_len, 0, 4, s));
         }
     }
     if ((st = copy_out(g, bc, g->bc, g->n * 8, placement))) return st;

@@ -1,0 +1,28 @@
+"""Times gcgt_load / gcgt_bfs (host output) / gcgt_unload separately on a config (diagnostics for bench e2e)."""
+import os
+import sys
+import time
+
+sys.path.insert(0, os.path.dirname(os.path.dirname(os.path.abspath(__file__))))
+import torch  # noqa: E402
+
+import paper_conf_sigmod_shalt19_b200 as G  # noqa: E402
+import synth  # noqa: E402
+
+cfg = synth.CONFIGS[sys.argv[1] if len(sys.argv) > 1 else "c2"]
+ro, co = cfg.make()
+cgr = G.encode(ro, co, cfg.min_interval_len, cfg.residual_segment_len, cfg.zeta_k)
+root = synth.pick_roots(ro, 1)[0]
+levels = torch.empty(ro.size - 1, dtype=torch.int32).pin_memory()
+for i in range(3):
+    torch.cuda.synchronize()
+    t0 = time.perf_counter()
+    g = G.load(cgr, stream="torch")
+    torch.cuda.synchronize()
+    t1 = time.perf_counter()
+    g.bfs(root, out=levels)
+    t2 = time.perf_counter()
+    g.unload()
+    torch.cuda.synchronize()
+    t3 = time.perf_counter()
+    print(f"load {1e3*(t1-t0):.1f} ms  bfs {1e3*(t2-t1):.1f} ms  unload {1e3*(t3-t2):.1f} ms  stats {g.last_stats}")

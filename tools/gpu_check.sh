@@ -3,4 +3,5 @@ TAG=${1:-run}
 mkdir -p gpurun_out
 python -c "import __graft_entry__ as e; e.smoke()" 2>&1 | tail -3
 timeout 1500 python -m pytest tests -m gpu -x -q 2>&1 | tail -15
+timeout 300 python tools/e2e_breakdown.py c2 2>&1 | tail -3
 timeout 900 python bench.py --steps 8 --warmup 3 --no-cpu-baseline > gpurun_out/bench_$TAG.json 2> gpurun_out/bench_$TAG.err; tail -3 gpurun_out/bench_$TAG.err; cat gpurun_out/bench_$TAG.json
