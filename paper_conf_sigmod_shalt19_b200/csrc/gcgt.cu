@@ -160,6 +160,18 @@ struct QueueFront {
     }
 };
 
+// The level's heavy-vertex queue: one vertex per entry.
+struct HeavyFront {
+    const HeavyEntry* __restrict__ q;
+    const uint32_t* __restrict__ len_p;
+    __device__ __forceinline__ uint64_t size() const { return *len_p; }
+    __device__ __forceinline__ void get(uint64_t i, uint32_t& w, uint32_t& bits) const {
+        const uint32_t u = q[i].u;
+        w = u >> 5;
+        bits = 1u << (u & 31);
+    }
+};
+
 // Every vertex of [lo, hi) (CC's hooking pass).
 struct DenseFront {
     uint64_t lo, hi;
@@ -196,9 +208,11 @@ __device__ __forceinline__ uint32_t decode_segment(const uint64_t* __restrict__ 
 // Phase B (segmented format): the batch's segments are flattened with a warp scan and decoded one segment per
 //   lane (segments are self-contained, R17), so lane work is bounded by 2 segBits bits regardless of degree.
 //   Vertices with more than kHubSegs segments go to the hub queue (hub_kernel, whole grid).
-// Heavy vertices (long interval area, or long unsegmented list) go to the level's heavy queue; heavy_kernel then
-//   decodes each with a whole warp via warp_decode (Alg. 4): intervals are paired and their starts recovered
-//   with a warp scan, residual ids likewise.
+// Heavy vertices (long interval area, or long unsegmented list) go to the level's heavy queue, which a second
+//   pass of the same kernel (DEFER = false) drains one lane per heavy vertex over the whole grid, so a long
+//   record never stalls a batch.  (A whole-warp Alg. 4 decode of the long record was measured slower on B200:
+//   each window step is a ~1.5k-cycle dependent chain for ~5 codewords vs ~60 cycles per codeword serially;
+//   DESIGN.md §6.)
 constexpr uint32_t kHeavyItv = 16;   // interval count above which the heavy kernel takes the interval area
 constexpr uint32_t kHeavyRes = 64;   // unsegmented residual count above which the heavy kernel takes the list
 
@@ -208,82 +222,9 @@ struct WarpSmem {
     uint64_t base[32];
 };
 
-struct HeavySmem {
-    uint64_t codes[64];
-};
-
-// Heavy vertex u (warp-uniform arguments), p = first bit after the itvNum field.
-template <int K, bool SEG, class App>
-__device__ __forceinline__ void heavy_vertex(const Ctx& c, const App& app, HeavySmem& sm, uint32_t u, uint64_t p,
-                                             uint64_t itv, uint64_t deg, uint64_t& na) {
-    const uint32_t lane = lane_id();
-    App t = app;
-    t.begin(u);
-    int64_t prev_end = 0;        // warp-uniform
-    uint64_t pairs_done = 0, in_itv = 0;
-    p = warp_decode<K>(c.W, p, 2 * itv, [&](uint64_t base, uint32_t take, uint64_t idx, uint64_t v, bool act) {
-        if (act) sm.codes[idx & 63] = v;
-        __syncwarp();
-        const uint64_t npairs = (base + take) / 2 - pairs_done;
-        if (npairs) {
-            const uint64_t j = pairs_done + lane;
-            const bool has = lane < npairs;
-            uint64_t len = 0;
-            int64_t a = 0;
-            if (has) {
-                const uint64_t g = sm.codes[(2 * j) & 63];
-                len = sm.codes[(2 * j + 1) & 63] - 1 + c.min_len;
-                a = j == 0 ? unmap_first(u, g) + (int64_t)len - 1 : (int64_t)g + (int64_t)len - 1;
-            }
-            int64_t incl = a;
-            for (int o = 1; o < 32; o <<= 1) {
-                const int64_t tt = __shfl_up_sync(0xffffffffu, incl, o);
-                if (lane >= (uint32_t)o) incl += tt;
-            }
-            if (has) {
-                const int64_t end = prev_end + incl;
-                t.range((uint32_t)(end - (int64_t)len + 1), (uint32_t)len);
-                in_itv += len;
-            }
-            prev_end += __shfl_sync(0xffffffffu, incl, (int)npairs - 1);
-            pairs_done += npairs;
-        }
-        __syncwarp();
-    });
-    na += in_itv;
-    if (SEG) {
-        uint64_t q = p;
-        const uint64_t nseg = decode<K>(c.W, q) - 1;  // every lane decodes the same field
-        if (nseg > kHubSegs) {
-            if (lane == 0) {
-                const unsigned long long old = atomicAdd(c.hub_ctr, (1ull << 32) | (unsigned long long)nseg);
-                c.hubq[old >> 32] = HubEntry{q, u, (uint32_t)(old & 0xffffffffu)};
-            }
-        } else if (lane < nseg) {
-            na += decode_segment<K>(c.W, q + (uint64_t)lane * c.seg_bits, u, t);
-        }
-    } else {
-        uint64_t tot_itv = in_itv;
-        for (int o = 16; o; o >>= 1) tot_itv += __shfl_xor_sync(0xffffffffu, tot_itv, o);
-        const uint64_t nres = deg - tot_itv;
-        int64_t cur = 0;  // warp-uniform: last residual id
-        warp_decode<K>(c.W, p, nres, [&](uint64_t base, uint32_t take, uint64_t idx, uint64_t v, bool act) {
-            int64_t a = 0;
-            if (act) a = idx == 0 ? unmap_first(u, v) : (int64_t)v;
-            int64_t incl = a;
-            for (int o = 1; o < 32; o <<= 1) {
-                const int64_t tt = __shfl_up_sync(0xffffffffu, incl, o);
-                if (lane >= (uint32_t)o) incl += tt;
-            }
-            if (act) t.one((uint32_t)(cur + incl));
-            cur += __shfl_sync(0xffffffffu, incl, 31);
-        });
-        if (lane == 0) na += nres;
-    }
-    t.end();
-}
-
-template <int K, bool SEG, class App, class Front>
+// DEFER = true: the level's frontier pass (heavy vertices are queued); false: the heavy pass over that queue
+// (same engine, one lane per heavy vertex, nothing deferred, App::vertex and vertex stats already done).
+template <int K, bool SEG, class App, class Front, bool DEFER>
 __global__ void __launch_bounds__(kBlock, 6) expand_kernel(Ctx c, Front fr, App app, uint32_t wpb) {
     __shared__ WarpSmem smem[kWarps];
     const uint32_t wid = threadIdx.x >> 5, lane = lane_id();
@@ -321,15 +262,17 @@ __global__ void __launch_bounds__(kBlock, 6) expand_kernel(Ctx c, Front fr, App 
                 }
                 u = sm.w[lo] * 32 + __fns(sm.b[lo], 0, (int)(j - sm.pre[lo]) + 1);
                 uint64_t p = ldg64(c.offs + u);
-                nb += ldg64(c.offs + u + 1) - p;
-                nv++;
                 App t = app;
                 t.begin(u);
-                t.vertex(u);
+                if (DEFER) {
+                    nb += ldg64(c.offs + u + 1) - p;
+                    nv++;
+                    t.vertex(u);
+                }
                 uint64_t deg = 0;
                 if (!SEG) deg = decode<K>(c.W, p) - 1;
                 const uint64_t itv = decode<K>(c.W, p) - 1;
-                if (itv > kHeavyItv || (!SEG && deg > kHeavyRes)) {  // heavy: the whole grid takes it later
+                if (DEFER && (itv > kHeavyItv || (!SEG && deg > kHeavyRes))) {  // heavy: deferred to the heavy pass
                     cg::coalesced_group grp = cg::coalesced_threads();
                     uint32_t slot = 0;
                     if (grp.thread_rank() == 0) slot = atomicAdd(c.heavy_len, grp.size());
@@ -411,20 +354,6 @@ __global__ void __launch_bounds__(kBlock, 6) expand_kernel(Ctx c, Front fr, App 
             c.cursor[1] = 0;
         }
     }
-}
-
-// Heavy vertices of the level: one warp per vertex (warp_decode), warps strided over the queue.
-template <int K, bool SEG, class App>
-__global__ void __launch_bounds__(kBlock) heavy_kernel(Ctx c, App app) {
-    __shared__ HeavySmem smem[kWarps];
-    const uint32_t nh = *c.heavy_len;
-    uint64_t na = 0;
-    for (uint64_t h = ((uint64_t)blockIdx.x * blockDim.x + threadIdx.x) >> 5; h < nh;
-         h += ((uint64_t)gridDim.x * blockDim.x) >> 5) {
-        const HeavyEntry e = c.heavyq[h];
-        heavy_vertex<K, SEG>(c, app, smem[threadIdx.x >> 5], e.u, e.p, e.itv, e.deg, na);
-    }
-    add_stats(c.st, 0, na, 0);
 }
 
 // Hub segments of the level, flattened over the whole grid (one segment per thread at a time).
@@ -668,7 +597,7 @@ __global__ void count_special(const uint64_t* __restrict__ W, const uint64_t* __
 
 // ---- dispatch -------------------------------------------------------------------------------------------------------
 // Persistent launch: at most one wave (occupancy calculator), never more blocks than the work needs.
-template <int K, bool SEG, class App, class Front>
+template <int K, bool SEG, class App, class Front, bool DEFER>
 inline void launch_expand_k(int grid, cudaStream_t s, const Ctx& c, const Front& fr, const App& app, uint32_t wpb) {
     static int per_sm = 0;
     static int sms = 0;
@@ -676,36 +605,35 @@ inline void launch_expand_k(int grid, cudaStream_t s, const Ctx& c, const Front&
         int dev = 0;
         cudaGetDevice(&dev);
         cudaDeviceGetAttribute(&sms, cudaDevAttrMultiProcessorCount, dev);
-        cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per_sm, expand_kernel<K, SEG, App, Front>, kBlock, 0);
+        cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per_sm, expand_kernel<K, SEG, App, Front, DEFER>, kBlock, 0);
         if (per_sm < 1) per_sm = 1;
     }
     grid = std::max(1, std::min(grid, per_sm * sms));
-    expand_kernel<K, SEG, App, Front><<<grid, kBlock, 0, s>>>(c, fr, app, wpb);
+    expand_kernel<K, SEG, App, Front, DEFER><<<grid, kBlock, 0, s>>>(c, fr, app, wpb);
 }
 
-template <class App, class Front>
+template <class App, class Front, bool DEFER = true>
 inline void launch_expand(const gcgt_params& P, int grid, cudaStream_t s, const Ctx& c, const Front& fr,
                           const App& app, uint32_t wpb) {
     const bool seg = P.residual_segment_len != 0;
+#define GCGT_EXP(KK)                                                                                  \
+    (seg ? launch_expand_k<KK, true, App, Front, DEFER>(grid, s, c, fr, app, wpb)                      \
+         : launch_expand_k<KK, false, App, Front, DEFER>(grid, s, c, fr, app, wpb))
     switch (P.zeta_k) {
-        case 1: seg ? launch_expand_k<1, true>(grid, s, c, fr, app, wpb) : launch_expand_k<1, false>(grid, s, c, fr, app, wpb); break;
-        case 2: seg ? launch_expand_k<2, true>(grid, s, c, fr, app, wpb) : launch_expand_k<2, false>(grid, s, c, fr, app, wpb); break;
-        case 3: seg ? launch_expand_k<3, true>(grid, s, c, fr, app, wpb) : launch_expand_k<3, false>(grid, s, c, fr, app, wpb); break;
-        case 4: seg ? launch_expand_k<4, true>(grid, s, c, fr, app, wpb) : launch_expand_k<4, false>(grid, s, c, fr, app, wpb); break;
-        default: seg ? launch_expand_k<5, true>(grid, s, c, fr, app, wpb) : launch_expand_k<5, false>(grid, s, c, fr, app, wpb); break;
+        case 1: GCGT_EXP(1); break;
+        case 2: GCGT_EXP(2); break;
+        case 3: GCGT_EXP(3); break;
+        case 4: GCGT_EXP(4); break;
+        default: GCGT_EXP(5); break;
     }
+#undef GCGT_EXP
 }
 
+// Heavy pass: the same engine over the level's heavy queue, 32 heavy vertices per warp batch.
 template <class App>
-inline void launch_heavy(const gcgt_params& P, int grid, cudaStream_t s, const Ctx& c, const App& app) {
-    const bool seg = P.residual_segment_len != 0;
-    switch (P.zeta_k) {
-        case 1: seg ? heavy_kernel<1, true, App><<<grid, kBlock, 0, s>>>(c, app) : heavy_kernel<1, false, App><<<grid, kBlock, 0, s>>>(c, app); break;
-        case 2: seg ? heavy_kernel<2, true, App><<<grid, kBlock, 0, s>>>(c, app) : heavy_kernel<2, false, App><<<grid, kBlock, 0, s>>>(c, app); break;
-        case 3: seg ? heavy_kernel<3, true, App><<<grid, kBlock, 0, s>>>(c, app) : heavy_kernel<3, false, App><<<grid, kBlock, 0, s>>>(c, app); break;
-        case 4: seg ? heavy_kernel<4, true, App><<<grid, kBlock, 0, s>>>(c, app) : heavy_kernel<4, false, App><<<grid, kBlock, 0, s>>>(c, app); break;
-        default: seg ? heavy_kernel<5, true, App><<<grid, kBlock, 0, s>>>(c, app) : heavy_kernel<5, false, App><<<grid, kBlock, 0, s>>>(c, app); break;
-    }
+inline void launch_heavy(const gcgt_graph* g, cudaStream_t s, const Ctx& c, const App& app) {
+    const HeavyFront fr{c.heavyq, c.heavy_len};
+    launch_expand<App, HeavyFront, false>(g->P, g->num_sms * 8, s, c, fr, app, 32);
 }
 
 template <class App>
@@ -1007,7 +935,7 @@ extern "C" gcgt_status gcgt_bfs(gcgt_graph* g, uint32_t source, int32_t* levels,
         if ((st = kprof_begin(g))) return st;
         launch_expand(g->P, grid, s, c, fr, app, wpb);
         if ((st = kprof_end(g))) return st;
-        launch_heavy(g->P, hub_grid(g), s, c, app);
+        launch_heavy(g, s, c, app);
         launch_hub(g->P, hub_grid(g), s, c, app);
         commit_dense<<<flat_grid(g, g->nw), kBlock, 0, s>>>(g->V, g->F, g->N, 0, g->nw, q[nxt], g->ctr + nxt, nullptr,
                                                              g->ctr + cur, g->hub_ctr, g->heavy_len);
@@ -1039,7 +967,7 @@ extern "C" gcgt_status gcgt_cc(gcgt_graph* g, uint32_t* labels, int placement, g
     if ((st = kprof_begin(g))) return st;
     launch_expand(g->P, grid, s, c, fr, app, wpb);
     if ((st = kprof_end(g))) return st;
-    launch_heavy(g->P, hub_grid(g), s, c, app);
+    launch_heavy(g, s, c, app);
     launch_hub(g->P, hub_grid(g), s, c, app);
     cc_jump<<<flat_grid(g, g->n), kBlock, 0, s>>>(g->parent, g->n);
     if ((st = copy_out(g, labels, g->parent, g->n * 4, placement))) return st;
@@ -1097,7 +1025,7 @@ extern "C" gcgt_status gcgt_bc(gcgt_graph* g, const uint32_t* sources, uint32_t 
             if ((st = kprof_begin(g))) return st;
             launch_expand(g->P, grid, s, c, fr, app, wpb);
             if ((st = kprof_end(g))) return st;
-            launch_heavy(g->P, hub_grid(g), s, c, app);
+            launch_heavy(g, s, c, app);
             launch_hub(g->P, hub_grid(g), s, c, app);
             commit_dense<<<flat_grid(g, g->nw), kBlock, 0, s>>>(g->V, nullptr, g->N, 0, g->nw, g->q + total,
                                                                  g->ctr + 2 + ((level + 1) & 1), g->qbits + total,
@@ -1119,7 +1047,7 @@ extern "C" gcgt_status gcgt_bc(gcgt_graph* g, const uint32_t* sources, uint32_t 
             const QueueFront fr{g->q + off, g->ctr + 4, nullptr, g->qbits + off};
             const BcBwdApp app{g->levels, g->sigma, g->delta, g->bc, d + 1, src, 0, 0.0, 0.0};
             launch_expand(g->P, grid, s, c, fr, app, wpb);
-            launch_heavy(g->P, hub_grid(g), s, c, app);
+            launch_heavy(g, s, c, app);
             launch_hub(g->P, hub_grid(g), s, c, app);
             CU(cudaMemsetAsync(g->hub_ctr, 0, sizeof(unsigned long long), s));
             CU(cudaMemsetAsync(g->heavy_len, 0, 4, s));
