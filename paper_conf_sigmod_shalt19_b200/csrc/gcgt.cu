@@ -112,7 +112,7 @@ constexpr int kWarps = kBlock / 32;
 // A vertex with more residual segments than this is not expanded by its own warp: its segments go to the
 // level's hub queue and are spread over the whole grid (segment-level work stealing, the B200 analogue of the
 // paper's Task Stealing + Residual Segmentation, §4.3 :884-930, §5.2 :1092-1136).
-constexpr uint32_t kHubSegs = 32;
+constexpr uint32_t kHubSegs = 8;
 
 __device__ __forceinline__ uint32_t lane_id() { return threadIdx.x & 31; }
 __device__ __forceinline__ uint32_t lanemask_lt() { uint32_t m; asm("mov.u32 %0, %%lanemask_lt;" : "=r"(m)); return m; }
@@ -231,11 +231,12 @@ __global__ void __launch_bounds__(kBlock, 6) expand_kernel(Ctx c, Front fr, App 
     WarpSmem& sm = smem[wid];
     const uint64_t qlen = fr.size();
     uint64_t nv = 0, na = 0, nb = 0;
+    unsigned long long next = 0;  // the next batch's cursor value is fetched one batch ahead (latency hidden)
+    if (lane == 0) next = atomicAdd(c.cursor, (unsigned long long)wpb);
     for (;;) {
-        uint64_t base = 0;
-        if (lane == 0) base = atomicAdd(c.cursor, (unsigned long long)wpb);
-        base = __shfl_sync(0xffffffffu, base, 0);
+        const uint64_t base = __shfl_sync(0xffffffffu, next, 0);
         if (base >= qlen) break;
+        if (lane == 0) next = atomicAdd(c.cursor, (unsigned long long)wpb);
         uint32_t w = 0, bits = 0;
         if (lane < wpb && base + lane < qlen) fr.get(base + lane, w, bits);
         uint32_t incl = __popc(bits);
@@ -302,7 +303,7 @@ __global__ void __launch_bounds__(kBlock, 6) expand_kernel(Ctx c, Front fr, App 
                     } else {
                         nseg = (uint32_t)(decode<K>(c.W, p) - 1);
                         segbase = p;
-                        if (nseg > kHubSegs) {  // hub: hand the segments to the whole grid
+                        if (nseg > kHubSegs || (!DEFER && nseg)) {  // hub: hand the segments to the whole grid
                             const unsigned long long old =
                                 atomicAdd(c.hub_ctr, (1ull << 32) | (unsigned long long)nseg);
                             c.hubq[old >> 32] = HubEntry{segbase, u, (uint32_t)(old & 0xffffffffu)};
@@ -653,7 +654,7 @@ inline void launch_hub(const gcgt_params& P, int grid, cudaStream_t s, const Ctx
 inline void frontier_launch(const gcgt_graph* g, uint64_t qlen, int* grid, uint32_t* wpb) {
     const uint64_t resident_warps = (uint64_t)g->num_sms * 48;
     uint64_t b = qlen / (resident_warps * 4);
-    b = std::max<uint64_t>(1, std::min<uint64_t>(b, 4));
+    b = std::max<uint64_t>(1, std::min<uint64_t>(b, 8));
     const uint64_t warps = (qlen + b - 1) / b;
     *grid = (int)std::max<uint64_t>(1, std::min<uint64_t>((warps + kWarps - 1) / kWarps, (uint64_t)g->num_sms * 32));
     *wpb = (uint32_t)b;
@@ -732,6 +733,16 @@ gcgt_status dalloc(T** p, uint64_t count) {
     return GCGT_OK;
 }
 
+// Graph buffers come from the device's stream-ordered memory pool, which keeps freed memory (release threshold =
+// max), so repeated load / unload cycles (the bench's end-to-end leg, query services) reuse device memory instead
+// of paying cudaMalloc / cudaFree each time.
+template <class T>
+gcgt_status galloc(const gcgt_graph* g, T** p, uint64_t count) {
+    cudaError_t e = cudaMallocAsync((void**)p, std::max<uint64_t>(1, count) * sizeof(T), g->stream);
+    if (e != cudaSuccess) return fail(GCGT_ENOMEM, std::string("cudaMallocAsync: ") + cudaGetErrorString(e));
+    return GCGT_OK;
+}
+
 }  // namespace
 
 // ------------------------------------------------------------------------------------------------------------------
@@ -740,11 +751,14 @@ gcgt_status dalloc(T** p, uint64_t count) {
 extern "C" void gcgt_unload(gcgt_graph* g) {
     if (!g) return;
     cudaSetDevice(g->device);
-    if (g->stream) cudaStreamSynchronize(g->stream);
-    cudaFree(g->W); cudaFree(g->offs); cudaFree(g->V); cudaFree(g->F); cudaFree(g->N); cudaFree(g->q);
-    cudaFree(g->qbits); cudaFree(g->ctr); cudaFree(g->hubq); cudaFree(g->hub_ctr); cudaFree(g->cursor);
-    cudaFree(g->heavyq); cudaFree(g->heavy_len); cudaFree(g->stats); cudaFree(g->levels); cudaFree(g->parent);
-    cudaFree(g->sigma); cudaFree(g->delta); cudaFree(g->bc);
+    void* bufs[] = {g->W,      g->offs,    g->V,      g->F,         g->N,        g->q,      g->qbits,
+                    g->ctr,    g->hubq,    g->hub_ctr, g->cursor,   g->heavyq,   g->heavy_len, g->stats,
+                    g->levels, g->parent,  g->sigma,  g->delta,     g->bc};
+    if (g->stream) {
+        for (void* b : bufs)
+            if (b) cudaFreeAsync(b, g->stream);
+        cudaStreamSynchronize(g->stream);
+    }
     if (g->h_ctr) cudaFreeHost(g->h_ctr);
     if (g->h_stats) cudaFreeHost(g->h_stats);
     if (g->ev0) cudaEventDestroy(g->ev0);
@@ -767,9 +781,14 @@ extern "C" gcgt_status gcgt_load(const gcgt_cgr* c, const gcgt_load_opts* opts, 
     std::unique_ptr<gcgt_graph, void (*)(gcgt_graph*)> g(new gcgt_graph(), gcgt_unload);
     g->device = o.device;
     CU(cudaSetDevice(o.device));
-    cudaDeviceProp prop;
-    CU(cudaGetDeviceProperties(&prop, o.device));
-    g->num_sms = prop.multiProcessorCount;
+    {   // keep freed pool memory for the next load (see galloc)
+        cudaMemPool_t pool;
+        if (cudaDeviceGetDefaultMemPool(&pool, o.device) == cudaSuccess) {
+            uint64_t thr = UINT64_MAX;
+            cudaMemPoolSetAttribute(pool, cudaMemPoolAttrReleaseThreshold, &thr);
+        }
+    }
+    CU(cudaDeviceGetAttribute(&g->num_sms, cudaDevAttrMultiProcessorCount, o.device));
     if (o.stream) g->stream = (cudaStream_t)o.stream;
     else {
         CU(cudaStreamCreateWithFlags(&g->stream, cudaStreamNonBlocking));
@@ -783,12 +802,12 @@ extern "C" gcgt_status gcgt_load(const gcgt_cgr* c, const gcgt_load_opts* opts, 
     g->nw = (c->n + 31) / 32 + 1;
     const uint64_t nwords = (c->nbits + 63) / 64 + 2;
     gcgt_status st;
-    if ((st = dalloc(&g->W, nwords)) || (st = dalloc(&g->offs, g->n + 1)) || (st = dalloc(&g->V, g->nw)) ||
-        (st = dalloc(&g->F, g->nw)) || (st = dalloc(&g->N, g->nw)) || (st = dalloc(&g->ctr, 8)) ||
-        (st = dalloc(&g->stats, 1)) || (st = dalloc(&g->levels, g->n)))
+    if ((st = galloc(g.get(), &g->W, nwords)) || (st = galloc(g.get(), &g->offs, g->n + 1)) || (st = galloc(g.get(), &g->V, g->nw)) ||
+        (st = galloc(g.get(), &g->F, g->nw)) || (st = galloc(g.get(), &g->N, g->nw)) || (st = galloc(g.get(), &g->ctr, 8)) ||
+        (st = galloc(g.get(), &g->stats, 1)) || (st = galloc(g.get(), &g->levels, g->n)))
         return st;
     g->qcap = 2 * g->nw;
-    if ((st = dalloc(&g->q, g->qcap))) return st;
+    if ((st = galloc(g.get(), &g->q, g->qcap))) return st;
     CU(cudaMallocHost((void**)&g->h_ctr, 8 * sizeof(uint32_t)));
     CU(cudaMallocHost((void**)&g->h_stats, sizeof(Stats)));
     CU(cudaEventCreate(&g->ev0));
@@ -800,10 +819,10 @@ extern "C" gcgt_status gcgt_load(const gcgt_cgr* c, const gcgt_load_opts* opts, 
                        g->stream));
     bswap_words<<<flat_grid(g.get(), nwords), kBlock, 0, g->stream>>>(g->W, nwords);
     CU(cudaMemsetAsync(g->N, 0, g->nw * 4, g->stream));
-    if ((st = dalloc(&g->hub_ctr, 1)) || (st = dalloc(&g->cursor, 2))) return st;
+    if ((st = galloc(g.get(), &g->hub_ctr, 1)) || (st = galloc(g.get(), &g->cursor, 2))) return st;
     CU(cudaMemsetAsync(g->cursor, 0, 16, g->stream));
     unsigned long long* dcount = nullptr;
-    if ((st = dalloc(&dcount, 2))) return st;
+    if ((st = galloc(g.get(), &dcount, 2))) return st;
     CU(cudaMemsetAsync(dcount, 0, 16, g->stream));
     {
         const int gr = flat_grid(g.get(), g->n);
@@ -820,11 +839,11 @@ extern "C" gcgt_status gcgt_load(const gcgt_cgr* c, const gcgt_load_opts* opts, 
     unsigned long long counts[2] = {0, 0};
     CU(cudaMemcpyAsync(counts, dcount, 16, cudaMemcpyDeviceToHost, g->stream));
     CU(cudaStreamSynchronize(g->stream));
-    cudaFree(dcount);
+    cudaFreeAsync(dcount, g->stream);
     const uint64_t nhubs = counts[0], nheavy = counts[1];
-    if ((st = dalloc(&g->heavyq, nheavy + 1)) || (st = dalloc(&g->heavy_len, 1))) return st;
+    if ((st = galloc(g.get(), &g->heavyq, nheavy + 1)) || (st = galloc(g.get(), &g->heavy_len, 1))) return st;
     CU(cudaMemsetAsync(g->heavy_len, 0, 4, g->stream));
-    if ((st = dalloc(&g->hubq, nhubs + 1))) return st;
+    if ((st = galloc(g.get(), &g->hubq, nhubs + nheavy + 1))) return st;
     CU(cudaMemsetAsync(g->hub_ctr, 0, 8, g->stream));
     CU(cudaStreamSynchronize(g->stream));
     CU(cudaGetLastError());
@@ -952,7 +971,7 @@ extern "C" gcgt_status gcgt_bfs(gcgt_graph* g, uint32_t source, int32_t* levels,
 extern "C" gcgt_status gcgt_cc(gcgt_graph* g, uint32_t* labels, int placement, gcgt_stats* stats) {
     if (!g || !labels) return fail(GCGT_EINVAL, "null argument");
     gcgt_status st;
-    if (!g->parent && (st = dalloc(&g->parent, g->n))) return st;
+    if (!g->parent && (st = galloc(g, &g->parent, g->n))) return st;
     if ((st = begin_call(g))) return st;
     cudaStream_t s = g->stream;
     CU(cudaMemsetAsync(g->hub_ctr, 0, sizeof(unsigned long long), s));
@@ -983,12 +1002,12 @@ extern "C" gcgt_status gcgt_bc(gcgt_graph* g, const uint32_t* sources, uint32_t 
         if (sources[i] >= g->n) return fail(GCGT_ERANGE, "source >= n");
     gcgt_status st;
     if (!g->sigma) {
-        if ((st = dalloc(&g->sigma, g->n)) || (st = dalloc(&g->delta, g->n)) || (st = dalloc(&g->bc, g->n)) ||
-            (st = dalloc(&g->qbits, g->n + g->nw)))
+        if ((st = galloc(g, &g->sigma, g->n)) || (st = galloc(g, &g->delta, g->n)) || (st = galloc(g, &g->bc, g->n)) ||
+            (st = galloc(g, &g->qbits, g->n + g->nw)))
             return st;
         uint32_t* bigq = nullptr;
-        if ((st = dalloc(&bigq, g->n + g->nw))) return st;
-        cudaFree(g->q);
+        if ((st = galloc(g, &bigq, g->n + g->nw))) return st;
+        cudaFreeAsync(g->q, g->stream);
         g->q = bigq;
         g->qcap = g->n + g->nw;
     }
