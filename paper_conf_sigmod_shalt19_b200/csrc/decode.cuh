@@ -204,3 +204,66 @@ __device__ __forceinline__ uint64_t warp_decode(const uint64_t* __restrict__ W, 
 }
 
 }  // namespace gcgt_dev
+
+namespace gcgt_dev {
+
+// Register-staged bit reader: a 256-bit window (four 64-bit stream words) held in registers and refilled with
+// four independent loads when a codeword may cross its end.  Decoding is then pure ALU work (CLZ + shifts):
+// one memory round trip per ~256 bits instead of one (L1) round trip per codeword.  Codewords longer than the
+// 64-bit path use the global-memory slow path.
+struct RegStream {
+    const uint64_t* __restrict__ W;
+    uint64_t p;      // absolute bit position of the next codeword
+    uint64_t base;   // word index of r0
+    uint64_t r0, r1, r2, r3;
+
+    __device__ __forceinline__ void fill(uint64_t wi) {
+        base = wi;
+        r0 = ldg64(W + wi);
+        r1 = ldg64(W + wi + 1);
+        r2 = ldg64(W + wi + 2);
+        r3 = ldg64(W + wi + 3);
+    }
+    __device__ __forceinline__ void init(const uint64_t* __restrict__ w, uint64_t pos) {
+        W = w;
+        p = pos;
+        fill(pos >> 6);
+    }
+    __device__ __forceinline__ void seek(uint64_t pos) {
+        p = pos;
+        const uint64_t wi = pos >> 6;
+        if (wi < base || wi + 1 > base + 3) fill(wi);
+    }
+    __device__ __forceinline__ uint64_t win() {
+        uint64_t wi = p >> 6;
+        if (wi + 1 > base + 3) {  // the 64-bit window would leave the staged words
+            fill(wi);
+        }
+        const uint32_t k = (uint32_t)(wi - base), s = (uint32_t)(p & 63);
+        const uint64_t a = k == 0 ? r0 : k == 1 ? r1 : r2;
+        const uint64_t b = k == 0 ? r1 : k == 1 ? r2 : r3;
+        return s ? (a << s) | (b >> (64 - s)) : a;
+    }
+    template <int K>
+    __device__ __forceinline__ uint64_t next() {
+        const uint64_t w = win();
+        const uint32_t z = (uint32_t)__clzll((long long)w);
+        if (K == 1) {
+            if (z < 32) {
+                const uint32_t L = 2 * z + 1;
+                p += L;
+                return w >> (64 - L);
+            }
+        } else {
+            const uint32_t h = z + 1, L = h * (K + 1);
+            if (L <= 64) {
+                p += L;
+                return (w << h) >> (64 - K * h);
+            }
+        }
+        const uint64_t v = decode_slow<K>(W, p);
+        return v;
+    }
+};
+
+}  // namespace gcgt_dev

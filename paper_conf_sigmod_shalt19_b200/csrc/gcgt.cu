@@ -187,14 +187,26 @@ struct DenseFront {
 
 // ---- decode helpers ---------------------------------------------------------------------------------------------------
 // One residual segment (FORMAT.md R17): count, first residual anchored at u, then gaps.  Returns the count.
+// The segment's bits are staged in registers (RegStream) and the neighbour ids are handed to the filter four at a
+// time (App::many), so their visited-bitmap probes are in flight together.
 template <int K, class T>
 __device__ __forceinline__ uint32_t decode_segment(const uint64_t* __restrict__ W, uint64_t q, uint32_t u, T& t) {
-    const uint32_t cnt = (uint32_t)(decode<K>(W, q) - 1);
-    int64_t cur = unmap_first(u, decode<K>(W, q));
-    t.one((uint32_t)cur);
-    for (uint32_t i = 1; i < cnt; i++) {
-        cur += (int64_t)decode<K>(W, q);
-        t.one((uint32_t)cur);
+    RegStream rs;
+    rs.init(W, q);
+    const uint32_t cnt = (uint32_t)(rs.next<K>() - 1);
+    int64_t cur = 0;
+    for (uint32_t done = 0; done < cnt; done += 4) {
+        uint32_t v[4];
+        const uint32_t nb = min(4u, cnt - done);
+#pragma unroll
+        for (uint32_t k = 0; k < 4; k++) {
+            if (k < nb) {
+                const uint64_t c = rs.next<K>();
+                cur = (done + k == 0) ? unmap_first(u, c) : cur + (int64_t)c;
+                v[k] = (uint32_t)cur;
+            }
+        }
+        t.many(v, nb);
     }
     return cnt;
 }
@@ -225,7 +237,7 @@ struct WarpSmem {
 // DEFER = true: the level's frontier pass (heavy vertices are queued); false: the heavy pass over that queue
 // (same engine, one lane per heavy vertex, nothing deferred, App::vertex and vertex stats already done).
 template <int K, bool SEG, class App, class Front, bool DEFER>
-__global__ void __launch_bounds__(kBlock, 6) expand_kernel(Ctx c, Front fr, App app, uint32_t wpb) {
+__global__ void __launch_bounds__(kBlock, 4) expand_kernel(Ctx c, Front fr, App app, uint32_t wpb) {
     __shared__ WarpSmem smem[kWarps];
     const uint32_t wid = threadIdx.x >> 5, lane = lane_id();
     WarpSmem& sm = smem[wid];
@@ -270,9 +282,12 @@ __global__ void __launch_bounds__(kBlock, 6) expand_kernel(Ctx c, Front fr, App 
                     nv++;
                     t.vertex(u);
                 }
+                RegStream rs;
+                rs.init(c.W, p);
                 uint64_t deg = 0;
-                if (!SEG) deg = decode<K>(c.W, p) - 1;
-                const uint64_t itv = decode<K>(c.W, p) - 1;
+                if (!SEG) deg = rs.next<K>() - 1;
+                const uint64_t itv = rs.next<K>() - 1;
+                p = rs.p;
                 if (DEFER && (itv > kHeavyItv || (!SEG && deg > kHeavyRes))) {  // heavy: deferred to the heavy pass
                     cg::coalesced_group grp = cg::coalesced_threads();
                     uint32_t slot = 0;
@@ -283,8 +298,8 @@ __global__ void __launch_bounds__(kBlock, 6) expand_kernel(Ctx c, Front fr, App 
                     int64_t prev_end = 0;
                     uint64_t in_itv = 0;
                     for (uint64_t i = 0; i < itv; i++) {
-                        const uint64_t g = decode<K>(c.W, p);
-                        const uint64_t len = decode<K>(c.W, p) - 1 + c.min_len;
+                        const uint64_t g = rs.next<K>();
+                        const uint64_t len = rs.next<K>() - 1 + c.min_len;
                         const int64_t start = i == 0 ? unmap_first(u, g) : prev_end + (int64_t)g;
                         t.range((uint32_t)start, (uint32_t)len);
                         prev_end = start + (int64_t)len - 1;
@@ -295,14 +310,14 @@ __global__ void __launch_bounds__(kBlock, 6) expand_kernel(Ctx c, Front fr, App 
                         const uint64_t nres = deg - in_itv;
                         int64_t cur = 0;
                         for (uint64_t i = 0; i < nres; i++) {
-                            const uint64_t cd = decode<K>(c.W, p);
+                            const uint64_t cd = rs.next<K>();
                             cur = i == 0 ? unmap_first(u, cd) : cur + (int64_t)cd;
                             t.one((uint32_t)cur);
                         }
                         na += nres;
                     } else {
-                        nseg = (uint32_t)(decode<K>(c.W, p) - 1);
-                        segbase = p;
+                        nseg = (uint32_t)(rs.next<K>() - 1);
+                        segbase = rs.p;
                         if (nseg > kHubSegs || (!DEFER && nseg)) {  // hub: hand the segments to the whole grid
                             const unsigned long long old =
                                 atomicAdd(c.hub_ctr, (1ull << 32) | (unsigned long long)nseg);
@@ -395,6 +410,17 @@ struct BfsApp {
         if (cand) atomicOr(N + w, cand);
     }
     __device__ __forceinline__ void one(uint32_t v) { claim(v >> 5, 1u << (v & 31)); }
+    // up to four ids: the four visited-bitmap probes are issued before any is consumed
+    __device__ __forceinline__ void many(const uint32_t (&v)[4], uint32_t n) {
+        uint32_t m[4];
+#pragma unroll
+        for (uint32_t k = 0; k < 4; k++) m[k] = k < n ? __ldg(V + (v[k] >> 5)) : 0xffffffffu;
+#pragma unroll
+        for (uint32_t k = 0; k < 4; k++) {
+            const uint32_t bit = 1u << (v[k] & 31);
+            if (k < n && !(m[k] & bit)) atomicOr(N + (v[k] >> 5), bit);
+        }
+    }
     __device__ __forceinline__ void range(uint32_t s, uint32_t len) {
         const uint32_t e = s + len;
         while (s < e) {
@@ -404,6 +430,12 @@ struct BfsApp {
         }
     }
 };
+
+// generic many() for filters without a batched form
+#define GCGT_MANY_BY_ONE                                                         \
+    __device__ __forceinline__ void many(const uint32_t (&v)[4], uint32_t n) {  \
+        for (uint32_t k = 0; k < n; k++) one(v[k]);                              \
+    }
 
 // BC forward (Fig. 7(d), Brandes [9]): an arc u->v with v not in V (levels <= d) has level(v) = d+1, so
 // sigma(v) += sigma(u); N collects level d+1.
@@ -429,6 +461,7 @@ struct BcFwdApp {
         }
     }
     __device__ __forceinline__ void one(uint32_t v) { claim(v >> 5, 1u << (v & 31)); }
+    GCGT_MANY_BY_ONE
     __device__ __forceinline__ void range(uint32_t s, uint32_t len) {
         const uint32_t e = s + len;
         while (s < e) {
@@ -456,6 +489,7 @@ struct BcBwdApp {
     __device__ __forceinline__ void one(uint32_t w) {
         if (levels[w] == next) acc += sv / sigma[w] * (1.0 + delta[w]);
     }
+    GCGT_MANY_BY_ONE
     __device__ __forceinline__ void range(uint32_t s, uint32_t len) {
         for (uint32_t t = 0; t < len; t++) one(s + t);
     }
@@ -499,6 +533,7 @@ struct CcApp {
             rv = cc_find(parent, rv);
         }
     }
+    GCGT_MANY_BY_ONE
     __device__ __forceinline__ void range(uint32_t s, uint32_t len) {
         for (uint32_t t = 0; t < len; t++) one(s + t);
     }
