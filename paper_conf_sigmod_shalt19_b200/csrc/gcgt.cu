@@ -19,6 +19,7 @@
 #include <algorithm>
 #include <memory>
 #include <string>
+#include <type_traits>
 #include <vector>
 
 #include "decode.cuh"
@@ -88,6 +89,9 @@ struct gcgt_graph {
     HubEntry* hubq = nullptr;   // per-level hub queue (capacity = hub vertices + 1)
     unsigned long long* cursor = nullptr;  // [0] work cursor, [1] finished-warp count (expand_kernel)
     HeavyEntry* heavyq = nullptr;          // per-level heavy-vertex queue (capacity = heavy vertices + 1)
+    // tuning knobs (defaults; GCGT_TUNE="staged=0,heavy_itv=16,hub_segs=8,wpb_max=8" overrides at load)
+    bool staged = true;
+    uint32_t heavy_itv = 16, heavy_res = 64, hub_segs = 8, wpb_max = 8;
     uint32_t* heavy_len = nullptr;
     unsigned long long* hub_ctr = nullptr;
     Stats* stats = nullptr;
@@ -112,7 +116,6 @@ constexpr int kWarps = kBlock / 32;
 // A vertex with more residual segments than this is not expanded by its own warp: its segments go to the
 // level's hub queue and are spread over the whole grid (segment-level work stealing, the B200 analogue of the
 // paper's Task Stealing + Residual Segmentation, §4.3 :884-930, §5.2 :1092-1136).
-constexpr uint32_t kHubSegs = 8;
 
 __device__ __forceinline__ uint32_t lane_id() { return threadIdx.x & 31; }
 __device__ __forceinline__ uint32_t lanemask_lt() { uint32_t m; asm("mov.u32 %0, %%lanemask_lt;" : "=r"(m)); return m; }
@@ -129,6 +132,9 @@ struct Ctx {
     unsigned long long* cursor;   // work cursor over the frontier queue (reset per launch)
     HeavyEntry* heavyq;           // per-level heavy-vertex queue
     uint32_t* heavy_len;
+    uint32_t heavy_itv;           // interval count above which a vertex is deferred to the heavy pass
+    uint32_t heavy_res;           // unsegmented residual count above which a vertex is deferred
+    uint32_t hub_segs;            // segment count above which a vertex's segments go to the hub queue
 };
 
 __device__ __forceinline__ void add_stats(Stats* st, uint64_t v, uint64_t a, uint64_t b) {
@@ -189,11 +195,23 @@ struct DenseFront {
 // One residual segment (FORMAT.md R17): count, first residual anchored at u, then gaps.  Returns the count.
 // The segment's bits are staged in registers (RegStream) and the neighbour ids are handed to the filter four at a
 // time (App::many), so their visited-bitmap probes are in flight together.
-template <int K, class T>
+// Per-codeword global-window reader (the unstaged alternative to RegStream; same interface).
+struct WinStream {
+    const uint64_t* __restrict__ W;
+    uint64_t p;
+    __device__ __forceinline__ void init(const uint64_t* __restrict__ w, uint64_t pos) { W = w; p = pos; }
+    template <int K>
+    __device__ __forceinline__ uint64_t next() { return decode<K>(W, p); }
+};
+
+template <bool STAGED>
+using Reader = typename std::conditional<STAGED, RegStream, WinStream>::type;
+
+template <int K, bool STAGED, class T>
 __device__ __forceinline__ uint32_t decode_segment(const uint64_t* __restrict__ W, uint64_t q, uint32_t u, T& t) {
-    RegStream rs;
+    Reader<STAGED> rs;
     rs.init(W, q);
-    const uint32_t cnt = (uint32_t)(rs.next<K>() - 1);
+    const uint32_t cnt = (uint32_t)(rs.template next<K>() - 1);
     int64_t cur = 0;
     for (uint32_t done = 0; done < cnt; done += 4) {
         uint32_t v[4];
@@ -201,7 +219,7 @@ __device__ __forceinline__ uint32_t decode_segment(const uint64_t* __restrict__ 
 #pragma unroll
         for (uint32_t k = 0; k < 4; k++) {
             if (k < nb) {
-                const uint64_t c = rs.next<K>();
+                const uint64_t c = rs.template next<K>();
                 cur = (done + k == 0) ? unmap_first(u, c) : cur + (int64_t)c;
                 v[k] = (uint32_t)cur;
             }
@@ -225,8 +243,6 @@ __device__ __forceinline__ uint32_t decode_segment(const uint64_t* __restrict__ 
 //   record never stalls a batch.  (A whole-warp Alg. 4 decode of the long record was measured slower on B200:
 //   each window step is a ~1.5k-cycle dependent chain for ~5 codewords vs ~60 cycles per codeword serially;
 //   DESIGN.md §6.)
-constexpr uint32_t kHeavyItv = 16;   // interval count above which the heavy kernel takes the interval area
-constexpr uint32_t kHeavyRes = 64;   // unsegmented residual count above which the heavy kernel takes the list
 
 struct WarpSmem {
     uint32_t w[32], b[32], pre[33];
@@ -236,7 +252,7 @@ struct WarpSmem {
 
 // DEFER = true: the level's frontier pass (heavy vertices are queued); false: the heavy pass over that queue
 // (same engine, one lane per heavy vertex, nothing deferred, App::vertex and vertex stats already done).
-template <int K, bool SEG, class App, class Front, bool DEFER>
+template <int K, bool SEG, class App, class Front, bool DEFER, bool STAGED>
 __global__ void __launch_bounds__(kBlock, 4) expand_kernel(Ctx c, Front fr, App app, uint32_t wpb) {
     __shared__ WarpSmem smem[kWarps];
     const uint32_t wid = threadIdx.x >> 5, lane = lane_id();
@@ -282,13 +298,13 @@ __global__ void __launch_bounds__(kBlock, 4) expand_kernel(Ctx c, Front fr, App 
                     nv++;
                     t.vertex(u);
                 }
-                RegStream rs;
+                Reader<STAGED> rs;
                 rs.init(c.W, p);
                 uint64_t deg = 0;
-                if (!SEG) deg = rs.next<K>() - 1;
-                const uint64_t itv = rs.next<K>() - 1;
+                if (!SEG) deg = rs.template next<K>() - 1;
+                const uint64_t itv = rs.template next<K>() - 1;
                 p = rs.p;
-                if (DEFER && (itv > kHeavyItv || (!SEG && deg > kHeavyRes))) {  // heavy: deferred to the heavy pass
+                if (DEFER && (itv > c.heavy_itv || (!SEG && deg > c.heavy_res))) {  // heavy: deferred to the heavy pass
                     cg::coalesced_group grp = cg::coalesced_threads();
                     uint32_t slot = 0;
                     if (grp.thread_rank() == 0) slot = atomicAdd(c.heavy_len, grp.size());
@@ -298,8 +314,8 @@ __global__ void __launch_bounds__(kBlock, 4) expand_kernel(Ctx c, Front fr, App 
                     int64_t prev_end = 0;
                     uint64_t in_itv = 0;
                     for (uint64_t i = 0; i < itv; i++) {
-                        const uint64_t g = rs.next<K>();
-                        const uint64_t len = rs.next<K>() - 1 + c.min_len;
+                        const uint64_t g = rs.template next<K>();
+                        const uint64_t len = rs.template next<K>() - 1 + c.min_len;
                         const int64_t start = i == 0 ? unmap_first(u, g) : prev_end + (int64_t)g;
                         t.range((uint32_t)start, (uint32_t)len);
                         prev_end = start + (int64_t)len - 1;
@@ -310,15 +326,15 @@ __global__ void __launch_bounds__(kBlock, 4) expand_kernel(Ctx c, Front fr, App 
                         const uint64_t nres = deg - in_itv;
                         int64_t cur = 0;
                         for (uint64_t i = 0; i < nres; i++) {
-                            const uint64_t cd = rs.next<K>();
+                            const uint64_t cd = rs.template next<K>();
                             cur = i == 0 ? unmap_first(u, cd) : cur + (int64_t)cd;
                             t.one((uint32_t)cur);
                         }
                         na += nres;
                     } else {
-                        nseg = (uint32_t)(rs.next<K>() - 1);
+                        nseg = (uint32_t)(rs.template next<K>() - 1);
                         segbase = rs.p;
-                        if (nseg > kHubSegs || (!DEFER && nseg)) {  // hub: hand the segments to the whole grid
+                        if (nseg > c.hub_segs || (!DEFER && nseg)) {  // hub: hand the segments to the whole grid
                             const unsigned long long old =
                                 atomicAdd(c.hub_ctr, (1ull << 32) | (unsigned long long)nseg);
                             c.hubq[old >> 32] = HubEntry{segbase, u, (uint32_t)(old & 0xffffffffu)};
@@ -352,7 +368,7 @@ __global__ void __launch_bounds__(kBlock, 4) expand_kernel(Ctx c, Front fr, App 
                         const uint32_t su = sm.u[lo];
                         App t = app;
                         t.begin(su);
-                        na += decode_segment<K>(c.W, sm.base[lo] + (uint64_t)(sj - sm.spre[lo]) * c.seg_bits, su, t);
+                        na += decode_segment<K, STAGED>(c.W, sm.base[lo] + (uint64_t)(sj - sm.spre[lo]) * c.seg_bits, su, t);
                         t.end();
                     }
                 }
@@ -373,7 +389,7 @@ __global__ void __launch_bounds__(kBlock, 4) expand_kernel(Ctx c, Front fr, App 
 }
 
 // Hub segments of the level, flattened over the whole grid (one segment per thread at a time).
-template <int K, class App>
+template <int K, bool STAGED, class App>
 __global__ void __launch_bounds__(kBlock) hub_kernel(Ctx c, App app) {
     const unsigned long long hc = *c.hub_ctr;
     const uint32_t nh = (uint32_t)(hc >> 32), S = (uint32_t)(hc & 0xffffffffu);
@@ -387,7 +403,7 @@ __global__ void __launch_bounds__(kBlock) hub_kernel(Ctx c, App app) {
         const HubEntry e = c.hubq[lo];
         App t = app;
         t.begin(e.u);
-        na += decode_segment<K>(c.W, e.base + (j - e.seg_off) * (uint64_t)c.seg_bits, e.u, t);
+        na += decode_segment<K, STAGED>(c.W, e.base + (j - e.seg_off) * (uint64_t)c.seg_bits, e.u, t);
         t.end();
     }
     add_stats(c.st, 0, na, 0);
@@ -608,17 +624,17 @@ __global__ void bswap_words(uint64_t* w, uint64_t n) {
 // interval area / unsegmented list); sizes the per-level hub and heavy queues.
 template <int K, bool SEG>
 __global__ void count_special(const uint64_t* __restrict__ W, const uint64_t* __restrict__ offs, uint64_t n,
-                              unsigned long long* out) {
+                              uint32_t heavy_itv, uint32_t heavy_res, uint32_t hub_segs, unsigned long long* out) {
     uint32_t hubs = 0, heavy = 0;
     for (uint64_t u = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; u < n; u += (uint64_t)gridDim.x * blockDim.x) {
         uint64_t p = ldg64(offs + u);
         uint64_t deg = 0;
         if (!SEG) deg = decode<K>(W, p) - 1;
         const uint64_t itv = decode<K>(W, p) - 1;
-        if (itv > kHeavyItv || (!SEG && deg > kHeavyRes)) heavy++;
+        if (itv > heavy_itv || (!SEG && deg > heavy_res)) heavy++;
         if (SEG) {
             for (uint64_t i = 0; i < 2 * itv; i++) decode<K>(W, p);
-            if (decode<K>(W, p) - 1 > kHubSegs) hubs++;
+            if (decode<K>(W, p) - 1 > hub_segs) hubs++;
         }
     }
     for (int o = 16; o; o >>= 1) {
@@ -633,7 +649,7 @@ __global__ void count_special(const uint64_t* __restrict__ W, const uint64_t* __
 
 // ---- dispatch -------------------------------------------------------------------------------------------------------
 // Persistent launch: at most one wave (occupancy calculator), never more blocks than the work needs.
-template <int K, bool SEG, class App, class Front, bool DEFER>
+template <int K, bool SEG, class App, class Front, bool DEFER, bool STAGED>
 inline void launch_expand_k(int grid, cudaStream_t s, const Ctx& c, const Front& fr, const App& app, uint32_t wpb) {
     static int per_sm = 0;
     static int sms = 0;
@@ -641,20 +657,23 @@ inline void launch_expand_k(int grid, cudaStream_t s, const Ctx& c, const Front&
         int dev = 0;
         cudaGetDevice(&dev);
         cudaDeviceGetAttribute(&sms, cudaDevAttrMultiProcessorCount, dev);
-        cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per_sm, expand_kernel<K, SEG, App, Front, DEFER>, kBlock, 0);
+        cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per_sm, expand_kernel<K, SEG, App, Front, DEFER, STAGED>, kBlock,
+                                                      0);
         if (per_sm < 1) per_sm = 1;
     }
     grid = std::max(1, std::min(grid, per_sm * sms));
-    expand_kernel<K, SEG, App, Front, DEFER><<<grid, kBlock, 0, s>>>(c, fr, app, wpb);
+    expand_kernel<K, SEG, App, Front, DEFER, STAGED><<<grid, kBlock, 0, s>>>(c, fr, app, wpb);
 }
 
 template <class App, class Front, bool DEFER = true>
-inline void launch_expand(const gcgt_params& P, int grid, cudaStream_t s, const Ctx& c, const Front& fr,
-                          const App& app, uint32_t wpb) {
+inline void launch_expand(const gcgt_params& P, bool staged, int grid, cudaStream_t s, const Ctx& c,
+                          const Front& fr, const App& app, uint32_t wpb) {
     const bool seg = P.residual_segment_len != 0;
-#define GCGT_EXP(KK)                                                                                  \
-    (seg ? launch_expand_k<KK, true, App, Front, DEFER>(grid, s, c, fr, app, wpb)                      \
-         : launch_expand_k<KK, false, App, Front, DEFER>(grid, s, c, fr, app, wpb))
+#define GCGT_EXP(KK)                                                                                          \
+    (staged ? (seg ? launch_expand_k<KK, true, App, Front, DEFER, true>(grid, s, c, fr, app, wpb)              \
+                   : launch_expand_k<KK, false, App, Front, DEFER, true>(grid, s, c, fr, app, wpb))            \
+            : (seg ? launch_expand_k<KK, true, App, Front, DEFER, false>(grid, s, c, fr, app, wpb)             \
+                   : launch_expand_k<KK, false, App, Front, DEFER, false>(grid, s, c, fr, app, wpb)))
     switch (P.zeta_k) {
         case 1: GCGT_EXP(1); break;
         case 2: GCGT_EXP(2); break;
@@ -669,19 +688,23 @@ inline void launch_expand(const gcgt_params& P, int grid, cudaStream_t s, const 
 template <class App>
 inline void launch_heavy(const gcgt_graph* g, cudaStream_t s, const Ctx& c, const App& app) {
     const HeavyFront fr{c.heavyq, c.heavy_len};
-    launch_expand<App, HeavyFront, false>(g->P, g->num_sms * 8, s, c, fr, app, 32);
+    launch_expand<App, HeavyFront, false>(g->P, g->staged, g->num_sms * 8, s, c, fr, app, 32);
 }
 
 template <class App>
-inline void launch_hub(const gcgt_params& P, int grid, cudaStream_t s, const Ctx& c, const App& app) {
+inline void launch_hub(const gcgt_params& P, bool staged, int grid, cudaStream_t s, const Ctx& c, const App& app) {
     if (!P.residual_segment_len) return;
+#define GCGT_HUB(KK)                                                            \
+    (staged ? hub_kernel<KK, true, App><<<grid, kBlock, 0, s>>>(c, app)         \
+            : hub_kernel<KK, false, App><<<grid, kBlock, 0, s>>>(c, app))
     switch (P.zeta_k) {
-        case 1: hub_kernel<1, App><<<grid, kBlock, 0, s>>>(c, app); break;
-        case 2: hub_kernel<2, App><<<grid, kBlock, 0, s>>>(c, app); break;
-        case 3: hub_kernel<3, App><<<grid, kBlock, 0, s>>>(c, app); break;
-        case 4: hub_kernel<4, App><<<grid, kBlock, 0, s>>>(c, app); break;
-        default: hub_kernel<5, App><<<grid, kBlock, 0, s>>>(c, app); break;
+        case 1: GCGT_HUB(1); break;
+        case 2: GCGT_HUB(2); break;
+        case 3: GCGT_HUB(3); break;
+        case 4: GCGT_HUB(4); break;
+        default: GCGT_HUB(5); break;
     }
+#undef GCGT_HUB
 }
 
 // Work granularity for a frontier of qlen words: every resident warp should take several batches (dynamic
@@ -689,7 +712,7 @@ inline void launch_hub(const gcgt_params& P, int grid, cudaStream_t s, const Ctx
 inline void frontier_launch(const gcgt_graph* g, uint64_t qlen, int* grid, uint32_t* wpb) {
     const uint64_t resident_warps = (uint64_t)g->num_sms * 48;
     uint64_t b = qlen / (resident_warps * 4);
-    b = std::max<uint64_t>(1, std::min<uint64_t>(b, 8));
+    b = std::max<uint64_t>(1, std::min<uint64_t>(b, g->wpb_max));
     const uint64_t warps = (qlen + b - 1) / b;
     *grid = (int)std::max<uint64_t>(1, std::min<uint64_t>((warps + kWarps - 1) / kWarps, (uint64_t)g->num_sms * 32));
     *wpb = (uint32_t)b;
@@ -704,7 +727,7 @@ inline int hub_grid(const gcgt_graph* g) { return g->num_sms * 4; }
 inline Ctx make_ctx(const gcgt_graph* g) {
     return Ctx{g->W,     g->offs,     g->P.min_interval_len, 8 * g->P.residual_segment_len,
                g->hubq, g->hub_ctr, g->stats,              g->cursor,
-               g->heavyq, g->heavy_len};
+               g->heavyq, g->heavy_len, g->heavy_itv, g->heavy_res, g->hub_segs};
 }
 
 gcgt_status copy_out(gcgt_graph* g, void* dst, const void* src, size_t bytes, int placement) {
@@ -832,6 +855,26 @@ extern "C" gcgt_status gcgt_load(const gcgt_cgr* c, const gcgt_load_opts* opts, 
     g->n = c->n;
     g->nbits = c->nbits;
     g->P = c->params;
+    if (const char* tune = getenv("GCGT_TUNE")) {  // development knob: key=value,... (results never change)
+        std::string t(tune);
+        size_t i = 0;
+        while (i < t.size()) {
+            size_t j = t.find(',', i);
+            if (j == std::string::npos) j = t.size();
+            const std::string kv = t.substr(i, j - i);
+            const size_t e = kv.find('=');
+            if (e != std::string::npos) {
+                const std::string k = kv.substr(0, e);
+                const unsigned long v = strtoul(kv.c_str() + e + 1, nullptr, 10);
+                if (k == "staged") g->staged = v != 0;
+                else if (k == "heavy_itv") g->heavy_itv = (uint32_t)v;
+                else if (k == "heavy_res") g->heavy_res = (uint32_t)v;
+                else if (k == "hub_segs") g->hub_segs = (uint32_t)v;
+                else if (k == "wpb_max") g->wpb_max = (uint32_t)std::max(1ul, std::min(32ul, v));
+            }
+            i = j + 1;
+        }
+    }
     g->lo = 0;
     g->hi = c->n;
     g->nw = (c->n + 31) / 32 + 1;
@@ -864,11 +907,11 @@ extern "C" gcgt_status gcgt_load(const gcgt_cgr* c, const gcgt_load_opts* opts, 
         const bool seg = g->P.residual_segment_len != 0;
         cudaStream_t s = g->stream;
         switch (g->P.zeta_k) {
-            case 1: seg ? count_special<1, true><<<gr, kBlock, 0, s>>>(g->W, g->offs, g->n, dcount) : count_special<1, false><<<gr, kBlock, 0, s>>>(g->W, g->offs, g->n, dcount); break;
-            case 2: seg ? count_special<2, true><<<gr, kBlock, 0, s>>>(g->W, g->offs, g->n, dcount) : count_special<2, false><<<gr, kBlock, 0, s>>>(g->W, g->offs, g->n, dcount); break;
-            case 3: seg ? count_special<3, true><<<gr, kBlock, 0, s>>>(g->W, g->offs, g->n, dcount) : count_special<3, false><<<gr, kBlock, 0, s>>>(g->W, g->offs, g->n, dcount); break;
-            case 4: seg ? count_special<4, true><<<gr, kBlock, 0, s>>>(g->W, g->offs, g->n, dcount) : count_special<4, false><<<gr, kBlock, 0, s>>>(g->W, g->offs, g->n, dcount); break;
-            default: seg ? count_special<5, true><<<gr, kBlock, 0, s>>>(g->W, g->offs, g->n, dcount) : count_special<5, false><<<gr, kBlock, 0, s>>>(g->W, g->offs, g->n, dcount); break;
+            case 1: seg ? count_special<1, true><<<gr, kBlock, 0, s>>>(g->W, g->offs, g->n, g->heavy_itv, g->heavy_res, g->hub_segs, dcount) : count_special<1, false><<<gr, kBlock, 0, s>>>(g->W, g->offs, g->n, g->heavy_itv, g->heavy_res, g->hub_segs, dcount); break;
+            case 2: seg ? count_special<2, true><<<gr, kBlock, 0, s>>>(g->W, g->offs, g->n, g->heavy_itv, g->heavy_res, g->hub_segs, dcount) : count_special<2, false><<<gr, kBlock, 0, s>>>(g->W, g->offs, g->n, g->heavy_itv, g->heavy_res, g->hub_segs, dcount); break;
+            case 3: seg ? count_special<3, true><<<gr, kBlock, 0, s>>>(g->W, g->offs, g->n, g->heavy_itv, g->heavy_res, g->hub_segs, dcount) : count_special<3, false><<<gr, kBlock, 0, s>>>(g->W, g->offs, g->n, g->heavy_itv, g->heavy_res, g->hub_segs, dcount); break;
+            case 4: seg ? count_special<4, true><<<gr, kBlock, 0, s>>>(g->W, g->offs, g->n, g->heavy_itv, g->heavy_res, g->hub_segs, dcount) : count_special<4, false><<<gr, kBlock, 0, s>>>(g->W, g->offs, g->n, g->heavy_itv, g->heavy_res, g->hub_segs, dcount); break;
+            default: seg ? count_special<5, true><<<gr, kBlock, 0, s>>>(g->W, g->offs, g->n, g->heavy_itv, g->heavy_res, g->hub_segs, dcount) : count_special<5, false><<<gr, kBlock, 0, s>>>(g->W, g->offs, g->n, g->heavy_itv, g->heavy_res, g->hub_segs, dcount); break;
         }
     }
     unsigned long long counts[2] = {0, 0};
@@ -987,10 +1030,10 @@ extern "C" gcgt_status gcgt_bfs(gcgt_graph* g, uint32_t source, int32_t* levels,
         const QueueFront fr{q[cur], g->ctr + cur, g->F, nullptr};
         const BfsApp app{g->V, g->N, g->levels, (int32_t)level};
         if ((st = kprof_begin(g))) return st;
-        launch_expand(g->P, grid, s, c, fr, app, wpb);
+        launch_expand(g->P, g->staged, grid, s, c, fr, app, wpb);
         if ((st = kprof_end(g))) return st;
         launch_heavy(g, s, c, app);
-        launch_hub(g->P, hub_grid(g), s, c, app);
+        launch_hub(g->P, g->staged, hub_grid(g), s, c, app);
         commit_dense<<<flat_grid(g, g->nw), kBlock, 0, s>>>(g->V, g->F, g->N, 0, g->nw, q[nxt], g->ctr + nxt, nullptr,
                                                              g->ctr + cur, g->hub_ctr, g->heavy_len);
         CU(cudaMemcpyAsync(g->h_ctr + nxt, g->ctr + nxt, 4, cudaMemcpyDeviceToHost, s));
@@ -1019,10 +1062,10 @@ extern "C" gcgt_status gcgt_cc(gcgt_graph* g, uint32_t* labels, int placement, g
     uint32_t wpb;
     frontier_launch(g, (g->hi - g->lo + 31) / 32 + 1, &grid, &wpb);
     if ((st = kprof_begin(g))) return st;
-    launch_expand(g->P, grid, s, c, fr, app, wpb);
+    launch_expand(g->P, g->staged, grid, s, c, fr, app, wpb);
     if ((st = kprof_end(g))) return st;
     launch_heavy(g, s, c, app);
-    launch_hub(g->P, hub_grid(g), s, c, app);
+    launch_hub(g->P, g->staged, hub_grid(g), s, c, app);
     cc_jump<<<flat_grid(g, g->n), kBlock, 0, s>>>(g->parent, g->n);
     if ((st = copy_out(g, labels, g->parent, g->n * 4, placement))) return st;
     CU(cudaStreamSynchronize(s));
@@ -1077,10 +1120,10 @@ extern "C" gcgt_status gcgt_bc(gcgt_graph* g, const uint32_t* sources, uint32_t 
             const QueueFront fr{g->q + off, g->ctr + 2 + (level & 1), nullptr, g->qbits + off};
             const BcFwdApp app{g->V, g->N, g->levels, g->sigma, (int32_t)level, 0.0};
             if ((st = kprof_begin(g))) return st;
-            launch_expand(g->P, grid, s, c, fr, app, wpb);
+            launch_expand(g->P, g->staged, grid, s, c, fr, app, wpb);
             if ((st = kprof_end(g))) return st;
             launch_heavy(g, s, c, app);
-            launch_hub(g->P, hub_grid(g), s, c, app);
+            launch_hub(g->P, g->staged, hub_grid(g), s, c, app);
             commit_dense<<<flat_grid(g, g->nw), kBlock, 0, s>>>(g->V, nullptr, g->N, 0, g->nw, g->q + total,
                                                                  g->ctr + 2 + ((level + 1) & 1), g->qbits + total,
                                                                  g->ctr + 2 + (level & 1), g->hub_ctr,
@@ -1100,9 +1143,9 @@ extern "C" gcgt_status gcgt_bc(gcgt_graph* g, const uint32_t* sources, uint32_t 
             frontier_launch(g, qlen, &grid, &wpb);
             const QueueFront fr{g->q + off, g->ctr + 4, nullptr, g->qbits + off};
             const BcBwdApp app{g->levels, g->sigma, g->delta, g->bc, d + 1, src, 0, 0.0, 0.0};
-            launch_expand(g->P, grid, s, c, fr, app, wpb);
+            launch_expand(g->P, g->staged, grid, s, c, fr, app, wpb);
             launch_heavy(g, s, c, app);
-            launch_hub(g->P, hub_grid(g), s, c, app);
+            launch_hub(g->P, g->staged, hub_grid(g), s, c, app);
             CU(cudaMemsetAsync(g->hub_ctr, 0, sizeof(unsigned long long), s));
             CU(cudaMemsetAsync(g->heavy_len, 0, 4, s));
         }

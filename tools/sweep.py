@@ -1,0 +1,33 @@
+"""Times BFS on a config for several GCGT_TUNE settings (one process; the knobs are read at gcgt_load)."""
+import os
+import sys
+import time
+
+sys.path.insert(0, os.path.dirname(os.path.dirname(os.path.abspath(__file__))))
+import torch  # noqa: E402
+
+import paper_conf_sigmod_shalt19_b200 as G  # noqa: E402
+import synth  # noqa: E402
+
+cfg = synth.CONFIGS[sys.argv[1]]
+tunes = sys.argv[2:]
+ro, co = cfg.make()
+cgr = G.encode(ro, co, cfg.min_interval_len, cfg.residual_segment_len, cfg.zeta_k)
+roots = synth.pick_roots(ro, 8)
+out = torch.empty(ro.size - 1, dtype=torch.int32, device="cuda")
+for tune in tunes:
+    os.environ["GCGT_TUNE"] = tune
+    g = G.load(cgr, stream="torch")
+    for r in roots[:2]:
+        g.bfs(r, out=out)
+    g.profile(True)
+    t = 0.0
+    k = 0.0
+    for r in roots:
+        g.bfs(r, out=out)
+        t += g.last_stats["device_ms"]
+        k += g.last_stats["kernel_ms"]
+    arcs = g.last_stats["arcs_decoded"]
+    print(f"{tune:50s} bfs {t / len(roots):7.3f} ms  expand {k / len(roots):7.3f} ms  "
+          f"~{arcs / (t / len(roots)) / 1e6:6.1f} GTEPS(last root arcs)", flush=True)
+    g.unload()
