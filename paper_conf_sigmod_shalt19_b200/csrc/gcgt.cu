@@ -90,8 +90,10 @@ struct gcgt_graph {
     unsigned long long* cursor = nullptr;  // [0] work cursor, [1] finished-warp count (expand_kernel)
     HeavyEntry* heavyq = nullptr;          // per-level heavy-vertex queue (capacity = heavy vertices + 1)
     // tuning knobs (defaults; GCGT_TUNE="staged=0,heavy_itv=16,hub_segs=8,wpb_max=8" overrides at load)
-    bool staged = true;
-    uint32_t heavy_itv = 16, heavy_res = 64, hub_segs = 8, wpb_max = 8;
+    // defaults from the C2 sweep (profiles/r1_sweep_c2.txt): per-codeword window reads beat register staging, and
+    // deferring long interval areas to a separate pass costs more than the in-batch straggler it removes
+    bool staged = false;
+    uint32_t heavy_itv = 0xFFFFFFFFu, heavy_res = 1024, hub_segs = 8, wpb_max = 8;
     uint32_t* heavy_len = nullptr;
     unsigned long long* hub_ctr = nullptr;
     Stats* stats = nullptr;
