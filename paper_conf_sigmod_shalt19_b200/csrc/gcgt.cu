@@ -93,6 +93,7 @@ struct gcgt_graph {
     // defaults from the C2 sweep (profiles/r1_sweep_c2.txt): per-codeword window reads beat register staging, and
     // deferring long interval areas to a separate pass costs more than the in-batch straggler it removes
     bool staged = false;
+    bool persistent = true;  // BFS: all levels in one cooperative launch (GCGT_TUNE persistent=0: host loop)
     uint32_t heavy_itv = 0xFFFFFFFFu, heavy_res = 1024, hub_segs = 8, wpb_max = 8;
     uint32_t* heavy_len = nullptr;
     unsigned long long* hub_ctr = nullptr;
@@ -255,12 +256,11 @@ struct WarpSmem {
 // DEFER = true: the level's frontier pass (heavy vertices are queued); false: the heavy pass over that queue
 // (same engine, one lane per heavy vertex, nothing deferred, App::vertex and vertex stats already done).
 template <int K, bool SEG, class App, class Front, bool DEFER, bool STAGED>
-__global__ void __launch_bounds__(kBlock, 4) expand_kernel(Ctx c, Front fr, App app, uint32_t wpb) {
-    __shared__ WarpSmem smem[kWarps];
+__device__ __forceinline__ void expand_phase(const Ctx& c, const Front& fr, const App& app, uint32_t wpb,
+                                             WarpSmem* smem, uint64_t& nv, uint64_t& na, uint64_t& nb) {
     const uint32_t wid = threadIdx.x >> 5, lane = lane_id();
     WarpSmem& sm = smem[wid];
     const uint64_t qlen = fr.size();
-    uint64_t nv = 0, na = 0, nb = 0;
     unsigned long long next = 0;  // the next batch's cursor value is fetched one batch ahead (latency hidden)
     if (lane == 0) next = atomicAdd(c.cursor, (unsigned long long)wpb);
     for (;;) {
@@ -379,9 +379,16 @@ __global__ void __launch_bounds__(kBlock, 4) expand_kernel(Ctx c, Front fr, App 
         }
         __syncwarp();
     }
+}
+
+template <int K, bool SEG, class App, class Front, bool DEFER, bool STAGED>
+__global__ void __launch_bounds__(kBlock, 4) expand_kernel(Ctx c, Front fr, App app, uint32_t wpb) {
+    __shared__ WarpSmem smem[kWarps];
+    uint64_t nv = 0, na = 0, nb = 0;
+    expand_phase<K, SEG, App, Front, DEFER, STAGED>(c, fr, app, wpb, smem, nv, na, nb);
     add_stats(c.st, nv, na, nb);
     // the last warp out resets the work cursor for the next launch
-    if (lane == 0) {
+    if (lane_id() == 0) {
         const unsigned long long nw = (unsigned long long)gridDim.x * kWarps;
         if (atomicAdd(c.cursor + 1, 1ull) == nw - 1) {
             c.cursor[0] = 0;
@@ -392,10 +399,9 @@ __global__ void __launch_bounds__(kBlock, 4) expand_kernel(Ctx c, Front fr, App 
 
 // Hub segments of the level, flattened over the whole grid (one segment per thread at a time).
 template <int K, bool STAGED, class App>
-__global__ void __launch_bounds__(kBlock) hub_kernel(Ctx c, App app) {
-    const unsigned long long hc = *c.hub_ctr;
+__device__ __forceinline__ void hub_phase(const Ctx& c, const App& app, uint64_t& na) {
+    const unsigned long long hc = *(volatile unsigned long long*)c.hub_ctr;
     const uint32_t nh = (uint32_t)(hc >> 32), S = (uint32_t)(hc & 0xffffffffu);
-    uint64_t na = 0;
     for (uint64_t j = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; j < S; j += (uint64_t)gridDim.x * blockDim.x) {
         uint32_t lo = 0, hi = nh - 1;  // entry: largest e with seg_off <= j
         while (lo < hi) {
@@ -408,6 +414,12 @@ __global__ void __launch_bounds__(kBlock) hub_kernel(Ctx c, App app) {
         na += decode_segment<K, STAGED>(c.W, e.base + (j - e.seg_off) * (uint64_t)c.seg_bits, e.u, t);
         t.end();
     }
+}
+
+template <int K, bool STAGED, class App>
+__global__ void __launch_bounds__(kBlock) hub_kernel(Ctx c, App app) {
+    uint64_t na = 0;
+    hub_phase<K, STAGED>(c, app, na);
     add_stats(c.st, 0, na, 0);
 }
 
@@ -573,10 +585,10 @@ __global__ void cc_init(uint32_t* parent, uint64_t n) {
 // ---- contraction ---------------------------------------------------------------------------------------------------
 // Dense scan of N over words [w_lo, w_hi): every non-zero word is folded into V (and F), cleared, and appended to
 // the next queue (one atomic per warp).  Also resets the hub counter and the consumed queue's length.
-__global__ void commit_dense(uint32_t* __restrict__ V, uint32_t* __restrict__ F, uint32_t* __restrict__ N,
-                             uint64_t w_lo, uint64_t w_hi, uint32_t* __restrict__ qn, uint32_t* __restrict__ qn_len,
-                             uint32_t* __restrict__ qbits_out, uint32_t* __restrict__ reset_ctr,
-                             unsigned long long* __restrict__ hub_ctr, uint32_t* __restrict__ heavy_len) {
+__device__ __forceinline__ void commit_phase(uint32_t* __restrict__ V, uint32_t* __restrict__ F,
+                                             uint32_t* __restrict__ N, uint64_t w_lo, uint64_t w_hi,
+                                             uint32_t* __restrict__ qn, uint32_t* __restrict__ qn_len,
+                                             uint32_t* __restrict__ qbits_out) {
     const uint32_t lane = lane_id();
     const uint64_t gw = ((uint64_t)blockIdx.x * blockDim.x + threadIdx.x) >> 5;
     const uint64_t nwarps = ((uint64_t)gridDim.x * blockDim.x) >> 5;
@@ -602,11 +614,69 @@ __global__ void commit_dense(uint32_t* __restrict__ V, uint32_t* __restrict__ F,
             }
         }
     }
+}
+
+__global__ void commit_dense(uint32_t* __restrict__ V, uint32_t* __restrict__ F, uint32_t* __restrict__ N,
+                             uint64_t w_lo, uint64_t w_hi, uint32_t* __restrict__ qn, uint32_t* __restrict__ qn_len,
+                             uint32_t* __restrict__ qbits_out, uint32_t* __restrict__ reset_ctr,
+                             unsigned long long* __restrict__ hub_ctr, uint32_t* __restrict__ heavy_len) {
+    commit_phase(V, F, N, w_lo, w_hi, qn, qn_len, qbits_out);
     if (blockIdx.x == 0 && threadIdx.x == 0) {
         if (reset_ctr) *reset_ctr = 0;
         if (hub_ctr) *hub_ctr = 0;
         if (heavy_len) *heavy_len = 0;
     }
+}
+
+// ---- persistent BFS: every level inside one cooperative launch ------------------------------------------------------
+// Per level: expansion (work cursor) | grid sync | hub segments | grid sync | contraction into the next queue |
+// grid sync.  No host round trip per level: the host launches once and waits once (high-diameter web graphs have
+// dozens of levels, and each host-driven level costs launches plus a stream synchronisation).
+struct BfsPersist {
+    uint32_t* q0;
+    uint32_t* q1;
+    uint32_t* ctr;     // [0], [1]: queue lengths (ping-pong); [6]: levels expanded (out)
+    uint32_t* V;
+    uint32_t* F;
+    uint32_t* N;
+    int32_t* levels;
+    uint64_t nw;
+    uint32_t wpb_max;
+};
+
+template <int K, bool SEG>
+__global__ void __launch_bounds__(kBlock, 4) bfs_persistent(Ctx c, BfsPersist b) {
+    __shared__ WarpSmem smem[kWarps];
+    cg::grid_group grid = cg::this_grid();
+    uint64_t nv = 0, na = 0, nb = 0;
+    const uint64_t nwarps = (uint64_t)gridDim.x * kWarps;
+    uint32_t level = 0;
+    for (;; level++) {
+        const int cur = level & 1, nxt = cur ^ 1;
+        uint32_t* qc = cur ? b.q1 : b.q0;
+        uint32_t* qn = cur ? b.q0 : b.q1;
+        const uint64_t qlen = *(volatile uint32_t*)(b.ctr + cur);
+        uint64_t wpb = qlen / (nwarps * 4);
+        wpb = wpb < 1 ? 1 : (wpb > b.wpb_max ? b.wpb_max : wpb);
+        const QueueFront fr{qc, b.ctr + cur, b.F, nullptr};
+        const BfsApp app{b.V, b.N, b.levels, (int32_t)level};
+        expand_phase<K, SEG, BfsApp, QueueFront, true, false>(c, fr, app, (uint32_t)wpb, smem, nv, na, nb);
+        grid.sync();
+        if (SEG) {
+            hub_phase<K, false>(c, app, na);
+            grid.sync();
+        }
+        commit_phase(b.V, b.F, b.N, 0, b.nw, qn, b.ctr + nxt, nullptr);
+        if (blockIdx.x == 0 && threadIdx.x == 0) {
+            b.ctr[cur] = 0;
+            *c.hub_ctr = 0;
+            c.cursor[0] = 0;
+        }
+        grid.sync();
+        if (*(volatile uint32_t*)(b.ctr + nxt) == 0) break;
+    }
+    add_stats(c.st, nv, na, nb);
+    if (blockIdx.x == 0 && threadIdx.x == 0) b.ctr[6] = level + 1;
 }
 
 __global__ void bfs_seed(uint32_t s, uint32_t* V, uint32_t* F, uint32_t* q, uint32_t* qlen, uint32_t* qbits) {
@@ -691,6 +761,34 @@ template <class App>
 inline void launch_heavy(const gcgt_graph* g, cudaStream_t s, const Ctx& c, const App& app) {
     const HeavyFront fr{c.heavyq, c.heavy_len};
     launch_expand<App, HeavyFront, false>(g->P, g->staged, g->num_sms * 8, s, c, fr, app, 32);
+}
+
+// Cooperative launch of the persistent BFS (one wave, co-resident blocks).  Returns false if the device cannot
+// co-schedule the grid (then the host-driven level loop is used).
+template <int K, bool SEG>
+inline cudaError_t launch_bfs_persistent_k(const gcgt_graph* g, cudaStream_t s, Ctx c, BfsPersist b) {
+    static int per_sm = -1;
+    if (per_sm < 0) {
+        if (cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per_sm, bfs_persistent<K, SEG>, kBlock, 0) != cudaSuccess)
+            per_sm = 0;
+    }
+    if (per_sm < 1) return cudaErrorCooperativeLaunchTooLarge;
+    void* args[] = {(void*)&c, (void*)&b};
+    return cudaLaunchCooperativeKernel((const void*)bfs_persistent<K, SEG>, dim3(per_sm * g->num_sms), dim3(kBlock),
+                                       args, 0, s);
+}
+
+inline cudaError_t launch_bfs_persistent(const gcgt_graph* g, cudaStream_t s, Ctx c, const BfsPersist& b) {
+    c.heavy_itv = 0xFFFFFFFFu;  // nothing is deferred inside the persistent loop
+    c.heavy_res = 0xFFFFFFFFu;
+    const bool seg = g->P.residual_segment_len != 0;
+    switch (g->P.zeta_k) {
+        case 1: return seg ? launch_bfs_persistent_k<1, true>(g, s, c, b) : launch_bfs_persistent_k<1, false>(g, s, c, b);
+        case 2: return seg ? launch_bfs_persistent_k<2, true>(g, s, c, b) : launch_bfs_persistent_k<2, false>(g, s, c, b);
+        case 3: return seg ? launch_bfs_persistent_k<3, true>(g, s, c, b) : launch_bfs_persistent_k<3, false>(g, s, c, b);
+        case 4: return seg ? launch_bfs_persistent_k<4, true>(g, s, c, b) : launch_bfs_persistent_k<4, false>(g, s, c, b);
+        default: return seg ? launch_bfs_persistent_k<5, true>(g, s, c, b) : launch_bfs_persistent_k<5, false>(g, s, c, b);
+    }
 }
 
 template <class App>
@@ -869,6 +967,7 @@ extern "C" gcgt_status gcgt_load(const gcgt_cgr* c, const gcgt_load_opts* opts, 
                 const std::string k = kv.substr(0, e);
                 const unsigned long v = strtoul(kv.c_str() + e + 1, nullptr, 10);
                 if (k == "staged") g->staged = v != 0;
+                else if (k == "persistent") g->persistent = v != 0;
                 else if (k == "heavy_itv") g->heavy_itv = (uint32_t)v;
                 else if (k == "heavy_res") g->heavy_res = (uint32_t)v;
                 else if (k == "hub_segs") g->hub_segs = (uint32_t)v;
@@ -1024,6 +1123,22 @@ extern "C" gcgt_status gcgt_bfs(gcgt_graph* g, uint32_t source, int32_t* levels,
     const Ctx c = make_ctx(g);
     uint64_t qlen = 1;
     uint32_t level = 0;
+    if (g->persistent) {
+        const BfsPersist b{q[0], q[1], g->ctr, g->V, g->F, g->N, g->levels, g->nw, g->wpb_max};
+        if ((st = kprof_begin(g))) return st;
+        const cudaError_t e = launch_bfs_persistent(g, s, c, b);
+        if (e == cudaSuccess) {
+            if ((st = kprof_end(g))) return st;
+            CU(cudaMemcpyAsync(g->h_ctr + 6, g->ctr + 6, 4, cudaMemcpyDeviceToHost, s));
+            CU(cudaStreamSynchronize(s));
+            if ((st = kprof_collect(g))) return st;
+            level = g->h_ctr[6];
+            qlen = 0;  // done
+        } else {
+            cudaGetLastError();  // cannot co-schedule: fall through to the host-driven loop
+            g->persistent = false;
+        }
+    }
     while (qlen) {
         const int cur = level & 1, nxt = cur ^ 1;
         int grid;
