@@ -93,7 +93,7 @@ struct gcgt_graph {
     // defaults from the C2 sweep (profiles/r1_sweep_c2.txt): per-codeword window reads beat register staging, and
     // deferring long interval areas to a separate pass costs more than the in-batch straggler it removes
     bool staged = false;
-    bool persistent = true;  // BFS: all levels in one cooperative launch (GCGT_TUNE persistent=0: host loop)
+    bool persistent = false;  // BFS: all levels in one cooperative launch (measured slower on C2; GCGT_TUNE knob)
     uint32_t heavy_itv = 0xFFFFFFFFu, heavy_res = 1024, hub_segs = 8, wpb_max = 8;
     uint32_t* heavy_len = nullptr;
     unsigned long long* hub_ctr = nullptr;
@@ -261,6 +261,10 @@ __device__ __forceinline__ void expand_phase(const Ctx& c, const Front& fr, cons
     const uint32_t wid = threadIdx.x >> 5, lane = lane_id();
     WarpSmem& sm = smem[wid];
     const uint64_t qlen = fr.size();
+    if (wpb == 0) {  // sized on the device (host did not wait for the queue length): ~4 batches per resident warp
+        const uint64_t b = qlen / ((uint64_t)gridDim.x * kWarps * 4);
+        wpb = b < 1 ? 1 : (b > 8 ? 8 : (uint32_t)b);
+    }
     unsigned long long next = 0;  // the next batch's cursor value is fetched one batch ahead (latency hidden)
     if (lane == 0) next = atomicAdd(c.cursor, (unsigned long long)wpb);
     for (;;) {
@@ -677,6 +681,11 @@ __global__ void __launch_bounds__(kBlock, 4) bfs_persistent(Ctx c, BfsPersist b)
     }
     add_stats(c.st, nv, na, nb);
     if (blockIdx.x == 0 && threadIdx.x == 0) b.ctr[6] = level + 1;
+}
+
+// Counts expanded levels on the device: a level that produced a non-empty next queue adds one.
+__global__ void count_level(const uint32_t* qn_len, uint32_t* counter) {
+    if (*qn_len) *counter += 1;
 }
 
 __global__ void bfs_seed(uint32_t s, uint32_t* V, uint32_t* F, uint32_t* q, uint32_t* qlen, uint32_t* qbits) {
@@ -1139,26 +1148,38 @@ extern "C" gcgt_status gcgt_bfs(gcgt_graph* g, uint32_t source, int32_t* levels,
             g->persistent = false;
         }
     }
+    // Host-driven level loop without a per-level wait: the kernels size their work from the device-resident queue
+    // length, so the host enqueues kChunk levels at a time and checks for an empty queue once per chunk (levels
+    // enqueued past the end find an empty queue and exit at once).  With profiling on, the loop waits per level to
+    // time the expansion kernel.
+    constexpr uint32_t kChunk = 4;
     while (qlen) {
-        const int cur = level & 1, nxt = cur ^ 1;
-        int grid;
-        uint32_t wpb;
-        frontier_launch(g, qlen, &grid, &wpb);
-        const QueueFront fr{q[cur], g->ctr + cur, g->F, nullptr};
-        const BfsApp app{g->V, g->N, g->levels, (int32_t)level};
-        if ((st = kprof_begin(g))) return st;
-        launch_expand(g->P, g->staged, grid, s, c, fr, app, wpb);
-        if ((st = kprof_end(g))) return st;
-        launch_heavy(g, s, c, app);
-        launch_hub(g->P, g->staged, hub_grid(g), s, c, app);
-        commit_dense<<<flat_grid(g, g->nw), kBlock, 0, s>>>(g->V, g->F, g->N, 0, g->nw, q[nxt], g->ctr + nxt, nullptr,
-                                                             g->ctr + cur, g->hub_ctr, g->heavy_len);
-        CU(cudaMemcpyAsync(g->h_ctr + nxt, g->ctr + nxt, 4, cudaMemcpyDeviceToHost, s));
+        const uint32_t nlev = g->profile ? 1 : kChunk;
+        for (uint32_t i = 0; i < nlev; i++, level++) {
+            const int cur = level & 1, nxt = cur ^ 1;
+            int grid;
+            uint32_t wpb;
+            frontier_launch(g, level == 0 ? 1 : (uint64_t)g->nw, &grid, &wpb);
+            if (level == 0) wpb = 1;
+            else wpb = 0;  // device-side sizing
+            const QueueFront fr{q[cur], g->ctr + cur, g->F, nullptr};
+            const BfsApp app{g->V, g->N, g->levels, (int32_t)level};
+            if ((st = kprof_begin(g))) return st;
+            launch_expand(g->P, g->staged, grid, s, c, fr, app, wpb);
+            if ((st = kprof_end(g))) return st;
+            launch_heavy(g, s, c, app);
+            launch_hub(g->P, g->staged, hub_grid(g), s, c, app);
+            commit_dense<<<flat_grid(g, g->nw), kBlock, 0, s>>>(g->V, g->F, g->N, 0, g->nw, q[nxt], g->ctr + nxt,
+                                                                 nullptr, g->ctr + cur, g->hub_ctr, g->heavy_len);
+            count_level<<<1, 1, 0, s>>>(g->ctr + nxt, g->ctr + 6);
+        }
+        CU(cudaMemcpyAsync(g->h_ctr + 6, g->ctr + 6, 4, cudaMemcpyDeviceToHost, s));
+        CU(cudaMemcpyAsync(g->h_ctr + (level & 1), g->ctr + (level & 1), 4, cudaMemcpyDeviceToHost, s));
         CU(cudaStreamSynchronize(s));
         if ((st = kprof_collect(g))) return st;
-        qlen = g->h_ctr[nxt];
-        level++;
+        qlen = g->h_ctr[level & 1];
     }
+    if (!g->persistent || level == 0) level = g->h_ctr[6] + 1;  // non-empty levels expanded (seed level included)
     if ((st = copy_out(g, levels, g->levels, g->n * 4, placement))) return st;
     return end_call(g, stats, level);
 }
