@@ -267,3 +267,51 @@ struct RegStream {
 };
 
 }  // namespace gcgt_dev
+
+namespace gcgt_dev {
+
+// Sequential bit-buffer reader: the next stream bits left-aligned in a 64-bit register, refilled 32 bits at a
+// time (32-bit stream word j is ((const uint32_t*)W)[j ^ 1] because W holds 64-bit words in stream order on a
+// little-endian machine).  Per codeword: CLZ, two shifts, a length check and an occasional 32-bit load, all in
+// 32-bit-friendly arithmetic.  Codewords longer than the buffered bits take the global slow path.
+struct BitBuf {
+    uint64_t buf;    // next bits, MSB first
+    uint32_t avail;  // valid bits in buf
+    uint64_t nxt;    // next 32-bit stream word to load
+
+    __device__ __forceinline__ static uint32_t ld32(const uint64_t* __restrict__ W, uint64_t j) {
+        return __ldg(reinterpret_cast<const unsigned int*>(W) + (j ^ 1));
+    }
+    __device__ __forceinline__ void init(const uint64_t* __restrict__ W, uint64_t p) {
+        const uint64_t j = p >> 5;
+        const uint32_t off = (uint32_t)(p & 31);
+        buf = (((uint64_t)ld32(W, j) << 32) | ld32(W, j + 1)) << off;
+        avail = 64 - off;
+        nxt = j + 2;
+    }
+    __device__ __forceinline__ uint64_t pos() const { return nxt * 32 - avail; }
+    template <int K>
+    __device__ __forceinline__ uint64_t next(const uint64_t* __restrict__ W) {
+        if (avail <= 32) {
+            buf |= (uint64_t)ld32(W, nxt) << (32 - avail);
+            avail += 32;
+            nxt++;
+        }
+        const uint32_t z = (uint32_t)__clzll((long long)buf);
+        uint32_t L, h = 0;
+        if (K == 1) L = 2 * z + 1;
+        else { h = z + 1; L = h * (K + 1); }
+        if (L < 64 && L <= avail) {
+            const uint64_t v = K == 1 ? buf >> (64 - L) : (buf << h) >> (64 - K * h);
+            buf <<= L;
+            avail -= L;
+            return v;
+        }
+        uint64_t p = pos();  // long codeword (e.g. a segment's first residual): 64-bit window path, then re-seat
+        const uint64_t v = decode<K>(W, p);
+        init(W, p);
+        return v;
+    }
+};
+
+}  // namespace gcgt_dev

@@ -93,7 +93,8 @@ struct gcgt_graph {
     // defaults from the C2 sweep (profiles/r1_sweep_c2.txt): per-codeword window reads beat register staging, and
     // deferring long interval areas to a separate pass costs more than the in-batch straggler it removes
     bool staged = false;
-    bool persistent = false;  // BFS: all levels in one cooperative launch (measured slower on C2; GCGT_TUNE knob)
+    bool persistent = false;
+    uint32_t engine = 1;  // BFS: all levels in one cooperative launch (measured slower on C2; GCGT_TUNE knob)
     uint32_t heavy_itv = 0xFFFFFFFFu, heavy_res = 1024, hub_segs = 8, wpb_max = 8;
     uint32_t* heavy_len = nullptr;
     unsigned long long* hub_ctr = nullptr;
@@ -138,6 +139,7 @@ struct Ctx {
     uint32_t heavy_itv;           // interval count above which a vertex is deferred to the heavy pass
     uint32_t heavy_res;           // unsegmented residual count above which a vertex is deferred
     uint32_t hub_segs;            // segment count above which a vertex's segments go to the hub queue
+    uint32_t engine;              // 1 = state-machine kernel (sm_expand_kernel), 0 = phase kernel (expand_kernel)
 };
 
 __device__ __forceinline__ void add_stats(Stats* st, uint64_t v, uint64_t a, uint64_t b) {
@@ -393,6 +395,244 @@ __global__ void __launch_bounds__(kBlock, 4) expand_kernel(Ctx c, Front fr, App 
     add_stats(c.st, nv, na, nb);
     // the last warp out resets the work cursor for the next launch
     if (lane_id() == 0) {
+        const unsigned long long nw = (unsigned long long)gridDim.x * kWarps;
+        if (atomicAdd(c.cursor + 1, 1ull) == nw - 1) {
+            c.cursor[0] = 0;
+            c.cursor[1] = 0;
+        }
+    }
+}
+
+// ---- the state-machine expansion kernel (default) ---------------------------------------------------------------
+// Every lane runs a small state machine over "tasks": a vertex task decodes the record header and the interval
+// area (each interval handed over as a range claim) and queues the vertex's residual segments; a segment task
+// decodes one residual segment (FORMAT.md R17).  Each loop iteration every busy lane decodes exactly ONE codeword
+// (BitBuf) and acts on it, so the warp's lanes stay busy regardless of how skewed the records are; lanes that
+// finish take the next task at a warp-uniform refill point: first segments from the warp's ring (64 entries in
+// shared memory), then vertices of the current frontier batch, fetching a new batch from the global work cursor
+// when the batch is used up.  This is the paper's Task Stealing (Alg. 3, §4.3 :884-930) and Residual Segmentation
+// (§5.2) recast as a warp-level scheduler: idle lanes steal whole segments instead of decoded neighbours.
+// Vertices with more than hub_segs segments (or overflowing the ring) go to the grid-wide hub queue.
+constexpr uint32_t kRing = 64;
+constexpr uint32_t kList = 256;  // 8 queue words x 32 vertices
+
+struct SmWarp {
+    uint32_t list[kList];
+    uint32_t ring_u[kRing];
+    uint64_t ring_p[kRing];
+    uint32_t head, tail;
+};
+
+enum : uint32_t { ST_DONE = 0, ST_DEG, ST_ITVN, ST_GAP, ST_LEN, ST_SEGN, ST_RES, ST_SCNT, ST_SFIRST, ST_SGAP };
+
+template <int K, bool SEG, class App, class Front>
+__global__ void __launch_bounds__(kBlock, 4) sm_expand_kernel(Ctx c, Front fr, App app, uint32_t wpb) {
+    __shared__ SmWarp smem[kWarps];
+    const uint32_t wid = threadIdx.x >> 5, lane = lane_id(), lt = lanemask_lt();
+    SmWarp& sm = smem[wid];
+    const uint64_t qlen = fr.size();
+    if (wpb == 0) {
+        const uint64_t b = qlen / ((uint64_t)gridDim.x * kWarps * 4);
+        wpb = b < 1 ? 1 : (b > 8 ? 8 : (uint32_t)b);
+    }
+    if (wpb > kList / 32) wpb = kList / 32;
+    if (lane == 0) sm.head = sm.tail = 0;
+    uint32_t list_n = 0, list_pos = 0;  // warp-uniform
+    bool cursor_done = false;
+    unsigned long long next = 0;
+    if (lane == 0) next = atomicAdd(c.cursor, (unsigned long long)wpb);
+    // per-lane task state
+    uint32_t state = ST_DONE, u = 0, i = 0, cnt = 0, start = 0, cur = 0, push_n = 0;
+    uint64_t push_base = 0, rem = 0;
+    BitBuf bb{0, 0, 0};
+    App t = app;
+    uint64_t nv = 0, na = 0, nb = 0;
+    __syncwarp();
+    for (;;) {
+        // ---- queue the segments produced by the last step (warp scan over the pushes)
+        const uint32_t pmask = __ballot_sync(0xffffffffu, push_n != 0);
+        if (pmask) {
+            uint32_t incl = push_n;
+            for (int o = 1; o < 32; o <<= 1) {
+                const uint32_t tt = __shfl_up_sync(0xffffffffu, incl, o);
+                if (lane >= (uint32_t)o) incl += tt;
+            }
+            const uint32_t head = sm.head, tail = sm.tail, space = kRing - (tail - head);
+            if (push_n) {
+                const uint32_t off = incl - push_n;
+                if (incl <= space) {
+                    for (uint32_t k = 0; k < push_n; k++) {
+                        const uint32_t slot = (tail + off + k) % kRing;
+                        sm.ring_u[slot] = u;
+                        sm.ring_p[slot] = push_base + (uint64_t)k * c.seg_bits;
+                    }
+                } else {  // ring full: the grid-wide hub queue takes them
+                    const unsigned long long old = atomicAdd(c.hub_ctr, (1ull << 32) | (unsigned long long)push_n);
+                    c.hubq[old >> 32] = HubEntry{push_base, u, (uint32_t)(old & 0xffffffffu)};
+                }
+                push_n = 0;
+            }
+            __syncwarp();
+            // pushes are stored in lane order while they fit, so the stored ones are a prefix of the pushers
+            const uint32_t stored = __reduce_max_sync(0xffffffffu, (incl <= space && (pmask >> lane) & 1u) ? incl : 0u);
+            if (lane == 0) sm.tail = tail + stored;
+            __syncwarp();
+        }
+        // ---- refill idle lanes (warp-uniform)
+        uint32_t idle = __ballot_sync(0xffffffffu, state == ST_DONE);
+        if (idle) {
+            const uint32_t head = sm.head, avail = sm.tail - head;
+            if (avail) {
+                const uint32_t r = __popc(idle & lt), take = min(avail, (uint32_t)__popc(idle));
+                if (state == ST_DONE && r < take) {
+                    const uint32_t slot = (head + r) % kRing;
+                    u = sm.ring_u[slot];
+                    bb.init(c.W, sm.ring_p[slot]);
+                    t = app;
+                    t.begin(u);
+                    state = ST_SCNT;
+                }
+                __syncwarp();
+                if (lane == 0) sm.head = head + take;
+                __syncwarp();
+                idle = __ballot_sync(0xffffffffu, state == ST_DONE);
+            }
+            while (idle) {
+                if (list_pos >= list_n) {
+                    if (cursor_done) break;
+                    const uint64_t base = __shfl_sync(0xffffffffu, next, 0);
+                    if (base >= qlen) {
+                        cursor_done = true;
+                        break;
+                    }
+                    if (lane == 0) next = atomicAdd(c.cursor, (unsigned long long)wpb);
+                    uint32_t w = 0, bits = 0;
+                    if (lane < wpb && base + lane < qlen) fr.get(base + lane, w, bits);
+                    uint32_t incl = __popc(bits);
+                    for (int o = 1; o < 32; o <<= 1) {
+                        const uint32_t tt = __shfl_up_sync(0xffffffffu, incl, o);
+                        if (lane >= (uint32_t)o) incl += tt;
+                    }
+                    uint32_t pos = incl - __popc(bits);
+                    for (uint32_t bm = bits; bm; bm &= bm - 1) sm.list[pos++] = w * 32 + (__ffs(bm) - 1);
+                    list_n = __shfl_sync(0xffffffffu, incl, 31);
+                    list_pos = 0;
+                    __syncwarp();
+                    continue;
+                }
+                const uint32_t r = __popc(idle & lt), take = min(list_n - list_pos, (uint32_t)__popc(idle));
+                if (state == ST_DONE && r < take) {
+                    u = sm.list[list_pos + r];
+                    const uint64_t p = ldg64(c.offs + u);
+                    nb += ldg64(c.offs + u + 1) - p;
+                    nv++;
+                    t = app;
+                    t.begin(u);
+                    t.vertex(u);
+                    bb.init(c.W, p);
+                    state = SEG ? ST_ITVN : ST_DEG;
+                }
+                list_pos += take;
+                idle = __ballot_sync(0xffffffffu, state == ST_DONE);
+            }
+            if (idle == 0xffffffffu) {
+                if (cursor_done && list_pos >= list_n && sm.head == sm.tail) break;
+                continue;  // (cannot happen with work pending; defensive)
+            }
+        }
+        // ---- one step: every busy lane decodes one codeword and acts on it
+        if (state != ST_DONE) {
+            const uint64_t v = bb.template next<K>(c.W);
+            bool itv_done = false;
+            switch (state) {
+                case ST_DEG:
+                    rem = v - 1;
+                    state = ST_ITVN;
+                    break;
+                case ST_ITVN:
+                    cnt = (uint32_t)(v - 1);
+                    i = 0;
+                    if (cnt) state = ST_GAP;
+                    else itv_done = true;
+                    break;
+                case ST_GAP:
+                    start = i == 0 ? (uint32_t)unmap_first(u, v) : cur + (uint32_t)v;
+                    state = ST_LEN;
+                    break;
+                case ST_LEN: {
+                    const uint32_t len = (uint32_t)(v - 1) + c.min_len;
+                    t.range(start, len);
+                    na += len;
+                    if (!SEG) rem -= len;
+                    cur = start + len - 1;
+                    if (++i < cnt) state = ST_GAP;
+                    else itv_done = true;
+                    break;
+                }
+                case ST_SEGN: {
+                    const uint32_t nseg = (uint32_t)(v - 1);
+                    t.end();
+                    state = ST_DONE;
+                    if (nseg > c.hub_segs) {
+                        const unsigned long long old = atomicAdd(c.hub_ctr, (1ull << 32) | (unsigned long long)nseg);
+                        c.hubq[old >> 32] = HubEntry{bb.pos(), u, (uint32_t)(old & 0xffffffffu)};
+                    } else if (nseg) {
+                        push_n = nseg;
+                        push_base = bb.pos();
+                    }
+                    break;
+                }
+                case ST_RES:
+                    cur = i == 0 ? (uint32_t)unmap_first(u, v) : cur + (uint32_t)v;
+                    t.one(cur);
+                    na++;
+                    if (++i == rem) {
+                        t.end();
+                        state = ST_DONE;
+                    }
+                    break;
+                case ST_SCNT:
+                    cnt = (uint32_t)(v - 1);
+                    i = 0;
+                    state = ST_SFIRST;
+                    break;
+                case ST_SFIRST:
+                    cur = (uint32_t)unmap_first(u, v);
+                    t.one(cur);
+                    na++;
+                    if (++i == cnt) {
+                        t.end();
+                        state = ST_DONE;
+                    } else {
+                        state = ST_SGAP;
+                    }
+                    break;
+                case ST_SGAP:
+                    cur += (uint32_t)v;
+                    t.one(cur);
+                    na++;
+                    if (++i == cnt) {
+                        t.end();
+                        state = ST_DONE;
+                    }
+                    break;
+            }
+            if (itv_done) {
+                if (SEG) {
+                    state = ST_SEGN;
+                } else if (rem) {
+                    state = ST_RES;
+                    i = 0;
+                } else {
+                    t.end();
+                    state = ST_DONE;
+                }
+            }
+        }
+        __syncwarp();
+    }
+    add_stats(c.st, nv, na, nb);
+    if (lane == 0) {
         const unsigned long long nw = (unsigned long long)gridDim.x * kWarps;
         if (atomicAdd(c.cursor + 1, 1ull) == nw - 1) {
             c.cursor[0] = 0;
@@ -732,12 +972,24 @@ __global__ void count_special(const uint64_t* __restrict__ W, const uint64_t* __
 // Persistent launch: at most one wave (occupancy calculator), never more blocks than the work needs.
 template <int K, bool SEG, class App, class Front, bool DEFER, bool STAGED>
 inline void launch_expand_k(int grid, cudaStream_t s, const Ctx& c, const Front& fr, const App& app, uint32_t wpb) {
-    static int per_sm = 0;
     static int sms = 0;
-    if (!per_sm) {
+    if (!sms) {
         int dev = 0;
         cudaGetDevice(&dev);
         cudaDeviceGetAttribute(&sms, cudaDevAttrMultiProcessorCount, dev);
+    }
+    if (DEFER && c.engine == 1) {  // state-machine kernel (default); no heavy deferral needed
+        static int per_sm = 0;
+        if (!per_sm) {
+            cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per_sm, sm_expand_kernel<K, SEG, App, Front>, kBlock, 0);
+            if (per_sm < 1) per_sm = 1;
+        }
+        grid = std::max(1, std::min(grid, per_sm * sms));
+        sm_expand_kernel<K, SEG, App, Front><<<grid, kBlock, 0, s>>>(c, fr, app, wpb);
+        return;
+    }
+    static int per_sm = 0;
+    if (!per_sm) {
         cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per_sm, expand_kernel<K, SEG, App, Front, DEFER, STAGED>, kBlock,
                                                       0);
         if (per_sm < 1) per_sm = 1;
@@ -768,6 +1020,7 @@ inline void launch_expand(const gcgt_params& P, bool staged, int grid, cudaStrea
 // Heavy pass: the same engine over the level's heavy queue, 32 heavy vertices per warp batch.
 template <class App>
 inline void launch_heavy(const gcgt_graph* g, cudaStream_t s, const Ctx& c, const App& app) {
+    if (c.engine == 1) return;  // the state-machine kernel never defers
     const HeavyFront fr{c.heavyq, c.heavy_len};
     launch_expand<App, HeavyFront, false>(g->P, g->staged, g->num_sms * 8, s, c, fr, app, 32);
 }
@@ -836,7 +1089,7 @@ inline int hub_grid(const gcgt_graph* g) { return g->num_sms * 4; }
 inline Ctx make_ctx(const gcgt_graph* g) {
     return Ctx{g->W,     g->offs,     g->P.min_interval_len, 8 * g->P.residual_segment_len,
                g->hubq, g->hub_ctr, g->stats,              g->cursor,
-               g->heavyq, g->heavy_len, g->heavy_itv, g->heavy_res, g->hub_segs};
+               g->heavyq, g->heavy_len, g->heavy_itv, g->heavy_res, g->hub_segs, g->engine};
 }
 
 gcgt_status copy_out(gcgt_graph* g, void* dst, const void* src, size_t bytes, int placement) {
@@ -977,6 +1230,7 @@ extern "C" gcgt_status gcgt_load(const gcgt_cgr* c, const gcgt_load_opts* opts, 
                 const unsigned long v = strtoul(kv.c_str() + e + 1, nullptr, 10);
                 if (k == "staged") g->staged = v != 0;
                 else if (k == "persistent") g->persistent = v != 0;
+                else if (k == "engine") g->engine = (uint32_t)v;
                 else if (k == "heavy_itv") g->heavy_itv = (uint32_t)v;
                 else if (k == "heavy_res") g->heavy_res = (uint32_t)v;
                 else if (k == "hub_segs") g->hub_segs = (uint32_t)v;

@@ -27,7 +27,12 @@ for tune in tunes:
         g.bfs(r, out=out)
         t += g.last_stats["device_ms"]
         k += g.last_stats["kernel_ms"]
+    g.profile(False)
+    t2 = 0.0
+    for r in roots:
+        g.bfs(r, out=out)
+        t2 += g.last_stats["device_ms"]
     arcs = g.last_stats["arcs_decoded"]
-    print(f"{tune:50s} bfs {t / len(roots):7.3f} ms  expand {k / len(roots):7.3f} ms  "
-          f"~{arcs / (t / len(roots)) / 1e6:6.1f} GTEPS(last root arcs)", flush=True)
+    print(f"{tune:45s} bfs {t2 / len(roots):7.3f} ms (profiled {t / len(roots):7.3f})  expand {k / len(roots):7.3f} ms"
+          f"  ~{arcs / (t2 / len(roots)) / 1e6:6.1f} GTEPS", flush=True)
     g.unload()
