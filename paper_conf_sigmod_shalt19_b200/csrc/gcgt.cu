@@ -94,7 +94,7 @@ struct gcgt_graph {
     // deferring long interval areas to a separate pass costs more than the in-batch straggler it removes
     bool staged = false;
     bool persistent = false;
-    uint32_t engine = 1;  // BFS: all levels in one cooperative launch (measured slower on C2; GCGT_TUNE knob)
+    uint32_t engine = 0;  // 0 = phase kernel; 1 = state-machine kernel (measured slower on C2: lone long tasks)  // BFS: all levels in one cooperative launch (measured slower on C2; GCGT_TUNE knob)
     uint32_t heavy_itv = 0xFFFFFFFFu, heavy_res = 1024, hub_segs = 8, wpb_max = 8;
     uint32_t* heavy_len = nullptr;
     unsigned long long* hub_ctr = nullptr;
@@ -209,8 +209,26 @@ struct WinStream {
     __device__ __forceinline__ uint64_t next() { return decode<K>(W, p); }
 };
 
+// Sequential reader over BitBuf (the 32-bit refill bit buffer); same interface.
+struct BufStream {
+    const uint64_t* __restrict__ W;
+    BitBuf bb;
+    uint64_t p;  // only meaningful after sync()
+    __device__ __forceinline__ void init(const uint64_t* __restrict__ w, uint64_t pos) {
+        W = w;
+        bb.init(w, pos);
+        p = pos;
+    }
+    template <int K>
+    __device__ __forceinline__ uint64_t next() {
+        const uint64_t v = bb.template next<K>(W);
+        p = bb.pos();
+        return v;
+    }
+};
+
 template <bool STAGED>
-using Reader = typename std::conditional<STAGED, RegStream, WinStream>::type;
+using Reader = typename std::conditional<STAGED, BufStream, WinStream>::type;
 
 template <int K, bool STAGED, class T>
 __device__ __forceinline__ uint32_t decode_segment(const uint64_t* __restrict__ W, uint64_t q, uint32_t u, T& t) {

@@ -3,6 +3,6 @@ TAG=${1:-run}; KRE=${2:-expand_kernel}; SKIP=${3:-12}
 mkdir -p gpurun_out
 timeout 600 ncu --metrics gpu__time_duration.sum --clock-control none --csv --log-file gpurun_out/launches_$TAG.csv \
   python tools/prof_bfs.py --reps 1 > gpurun_out/launches_$TAG.log 2>&1
-timeout 900 ncu --set full --clock-control none --import-source on -k regex:"$KRE" -s $SKIP -c 1 \
+timeout 900 ncu --set full --clock-control none --import-source on --kernel-name-base demangled -k regex:"$KRE" -s $SKIP -c 1 \
   -o gpurun_out/prof_$TAG python tools/prof_bfs.py --reps 1 > gpurun_out/prof_$TAG.log 2>&1
 tail -3 gpurun_out/prof_$TAG.log
