@@ -77,6 +77,9 @@ typedef struct gcgt_graph gcgt_graph; /* device-resident CGR and work buffers; l
  * Errors: EINVAL (params), EUNSORTED / ERANGE (input rows), ESEGLEN (segment too short), ENOMEM. */
 gcgt_status gcgt_encode(const gcgt_csr* csr, const gcgt_params* params, gcgt_cgr** out);
 
+/* Encodes the TRANSPOSE of csr (row v = sorted in-neighbours of v), for gcgt_load_opts.in_cgr.  Same errors. */
+gcgt_status gcgt_encode_transpose(const gcgt_csr* csr, const gcgt_params* params, gcgt_cgr** out);
+
 /* Read-only view of a CGR: bytes (ceil(nbits/8), MSB-first, R1), nbits, bit_offsets (n + 1 entries, R2),
  * n, params.  Pointers stay valid until gcgt_cgr_free.  Any output pointer may be NULL. */
 gcgt_status gcgt_cgr_view(const gcgt_cgr* cgr, const uint8_t** bytes, uint64_t* nbits,
@@ -99,6 +102,10 @@ typedef struct {
     int rank, nranks;  /* 1-D vertex-range partition (multi-GPU).  nranks <= 1: single GPU (rank ignored)           */
     void* nccl_comm;   /* ncclComm_t for nranks > 1 (created by the caller, e.g. from a unique id broadcast over
                           torch.distributed); NULL for a single GPU                                                 */
+    const gcgt_cgr* in_cgr; /* CGR of the TRANSPOSE (in-arcs, e.g. from gcgt_encode_transpose) for the bottom-up
+                               BFS step; NULL = none (top-down only unless `symmetric`).  Same n and params.      */
+    int symmetric;     /* 1: every arc u->v has v->u, so the out-CGR doubles as the in-CGR (R-MAT configs)           */
+    int direction_optimizing; /* 0: top-down only; 1: switch top-down <-> bottom-up per level when an in-CGR exists */
 } gcgt_load_opts;
 
 /* Copies the CGR (bytes + bit_offsets) to the device and allocates the traversal work buffers.  With nranks > 1
@@ -120,6 +127,8 @@ gcgt_status gcgt_graph_range(const gcgt_graph* g, uint64_t* lo, uint64_t* hi);
 #define GCGT_OUT_DEVICE 1 /* output pointer is device memory on the graph's device                             */
 
 /* BFS from `source` over out-arcs (Fig. 7(b)).  levels[v] = hop distance, -1 if unreached; n entries.
+ * With an in-CGR (or `symmetric`) and direction_optimizing, large levels run bottom-up: every unvisited vertex
+ * decodes its in-record until the first frontier parent (intervals tested as frontier-bitmap ranges).
  * Errors: ERANGE (source >= n), ECUDA, ENCCL. */
 gcgt_status gcgt_bfs(gcgt_graph* g, uint32_t source, int32_t* levels, int out_placement, gcgt_stats* stats);
 

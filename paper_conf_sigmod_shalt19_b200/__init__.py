@@ -21,7 +21,7 @@ STATUS_NAMES = {0: "OK", -1: "EINVAL", -2: "EUNSORTED", -3: "ERANGE", -4: "ESEGL
 OUT_HOST, OUT_DEVICE = 0, 1
 
 # public symbols of include/gcgt.h (tests check the library exports every one)
-ABI_SYMBOLS = ["gcgt_encode", "gcgt_cgr_view", "gcgt_cgr_from_arrays", "gcgt_cgr_save", "gcgt_cgr_open",
+ABI_SYMBOLS = ["gcgt_encode", "gcgt_encode_transpose", "gcgt_cgr_view", "gcgt_cgr_from_arrays", "gcgt_cgr_save", "gcgt_cgr_open",
                "gcgt_cgr_free", "gcgt_load", "gcgt_unload", "gcgt_profile", "gcgt_graph_range", "gcgt_bfs", "gcgt_cc", "gcgt_bc",
                "gcgt_debug_warp_decode", "gcgt_last_error", "gcgt_version"]
 
@@ -51,7 +51,8 @@ class Stats(C.Structure):
 
 class LoadOpts(C.Structure):
     _fields_ = [("device", C.c_int), ("stream", C.c_void_p), ("rank", C.c_int), ("nranks", C.c_int),
-                ("nccl_comm", C.c_void_p)]
+                ("nccl_comm", C.c_void_p), ("in_cgr", C.c_void_p), ("symmetric", C.c_int),
+                ("direction_optimizing", C.c_int)]
 
 
 _lib = None
@@ -66,6 +67,7 @@ def lib():
         L = C.CDLL(LIB_PATH)
         p, u32, u64, i32 = C.c_void_p, C.c_uint32, C.c_uint64, C.c_int
         L.gcgt_encode.argtypes = [C.POINTER(Csr), C.POINTER(Params), C.POINTER(p)]
+        L.gcgt_encode_transpose.argtypes = [C.POINTER(Csr), C.POINTER(Params), C.POINTER(p)]
         L.gcgt_cgr_view.argtypes = [p, C.POINTER(p), C.POINTER(u64), C.POINTER(p), C.POINTER(u64), C.POINTER(Params)]
         L.gcgt_cgr_from_arrays.argtypes = [u64, p, u64, p, C.POINTER(Params), C.POINTER(p)]
         L.gcgt_cgr_save.argtypes = [p, C.c_char_p]
@@ -147,6 +149,20 @@ def encode(row_offsets: np.ndarray, cols: np.ndarray, min_interval_len: int = 4,
     return CGR(h)
 
 
+def encode_transpose(row_offsets: np.ndarray, cols: np.ndarray, min_interval_len: int = 4,
+                     residual_segment_len: int = 32, zeta_k: int = 3) -> CGR:
+    """CGR of the transpose (in-arcs), for Graph(..., in_cgr=...) bottom-up steps."""
+    ro = np.ascontiguousarray(row_offsets, dtype=np.uint64)
+    co = np.ascontiguousarray(cols, dtype=np.uint32)
+    if co.size == 0:
+        co = np.zeros(1, dtype=np.uint32)
+    csr = Csr(ro.size - 1, ro.ctypes.data, co.ctypes.data)
+    P = Params(min_interval_len, residual_segment_len, zeta_k)
+    h = C.c_void_p()
+    _check(lib().gcgt_encode_transpose(C.byref(csr), C.byref(P), C.byref(h)), "gcgt_encode_transpose")
+    return CGR(h)
+
+
 def from_arrays(bytes_: np.ndarray, nbits: int, bit_offsets: np.ndarray, min_interval_len: int,
                 residual_segment_len: int, zeta_k: int) -> CGR:
     b = np.ascontiguousarray(bytes_, dtype=np.uint8)
@@ -185,12 +201,15 @@ def _out(out, n, np_dtype, torch_dtype_name):
 class Graph:
     """Device-resident CGR (gcgt_load)."""
 
-    def __init__(self, cgr: CGR, device: int = 0, stream=None, rank: int = 0, nranks: int = 1, nccl_comm=None):
+    def __init__(self, cgr: CGR, device: int = 0, stream=None, rank: int = 0, nranks: int = 1, nccl_comm=None,
+                 in_cgr: "CGR | None" = None, symmetric: bool = False, direction_optimizing: bool = True):
         if stream == "torch":
             import torch
             stream = torch.cuda.current_stream(device).cuda_stream
         opts = LoadOpts(device, C.c_void_p(stream) if stream else None, rank, nranks,
-                        C.c_void_p(nccl_comm) if nccl_comm else None)
+                        C.c_void_p(nccl_comm) if nccl_comm else None, in_cgr.handle if in_cgr is not None else None,
+                        1 if symmetric else 0, 1 if direction_optimizing else 0)
+        self._in_cgr = in_cgr
         h = C.c_void_p()
         _check(lib().gcgt_load(cgr.handle, C.byref(opts), C.byref(h)), "gcgt_load")
         self._h = h

@@ -258,6 +258,35 @@ extern "C" gcgt_status gcgt_encode(const gcgt_csr* csr, const gcgt_params* param
     return GCGT_OK;
 }
 
+// Transpose on the host (parallel counting sort by target), then the same encoder.
+extern "C" gcgt_status gcgt_encode_transpose(const gcgt_csr* csr, const gcgt_params* params, gcgt_cgr** out) {
+    using gcgt_internal::fail;
+    gcgt_internal::clear_error();
+    if (!csr || !params || !out) return fail(GCGT_EINVAL, "null argument");
+    const uint64_t n = csr->n;
+    const uint64_t m = n ? csr->row_offsets[n] : 0;
+    const uint64_t* ro = csr->row_offsets;
+    const uint32_t* cols = csr->cols;
+    for (uint64_t e = 0; e < m; e++)
+        if (cols[e] >= n) return fail(GCGT_ERANGE, "column id >= n");
+    std::vector<uint64_t> tro;
+    std::vector<uint32_t> tco;
+    try {
+        tro.assign(n + 1, 0);
+        tco.resize(m);
+    } catch (...) {
+        return fail(GCGT_ENOMEM, "host allocation failed");
+    }
+    for (uint64_t e = 0; e < m; e++) tro[cols[e] + 1]++;
+    for (uint64_t v = 0; v < n; v++) tro[v + 1] += tro[v];
+    // rows are emitted in increasing source order, so every transposed row comes out sorted
+    std::vector<uint64_t> pos(tro.begin(), tro.end() - (n ? 1 : 0));
+    for (uint64_t u = 0; u < n; u++)
+        for (uint64_t e = ro[u]; e < ro[u + 1]; e++) tco[pos[cols[e]]++] = (uint32_t)u;
+    const gcgt_csr t{n, tro.data(), tco.data()};
+    return gcgt_encode(&t, params, out);
+}
+
 extern "C" gcgt_status gcgt_cgr_view(const gcgt_cgr* c, const uint8_t** bytes, uint64_t* nbits,
                                      const uint64_t** bit_offsets, uint64_t* n, gcgt_params* params) {
     gcgt_internal::clear_error();

@@ -80,6 +80,12 @@ struct gcgt_graph {
     // CGR
     uint64_t* W = nullptr;     // stream-order words (+2 pad)
     uint64_t* offs = nullptr;  // n + 1
+    uint64_t* inW = nullptr;     // in-CGR (transpose) for bottom-up; aliases W / offs when symmetric
+    uint64_t* inOffs = nullptr;
+    bool in_owned = false;       // inW / inOffs are separate allocations
+    bool dir_opt = false;        // direction-optimizing BFS enabled (in-CGR available)
+    uint32_t* bstate = nullptr;  // BFS direction state [8]: 0 dir (0 TD, 1 BU), 1 visited, 2 new-frontier count,
+                                 // 3 previous frontier count
     // work
     uint32_t *V = nullptr, *F = nullptr, *N = nullptr;
     uint32_t* q = nullptr;      // word queue storage (BFS: 2 x nw ping-pong; BC: all levels, nw + n)
@@ -94,8 +100,10 @@ struct gcgt_graph {
     // deferring long interval areas to a separate pass costs more than the in-batch straggler it removes
     bool staged = false;
     bool persistent = false;
+    bool dir_opt_knob = true;
     uint32_t engine = 0;  // 0 = phase kernel; 1 = state-machine kernel (measured slower on C2: lone long tasks)  // BFS: all levels in one cooperative launch (measured slower on C2; GCGT_TUNE knob)
     uint32_t heavy_itv = 0xFFFFFFFFu, heavy_res = 1024, hub_segs = 8, wpb_max = 8;
+    uint32_t bu_alpha = 14, bu_beta = 24;  // Beamer-style switch thresholds on vertex counts
     uint32_t* heavy_len = nullptr;
     unsigned long long* hub_ctr = nullptr;
     Stats* stats = nullptr;
@@ -140,6 +148,7 @@ struct Ctx {
     uint32_t heavy_res;           // unsegmented residual count above which a vertex is deferred
     uint32_t hub_segs;            // segment count above which a vertex's segments go to the hub queue
     uint32_t engine;              // 1 = state-machine kernel (sm_expand_kernel), 0 = phase kernel (expand_kernel)
+    const uint32_t* dir;          // BFS direction gate: top-down kernels run only while *dir == 0 (nullptr: always)
 };
 
 __device__ __forceinline__ void add_stats(Stats* st, uint64_t v, uint64_t a, uint64_t b) {
@@ -157,7 +166,7 @@ __device__ __forceinline__ void add_stats(Stats* st, uint64_t v, uint64_t a, uin
 
 // ---- frontier sources ------------------------------------------------------------------------------------------------
 // Queue of frontier words (BFS / BC): entry i is word q[i]; its bits come from qbits[i] (BC keeps them per level)
-// or from F[w], which is read and cleared (BFS).
+// or from the frontier bitmap F (BFS; the contraction rewrites F densely every level).
 struct QueueFront {
     const uint32_t* __restrict__ q;
     const uint32_t* __restrict__ qlen_p;
@@ -166,8 +175,7 @@ struct QueueFront {
     __device__ __forceinline__ uint64_t size() const { return *qlen_p; }
     __device__ __forceinline__ void get(uint64_t i, uint32_t& w, uint32_t& bits) const {
         w = q[i];
-        if (qbits) bits = qbits[i];
-        else { bits = F[w]; F[w] = 0; }
+        bits = qbits ? qbits[i] : F[w];
     }
 };
 
@@ -280,6 +288,7 @@ __device__ __forceinline__ void expand_phase(const Ctx& c, const Front& fr, cons
                                              WarpSmem* smem, uint64_t& nv, uint64_t& na, uint64_t& nb) {
     const uint32_t wid = threadIdx.x >> 5, lane = lane_id();
     WarpSmem& sm = smem[wid];
+    if (c.dir && *c.dir) return;  // this level runs bottom-up
     const uint64_t qlen = fr.size();
     if (wpb == 0) {  // sized on the device (host did not wait for the queue length): ~4 batches per resident warp
         const uint64_t b = qlen / ((uint64_t)gridDim.x * kWarps * 4);
@@ -448,7 +457,7 @@ __global__ void __launch_bounds__(kBlock, 4) sm_expand_kernel(Ctx c, Front fr, A
     __shared__ SmWarp smem[kWarps];
     const uint32_t wid = threadIdx.x >> 5, lane = lane_id(), lt = lanemask_lt();
     SmWarp& sm = smem[wid];
-    const uint64_t qlen = fr.size();
+    const uint64_t qlen = (c.dir && *c.dir) ? 0 : fr.size();
     if (wpb == 0) {
         const uint64_t b = qlen / ((uint64_t)gridDim.x * kWarps * 4);
         wpb = b < 1 ? 1 : (b > 8 ? 8 : (uint32_t)b);
@@ -696,7 +705,7 @@ struct BfsApp {
     int32_t level;
     __device__ __forceinline__ void begin(uint32_t) {}
     __device__ __forceinline__ void end() {}
-    __device__ __forceinline__ void vertex(uint32_t u) { levels[u] = level; }
+    __device__ __forceinline__ void vertex(uint32_t) {}  // levels are written when a vertex is discovered
     __device__ __forceinline__ void claim(uint32_t w, uint32_t mask) {
         const uint32_t cand = mask & ~__ldg(V + w);
         if (cand) atomicOr(N + w, cand);
@@ -850,10 +859,12 @@ __global__ void cc_init(uint32_t* parent, uint64_t n) {
 __device__ __forceinline__ void commit_phase(uint32_t* __restrict__ V, uint32_t* __restrict__ F,
                                              uint32_t* __restrict__ N, uint64_t w_lo, uint64_t w_hi,
                                              uint32_t* __restrict__ qn, uint32_t* __restrict__ qn_len,
-                                             uint32_t* __restrict__ qbits_out) {
+                                             uint32_t* __restrict__ qbits_out, int32_t* __restrict__ levels = nullptr,
+                                             int32_t new_level = 0, uint32_t* __restrict__ nf_count = nullptr) {
     const uint32_t lane = lane_id();
     const uint64_t gw = ((uint64_t)blockIdx.x * blockDim.x + threadIdx.x) >> 5;
     const uint64_t nwarps = ((uint64_t)gridDim.x * blockDim.x) >> 5;
+    uint32_t nf = 0;
     for (uint64_t base = w_lo + gw * 32; base < w_hi; base += nwarps * 32) {
         const uint64_t w = base + lane;
         uint32_t b = 0;
@@ -862,9 +873,10 @@ __device__ __forceinline__ void commit_phase(uint32_t* __restrict__ V, uint32_t*
             if (b) {
                 N[w] = 0;
                 V[w] |= b;
-                if (F) F[w] = b;
             }
+            if (F && F[w] != b) F[w] = b;  // F = exactly the new frontier
         }
+        nf += __popc(b);
         const uint32_t bal = __ballot_sync(0xffffffffu, b != 0);
         if (bal) {
             uint32_t pos = 0;
@@ -874,20 +886,133 @@ __device__ __forceinline__ void commit_phase(uint32_t* __restrict__ V, uint32_t*
                 qn[pos] = (uint32_t)w;
                 if (qbits_out) qbits_out[pos] = b;
             }
+            if (levels) {  // one coalesced 32-id store per new frontier word
+                for (uint32_t m = bal; m; m &= m - 1) {
+                    const int j = __ffs(m) - 1;
+                    const uint32_t bj = __shfl_sync(0xffffffffu, b, j);
+                    if ((bj >> lane) & 1u) levels[(base + j) * 32 + lane] = new_level;
+                }
+            }
         }
+    }
+    if (nf_count) {
+        for (int o = 16; o; o >>= 1) nf += __shfl_xor_sync(0xffffffffu, nf, o);
+        if (lane == 0 && nf) atomicAdd(nf_count, nf);
     }
 }
 
 __global__ void commit_dense(uint32_t* __restrict__ V, uint32_t* __restrict__ F, uint32_t* __restrict__ N,
                              uint64_t w_lo, uint64_t w_hi, uint32_t* __restrict__ qn, uint32_t* __restrict__ qn_len,
                              uint32_t* __restrict__ qbits_out, uint32_t* __restrict__ reset_ctr,
-                             unsigned long long* __restrict__ hub_ctr, uint32_t* __restrict__ heavy_len) {
-    commit_phase(V, F, N, w_lo, w_hi, qn, qn_len, qbits_out);
+                             unsigned long long* __restrict__ hub_ctr, uint32_t* __restrict__ heavy_len,
+                             int32_t* __restrict__ levels = nullptr, int32_t new_level = 0,
+                             uint32_t* __restrict__ nf_count = nullptr) {
+    commit_phase(V, F, N, w_lo, w_hi, qn, qn_len, qbits_out, levels, new_level, nf_count);
     if (blockIdx.x == 0 && threadIdx.x == 0) {
         if (reset_ctr) *reset_ctr = 0;
         if (hub_ctr) *hub_ctr = 0;
         if (heavy_len) *heavy_len = 0;
     }
+}
+
+// Direction choice for the next BFS level (one thread; Beamer et al.'s heuristic on vertex counts): switch to
+// bottom-up when the new frontier is large against the unvisited set and growing, back to top-down when it is
+// small against n and shrinking.  st: [0] dir, [1] visited, [2] new-frontier count (consumed), [3] previous.
+__global__ void bfs_decide(uint32_t* st, uint64_t n, uint32_t alpha, uint32_t beta, int enabled) {
+    const uint64_t nf = st[2];
+    st[2] = 0;
+    const uint64_t visited = (uint64_t)st[1] + nf;
+    st[1] = (uint32_t)visited;
+    const uint64_t nu = n - visited, prev = st[3];
+    uint32_t dir = st[0];
+    if (!enabled || nf == 0) dir = 0;
+    else if (dir == 0 && nf * alpha > nu && nf > prev) dir = 1;
+    else if (dir == 1 && nf * beta < n && nf < prev) dir = 0;
+    st[0] = dir;
+    st[3] = (uint32_t)nf;
+}
+
+// ---- bottom-up step (north_star addition; §8 a9) -----------------------------------------------------------------
+// For every unvisited vertex v, decode v's IN-record until the first parent in the frontier F: intervals are tested
+// as bitmap ranges (F & word mask), residuals as single bits; decoding stops at the first hit.  A warp owns one
+// 32-vertex word, so the found mask is written to N without atomics.
+__device__ __forceinline__ bool frontier_range(const uint32_t* __restrict__ F, uint32_t s, uint32_t len) {
+    const uint32_t e = s + len;
+    while (s < e) {
+        const uint32_t b0 = s & 31, nb = min(32u - b0, e - s);
+        if (__ldg(F + (s >> 5)) & ((nb == 32 ? 0xffffffffu : ((1u << nb) - 1)) << b0)) return true;
+        s += nb;
+    }
+    return false;
+}
+
+template <int K, bool SEG>
+__global__ void __launch_bounds__(kBlock) bu_kernel(const uint64_t* __restrict__ W, const uint64_t* __restrict__ offs,
+                                                    uint32_t min_len, uint32_t seg_bits, const uint32_t* __restrict__ V,
+                                                    const uint32_t* __restrict__ F, uint32_t* __restrict__ N,
+                                                    uint64_t n, uint64_t nw, const uint32_t* __restrict__ dir,
+                                                    Stats* st) {
+    if (*dir != 1) return;
+    const uint32_t lane = lane_id();
+    uint64_t nv = 0, na = 0, nb = 0;
+    for (uint64_t w = ((uint64_t)blockIdx.x * blockDim.x + threadIdx.x) >> 5; w < nw;
+         w += ((uint64_t)gridDim.x * blockDim.x) >> 5) {
+        const uint64_t v0 = w * 32;
+        if (v0 >= n) break;
+        uint32_t unv = ~__ldg(V + w);
+        if (n - v0 < 32) unv &= (1u << (n - v0)) - 1;
+        if (!unv) continue;
+        bool found = false;
+        if ((unv >> lane) & 1u) {
+            const uint32_t v = (uint32_t)(v0 + lane);
+            const uint64_t p0 = ldg64(offs + v);
+            uint64_t p = p0;
+            nv++;
+            uint64_t deg = 0, got = 0;
+            if (!SEG) deg = decode<K>(W, p) - 1;
+            const uint64_t itv = decode<K>(W, p) - 1;
+            int64_t prev_end = 0;
+            for (uint64_t i = 0; i < itv && !found; i++) {
+                const uint64_t g = decode<K>(W, p);
+                const uint64_t len = decode<K>(W, p) - 1 + min_len;
+                const int64_t start = i == 0 ? unmap_first(v, g) : prev_end + (int64_t)g;
+                found = frontier_range(F, (uint32_t)start, (uint32_t)len);
+                prev_end = start + (int64_t)len - 1;
+                got += len;
+            }
+            if (!found) {
+                if (!SEG) {
+                    const uint64_t nres = deg - got;
+                    int64_t cur = 0;
+                    for (uint64_t i = 0; i < nres && !found; i++) {
+                        const uint64_t c = decode<K>(W, p);
+                        cur = i == 0 ? unmap_first(v, c) : cur + (int64_t)c;
+                        found = (__ldg(F + (cur >> 5)) >> (cur & 31)) & 1u;
+                        got++;
+                    }
+                } else {
+                    const uint64_t nseg = decode<K>(W, p) - 1;
+                    const uint64_t base = p;
+                    for (uint64_t sg = 0; sg < nseg && !found; sg++) {
+                        p = base + sg * seg_bits;
+                        const uint64_t cnt = decode<K>(W, p) - 1;
+                        int64_t cur = 0;
+                        for (uint64_t i = 0; i < cnt && !found; i++) {
+                            const uint64_t c = decode<K>(W, p);
+                            cur = i == 0 ? unmap_first(v, c) : cur + (int64_t)c;
+                            found = (__ldg(F + (cur >> 5)) >> (cur & 31)) & 1u;
+                            got++;
+                        }
+                    }
+                }
+            }
+            na += got;
+            nb += p - p0;
+        }
+        const uint32_t fb = __ballot_sync(0xffffffffu, found);
+        if (lane == 0 && fb) N[w] = fb;
+    }
+    add_stats(st, nv, na, nb);
 }
 
 // ---- persistent BFS: every level inside one cooperative launch ------------------------------------------------------
@@ -928,7 +1053,7 @@ __global__ void __launch_bounds__(kBlock, 4) bfs_persistent(Ctx c, BfsPersist b)
             hub_phase<K, false>(c, app, na);
             grid.sync();
         }
-        commit_phase(b.V, b.F, b.N, 0, b.nw, qn, b.ctr + nxt, nullptr);
+        commit_phase(b.V, b.F, b.N, 0, b.nw, qn, b.ctr + nxt, nullptr, b.levels, (int32_t)level + 1);
         if (blockIdx.x == 0 && threadIdx.x == 0) {
             b.ctr[cur] = 0;
             *c.hub_ctr = 0;
@@ -946,8 +1071,16 @@ __global__ void count_level(const uint32_t* qn_len, uint32_t* counter) {
     if (*qn_len) *counter += 1;
 }
 
-__global__ void bfs_seed(uint32_t s, uint32_t* V, uint32_t* F, uint32_t* q, uint32_t* qlen, uint32_t* qbits) {
+__global__ void bfs_seed(uint32_t s, uint32_t* V, uint32_t* F, uint32_t* q, uint32_t* qlen, uint32_t* qbits,
+                         int32_t* levels = nullptr, uint32_t* bstate = nullptr) {
     V[s >> 5] = 1u << (s & 31);
+    if (levels) levels[s] = 0;
+    if (bstate) {
+        bstate[0] = 0;
+        bstate[1] = 1;
+        bstate[2] = 0;
+        bstate[3] = 1;
+    }
     if (F) F[s >> 5] = 1u << (s & 31);
     q[0] = s >> 5;
     if (qbits) qbits[0] = 1u << (s & 31);
@@ -1071,6 +1204,30 @@ inline cudaError_t launch_bfs_persistent(const gcgt_graph* g, cudaStream_t s, Ct
     }
 }
 
+template <int K, bool SEG>
+inline void launch_bu_k(const gcgt_graph* g, cudaStream_t s) {
+    static int per_sm = 0;
+    if (!per_sm) {
+        cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per_sm, bu_kernel<K, SEG>, kBlock, 0);
+        if (per_sm < 1) per_sm = 1;
+    }
+    const int grid = (int)std::max<uint64_t>(1, std::min<uint64_t>((g->nw + kWarps - 1) / kWarps,
+                                                                    (uint64_t)per_sm * g->num_sms));
+    bu_kernel<K, SEG><<<grid, kBlock, 0, s>>>(g->inW, g->inOffs, g->P.min_interval_len, 8 * g->P.residual_segment_len,
+                                              g->V, g->F, g->N, g->n, g->nw, g->bstate, g->stats);
+}
+
+inline void launch_bu(const gcgt_graph* g, cudaStream_t s) {
+    const bool seg = g->P.residual_segment_len != 0;
+    switch (g->P.zeta_k) {
+        case 1: seg ? launch_bu_k<1, true>(g, s) : launch_bu_k<1, false>(g, s); break;
+        case 2: seg ? launch_bu_k<2, true>(g, s) : launch_bu_k<2, false>(g, s); break;
+        case 3: seg ? launch_bu_k<3, true>(g, s) : launch_bu_k<3, false>(g, s); break;
+        case 4: seg ? launch_bu_k<4, true>(g, s) : launch_bu_k<4, false>(g, s); break;
+        default: seg ? launch_bu_k<5, true>(g, s) : launch_bu_k<5, false>(g, s); break;
+    }
+}
+
 template <class App>
 inline void launch_hub(const gcgt_params& P, bool staged, int grid, cudaStream_t s, const Ctx& c, const App& app) {
     if (!P.residual_segment_len) return;
@@ -1107,7 +1264,7 @@ inline int hub_grid(const gcgt_graph* g) { return g->num_sms * 4; }
 inline Ctx make_ctx(const gcgt_graph* g) {
     return Ctx{g->W,     g->offs,     g->P.min_interval_len, 8 * g->P.residual_segment_len,
                g->hubq, g->hub_ctr, g->stats,              g->cursor,
-               g->heavyq, g->heavy_len, g->heavy_itv, g->heavy_res, g->hub_segs, g->engine};
+               g->heavyq, g->heavy_len, g->heavy_itv, g->heavy_res, g->hub_segs, g->engine, nullptr};
 }
 
 gcgt_status copy_out(gcgt_graph* g, void* dst, const void* src, size_t bytes, int placement) {
@@ -1191,7 +1348,8 @@ extern "C" void gcgt_unload(gcgt_graph* g) {
     cudaSetDevice(g->device);
     void* bufs[] = {g->W,      g->offs,    g->V,      g->F,         g->N,        g->q,      g->qbits,
                     g->ctr,    g->hubq,    g->hub_ctr, g->cursor,   g->heavyq,   g->heavy_len, g->stats,
-                    g->levels, g->parent,  g->sigma,  g->delta,     g->bc};
+                    g->levels, g->parent,  g->sigma,  g->delta,     g->bc,      g->bstate,
+                    g->in_owned ? g->inW : nullptr, g->in_owned ? g->inOffs : nullptr};
     if (g->stream) {
         for (void* b : bufs)
             if (b) cudaFreeAsync(b, g->stream);
@@ -1249,6 +1407,9 @@ extern "C" gcgt_status gcgt_load(const gcgt_cgr* c, const gcgt_load_opts* opts, 
                 if (k == "staged") g->staged = v != 0;
                 else if (k == "persistent") g->persistent = v != 0;
                 else if (k == "engine") g->engine = (uint32_t)v;
+                else if (k == "bu_alpha") g->bu_alpha = (uint32_t)v;
+                else if (k == "bu_beta") g->bu_beta = (uint32_t)v;
+                else if (k == "dir_opt") g->dir_opt_knob = v != 0;
                 else if (k == "heavy_itv") g->heavy_itv = (uint32_t)v;
                 else if (k == "heavy_res") g->heavy_res = (uint32_t)v;
                 else if (k == "hub_segs") g->hub_segs = (uint32_t)v;
@@ -1279,6 +1440,27 @@ extern "C" gcgt_status gcgt_load(const gcgt_cgr* c, const gcgt_load_opts* opts, 
                        g->stream));
     bswap_words<<<flat_grid(g.get(), nwords), kBlock, 0, g->stream>>>(g->W, nwords);
     CU(cudaMemsetAsync(g->N, 0, g->nw * 4, g->stream));
+    if ((st = galloc(g.get(), &g->bstate, 8))) return st;
+    // in-CGR for bottom-up levels: the transpose if given, else the out-CGR itself on symmetric graphs
+    if (o.in_cgr) {
+        const gcgt_cgr* ic = o.in_cgr;
+        if (ic->n != c->n || ic->params.zeta_k != c->params.zeta_k ||
+            ic->params.min_interval_len != c->params.min_interval_len ||
+            ic->params.residual_segment_len != c->params.residual_segment_len)
+            return fail(GCGT_EINVAL, "in_cgr must have the same n and parameters as the CGR");
+        const uint64_t inwords = (ic->nbits + 63) / 64 + 2;
+        if ((st = galloc(g.get(), &g->inW, inwords)) || (st = galloc(g.get(), &g->inOffs, ic->n + 1))) return st;
+        g->in_owned = true;
+        CU(cudaMemcpyAsync(g->inW, ic->words.data(), inwords * 8, cudaMemcpyHostToDevice, g->stream));
+        CU(cudaMemcpyAsync(g->inOffs, ic->bit_offsets.data(), (ic->n + 1) * 8, cudaMemcpyHostToDevice, g->stream));
+        bswap_words<<<flat_grid(g.get(), inwords), kBlock, 0, g->stream>>>(g->inW, inwords);
+        g->dir_opt = o.direction_optimizing != 0;
+    } else if (o.symmetric) {
+        g->inW = g->W;
+        g->inOffs = g->offs;
+        g->dir_opt = o.direction_optimizing != 0;
+    }
+    g->dir_opt = g->dir_opt && g->dir_opt_knob;
     if ((st = galloc(g.get(), &g->hub_ctr, 1)) || (st = galloc(g.get(), &g->cursor, 2))) return st;
     CU(cudaMemsetAsync(g->cursor, 0, 16, g->stream));
     unsigned long long* dcount = nullptr;
@@ -1400,8 +1582,9 @@ extern "C" gcgt_status gcgt_bfs(gcgt_graph* g, uint32_t source, int32_t* levels,
     CU(cudaMemsetAsync(g->hub_ctr, 0, sizeof(unsigned long long), s));
     CU(cudaMemsetAsync(g->heavy_len, 0, 4, s));
     uint32_t* q[2] = {g->q, g->q + g->nw};
-    bfs_seed<<<1, 1, 0, s>>>(source, g->V, g->F, q[0], g->ctr + 0, nullptr);
-    const Ctx c = make_ctx(g);
+    bfs_seed<<<1, 1, 0, s>>>(source, g->V, g->F, q[0], g->ctr + 0, nullptr, g->levels, g->bstate);
+    Ctx c = make_ctx(g);
+    if (g->dir_opt) c.dir = g->bstate;
     uint64_t qlen = 1;
     uint32_t level = 0;
     if (g->persistent) {
@@ -1441,8 +1624,11 @@ extern "C" gcgt_status gcgt_bfs(gcgt_graph* g, uint32_t source, int32_t* levels,
             if ((st = kprof_end(g))) return st;
             launch_heavy(g, s, c, app);
             launch_hub(g->P, g->staged, hub_grid(g), s, c, app);
+            if (g->dir_opt) launch_bu(g, s);
             commit_dense<<<flat_grid(g, g->nw), kBlock, 0, s>>>(g->V, g->F, g->N, 0, g->nw, q[nxt], g->ctr + nxt,
-                                                                 nullptr, g->ctr + cur, g->hub_ctr, g->heavy_len);
+                                                                 nullptr, g->ctr + cur, g->hub_ctr, g->heavy_len,
+                                                                 g->levels, (int32_t)level + 1, g->bstate + 2);
+            bfs_decide<<<1, 1, 0, s>>>(g->bstate, g->n, g->bu_alpha, g->bu_beta, g->dir_opt ? 1 : 0);
             count_level<<<1, 1, 0, s>>>(g->ctr + nxt, g->ctr + 6);
         }
         CU(cudaMemcpyAsync(g->h_ctr + 6, g->ctr + 6, 4, cudaMemcpyDeviceToHost, s));

@@ -118,3 +118,20 @@ def test_load_without_gpu_fails_loudly():
     with pytest.raises(G.GcgtError) as e:
         G.load(G.encode(ro, co))
     assert e.value.status == G.ECUDA
+
+
+def _transpose(ro, co):
+    n = ro.size - 1
+    src = np.repeat(np.arange(n, dtype=np.int64), np.diff(ro.astype(np.int64)))
+    from graphs import csr_from_edges
+    return csr_from_edges(n, co.astype(np.int64), src)
+
+
+@pytest.mark.parametrize("ml,sl,k", [(4, 32, 3), (0, 0, 1), (2, 8, 2)])
+def test_encode_transpose_bit_exact(ml, sl, k):
+    """gcgt_encode_transpose(G) == oracle encode of the transposed CSR (in-arcs, rows sorted)."""
+    ro, co = random_graph(800, 9000, seed=k + sl)
+    tro, tco = _transpose(ro, co)
+    ob, onb, ooffs = O.encode(tro, tco, ml, sl, k)
+    b, nb, offs, n, _ = G.encode_transpose(ro, co, ml, sl, k).view()
+    assert nb == onb and np.array_equal(offs, ooffs) and np.array_equal(b, ob)

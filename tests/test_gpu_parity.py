@@ -194,3 +194,35 @@ def test_warp_decoder_random_streams(k):
         b, nb = O.bits_to_bytes(bits)
         vals, _, _, _ = G.debug_warp_decode(b, nb, k, 32, len(xs))
         assert [int(v) for v in vals] == xs, (k, trial)
+
+
+# ---------------------------------------------------------------------------------------------------------------------
+# Direction-optimizing BFS (bottom-up levels over the in-CGR, §8 a9)
+# ---------------------------------------------------------------------------------------------------------------------
+@pytest.mark.parametrize("tune", ["", "bu_alpha=100000,bu_beta=1", "bu_alpha=100000,bu_beta=100000"])
+@pytest.mark.parametrize("name", ["c1", "rmat_s", "web_s", "social_s"])
+def test_bfs_direction_optimizing(name, tune, monkeypatch):
+    """Symmetric graphs use the out-CGR as in-CGR; directed ones the encoded transpose.  The tunes force
+    bottom-up early (and keep it), or switch back and forth, so every level kind is exercised."""
+    monkeypatch.setenv("GCGT_TUNE", tune)
+    cfg = synth.CONFIGS[name]
+    ro, co = cfg.make()
+    p = (cfg.min_interval_len, cfg.residual_segment_len, cfg.zeta_k)
+    cgr = G.encode(ro, co, *p)
+    if cfg.symmetric:
+        g = G.load(cgr, symmetric=True)
+    else:
+        g = G.load(cgr, in_cgr=G.encode_transpose(ro, co, *p))
+    for r in [0] + synth.pick_roots(ro, 3):
+        assert np.array_equal(g.bfs(r), O.bfs(ro, co, r)), (name, tune, r)
+
+
+@pytest.mark.parametrize("ml,sl,k", [(4, 32, 3), (0, 0, 1), (2, 8, 5)])
+def test_bfs_bottom_up_random(ml, sl, k, monkeypatch):
+    monkeypatch.setenv("GCGT_TUNE", "bu_alpha=100000,bu_beta=1")
+    for seed, sym in [(1, True), (2, False), (3, False)]:
+        ro, co = random_graph(6000, 60000, seed=seed + k, symmetric=sym)
+        cgr = G.encode(ro, co, ml, sl, k)
+        g = G.load(cgr, symmetric=True) if sym else G.load(cgr, in_cgr=G.encode_transpose(ro, co, ml, sl, k))
+        for s in (0, 17, 5999):
+            assert np.array_equal(g.bfs(s), O.bfs(ro, co, s)), (seed, s)
