@@ -110,6 +110,10 @@ CONFIGS = {
     "social_s": Config("social_s", "social", (100_000, 35.3, 20_000, 2010), False, 4, 32, 3,
                        "social recipe, 100K vertices"),
     "rmat_s": Config("rmat_s", "rmat", (16, 16, 16), True, 4, 32, 3, "R-MAT s16 ef16"),
+    # mid-size variants for performance sweeps
+    "rmat_m": Config("rmat_m", "rmat", (22, 16, 22), True, 4, 32, 3, "R-MAT s22 ef16"),
+    "social_m": Config("social_m", "social", (4_000_000, 35.3, 300_000, 2010), False, 4, 32, 3,
+                       "social recipe, 4M vertices"),
 }
 
 

@@ -12,12 +12,14 @@ import synth  # noqa: E402
 cfg = synth.CONFIGS[sys.argv[1]]
 tunes = sys.argv[2:]
 ro, co = cfg.make()
-cgr = G.encode(ro, co, cfg.min_interval_len, cfg.residual_segment_len, cfg.zeta_k)
+P = (cfg.min_interval_len, cfg.residual_segment_len, cfg.zeta_k)
+cgr = G.encode(ro, co, *P)
+incgr = None if cfg.symmetric else G.encode_transpose(ro, co, *P)
 roots = synth.pick_roots(ro, 8)
 out = torch.empty(ro.size - 1, dtype=torch.int32, device="cuda")
 for tune in tunes:
     os.environ["GCGT_TUNE"] = tune
-    g = G.load(cgr, stream="torch")
+    g = G.load(cgr, stream="torch", in_cgr=incgr, symmetric=cfg.symmetric)
     for r in roots[:2]:
         g.bfs(r, out=out)
     g.profile(True)
