@@ -183,18 +183,26 @@ def main():
     dev = torch.device("cuda", local)
 
     ro, co, tgen = make_graph(cfg)
+    P = (cfg.min_interval_len, cfg.residual_segment_len, cfg.zeta_k)
     t0 = time.time()
-    cgr = G.encode(ro, co, cfg.min_interval_len, cfg.residual_segment_len, cfg.zeta_k)
+    cgr = G.encode(ro, co, *P)
     tenc = time.time() - t0
+    # bottom-up levels need in-arcs: the transpose's CGR on directed graphs, the CGR itself on symmetric ones
+    incgr = None if cfg.symmetric else G.encode_transpose(ro, co, *P)
     _, nbits, _, n, _ = cgr.view()
-    g = G.load(cgr, device=local, stream="torch")
+    g = G.load(cgr, device=local, stream="torch", in_cgr=incgr, symmetric=cfg.symmetric)
     stream = torch.cuda.current_stream(dev)
     roots_all = choose_roots(ro, args.roots * max(ws, 1))
     roots = roots_all[rank::max(ws, 1)]
     levels = torch.empty(n, dtype=torch.int32, device=dev)
-    # L2 flush buffer (> 126 MB L2), written between timed steps, outside the per-step events
+    # L2 flush buffer (> 126 MB L2), written between timed steps, outside the per-step CUDA events
     flush = torch.empty(256 << 20, dtype=torch.uint8, device=dev)
-
+    # TEPS numerator per root: sum of out-degrees of the reached vertices, from the input CSR
+    deg = torch.from_numpy(np.diff(ro.astype(np.int64))).to(dev)
+    edges_of_root = {}
+    for r in sorted(set(roots)):
+        g.bfs(r, out=levels)
+        edges_of_root[r] = edges_of(cfg, int(deg[levels >= 0].sum().item()))
     for i in range(args.warmup):
         g.bfs(roots[i % len(roots)], out=levels)
     torch.cuda.synchronize()
@@ -202,17 +210,20 @@ def main():
     g.profile(True)
     evs = [(torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)) for _ in range(args.steps)]
     clocks = ClockSampler(torch.cuda.current_device() if "CUDA_VISIBLE_DEVICES" not in os.environ else local)
-    tot = {"arcs": 0, "bits": 0, "vertices": 0, "levels": 0, "kms": 0.0, "klaunch": 0}
+    tot = {"arcs": 0, "bits": 0, "vertices": 0, "levels": 0, "kms": 0.0, "klaunch": 0, "launches": 0, "edges": 0.0}
     if ws > 1:
         dist.barrier()
     torch.cuda.synchronize()
     clocks.start()
     for i in range(args.steps):
         flush.fill_(i & 0xFF)
+        r = roots[(args.warmup + i) % len(roots)]
         evs[i][0].record(stream)
-        g.bfs(roots[(args.warmup + i) % len(roots)], out=levels)
+        g.bfs(r, out=levels)
         evs[i][1].record(stream)
+        tot["edges"] += edges_of_root[r]
         st = g.last_stats
+        tot["launches"] += st["launches"]
         tot["arcs"] += st["arcs_decoded"]
         tot["bits"] += st["cgr_bits_decoded"]
         tot["vertices"] += st["vertices_expanded"]
@@ -225,7 +236,7 @@ def main():
     ck = clocks.stop()
     g.profile(False)
     t_ms = sum(a.elapsed_time(b) for a, b in evs)
-    edges = edges_of(cfg, tot["arcs"])
+    edges = tot["edges"]
     if ws > 1:
         tt = torch.tensor([t_ms], dtype=torch.float64, device=dev)
         dist.all_reduce(tt, op=dist.ReduceOp.MAX)
@@ -236,18 +247,18 @@ def main():
         edges_all = edges
     value = edges_all / (t_ms * 1e-3) / 1e9
 
-    # roofline of the dominant kernel (bfs_expand): algorithmic bytes per launch =
-    # CGR bytes of the expanded records + 8 B bit offset + 4 B level write per expanded vertex
+    # roofline of the dominant kernel span (each level's expansion: top-down kernel + hub segments, or the bottom-up
+    # kernel): algorithmic bytes = CGR bytes decoded + 8 B bit offset + 4 B level write per vertex
+    # expanded (top-down) or examined (bottom-up)
     peak, peak_src = hbm_peak()
     alg_bytes = tot["bits"] / 8 + 12 * tot["vertices"]
     k_s = tot["kms"] * 1e-3
     achieved = alg_bytes / k_s / 1e9 if k_s > 0 else 0.0
     cgr_gbs = tot["bits"] / 8 / k_s / 1e9 if k_s > 0 else 0.0
-    launches_per_step = 2 * tot["levels"] / args.steps + 1  # expand + commit per level, + seed
 
     e2e = None
     if not args.no_e2e:
-        e2e = measure_e2e(G, cgr, roots, cfg, n, nbits, dev, local, steps=min(args.steps, 3))
+        e2e = measure_e2e(G, cgr, incgr, roots, edges_of_root, cfg, n, nbits, dev, local, steps=min(args.steps, 3))
 
     cpu = None
     if rank == 0 and ws == 1 and not args.no_cpu_baseline:
@@ -261,16 +272,17 @@ def main():
                            "bits_per_arc": nbits / max(1, int(ro[-1])), "cgr_mb": nbits / 8e6,
                            "min_interval_len": cfg.min_interval_len, "residual_segment_len": cfg.residual_segment_len,
                            "zeta_k": cfg.zeta_k, "roots_per_rank": len(roots), "levels_per_bfs": tot["levels"] / args.steps,
+                           "direction_optimizing": True, "in_cgr": "transpose" if incgr is not None else "symmetric",
                            "edges_per_bfs": edges / args.steps,
                            "l2": "flushed between steps (256 MiB fill, outside the per-step CUDA events)",
                            "parallelism": f"{ws} x independent BFS queries (replicas)" if ws > 1 else "1 GPU",
                            "gen_s": round(tgen, 1), "encode_s": round(tenc, 1)},
                 "roofline": {"bound": "hbm", "achieved": achieved, "peak": peak, "unit": "GB/s",
-                             "frac": achieved / peak, "traffic": None, "kernel": "bfs_expand",
+                             "frac": achieved / peak, "traffic": None, "kernel": "level expansion (expand_kernel+hub_kernel | bu_kernel)",
                              "peak_source": peak_src, "cgr_only_gbs": cgr_gbs, "cgr_only_frac": cgr_gbs / peak,
                              "kernel_share_of_step": tot["kms"] / t_ms if t_ms else None,
                              "launches": tot["klaunch"]},
-                "cpu_baseline": cpu, "e2e": e2e, "gpu_launches": int(round(launches_per_step * args.steps)),
+                "cpu_baseline": cpu, "e2e": e2e, "gpu_launches": int(tot["launches"]),
                 "clocks": ck}
         print(json.dumps(line), flush=True)
     g.unload()
@@ -278,7 +290,7 @@ def main():
         dist.destroy_process_group()
 
 
-def measure_e2e(G, cgr, roots, cfg, n, nbits, dev, local, steps=3):
+def measure_e2e(G, cgr, incgr, roots, edges_of_root, cfg, n, nbits, dev, local, steps=3):
     """Same metric through the public API with HOST buffers: per step gcgt_load (H2D of the CGR bytes and bit
     offsets from pinned host memory) + gcgt_bfs into a pinned host levels array (D2H) + gcgt_unload."""
     import torch
@@ -291,6 +303,14 @@ def measure_e2e(G, cgr, roots, cfg, n, nbits, dev, local, steps=3):
     L.gcgt_cgr_view(cgr.handle, C.byref(bp), None, C.byref(op), None, None)
     nbytes_words = ((nbits + 63) // 64 + 2) * 8
     reg = [(bp.value, nbytes_words), (op.value, (n + 1) * 8)]
+    h2d = nbytes_words + (n + 1) * 8
+    if incgr is not None:
+        ib, io = C.c_void_p(), C.c_void_p()
+        inb = C.c_uint64()
+        L.gcgt_cgr_view(incgr.handle, C.byref(ib), C.byref(inb), C.byref(io), None, None)
+        inwords = ((inb.value + 63) // 64 + 2) * 8
+        reg += [(ib.value, inwords), (io.value, (n + 1) * 8)]
+        h2d += inwords + (n + 1) * 8
     for ptr, size in reg:
         cudart.cudaHostRegister(ptr, size, 0)
     levels = torch.empty(n, dtype=torch.int32).pin_memory()
@@ -299,19 +319,19 @@ def measure_e2e(G, cgr, roots, cfg, n, nbits, dev, local, steps=3):
         for i in range(steps):
             torch.cuda.synchronize()
             t0 = time.perf_counter()
-            g = G.load(cgr, device=local, stream="torch")
-            g.bfs(roots[i % len(roots)], out=levels)
-            arcs = g.last_stats["arcs_decoded"]
+            g = G.load(cgr, device=local, stream="torch", in_cgr=incgr, symmetric=cfg.symmetric)
+            r = roots[i % len(roots)]
+            g.bfs(r, out=levels)
             g.unload()
             torch.cuda.synchronize()
             tot_t += time.perf_counter() - t0
-            tot_e += edges_of(cfg, arcs)
+            tot_e += edges_of_root[r]
     finally:
         for ptr, _ in reg:
             cudart.cudaHostUnregister(ptr)
-    return {"value": tot_e / tot_t / 1e9, "unit": "GTEPS", "h2d_bytes_per_step": int(nbytes_words + (n + 1) * 8),
+    return {"value": tot_e / tot_t / 1e9, "unit": "GTEPS", "h2d_bytes_per_step": int(h2d),
             "d2h_bytes_per_step": int(4 * n),
-            "note": "per step: gcgt_load (CGR + bit offsets H2D from pinned host memory, device allocation) + "
+            "note": "per step: gcgt_load (CGR + in-CGR + bit offsets H2D from pinned host memory, pool allocation) + "
                     "gcgt_bfs with a pinned host levels array + gcgt_unload; host wall clock"}
 
 

@@ -67,6 +67,7 @@ typedef struct {
     double kernel_ms;           /* with gcgt_profile(g, 1): summed CUDA-event time of the call's dominant kernel
                                    (BFS/BC: frontier expansion; CC: hooking), else 0                              */
     uint64_t kernel_launches;   /* launches of that kernel in the call (0 unless profiling)                      */
+    uint64_t launches;          /* all library kernel launches of the call                                       */
 } gcgt_stats;
 
 typedef struct gcgt_cgr gcgt_cgr;     /* host CGR: canonical bytes + bit_offsets + params; library-owned     */

@@ -43,7 +43,7 @@ class Csr(C.Structure):
 class Stats(C.Structure):
     _fields_ = [("iterations", C.c_uint32), ("reserved", C.c_uint32), ("vertices_expanded", C.c_uint64),
                 ("arcs_decoded", C.c_uint64), ("cgr_bits_decoded", C.c_uint64), ("device_ms", C.c_double),
-                ("kernel_ms", C.c_double), ("kernel_launches", C.c_uint64)]
+                ("kernel_ms", C.c_double), ("kernel_launches", C.c_uint64), ("launches", C.c_uint64)]
 
     def as_dict(self):
         return {k: getattr(self, k) for k, _ in self._fields_ if k != "reserved"}

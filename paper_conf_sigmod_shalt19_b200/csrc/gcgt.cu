@@ -103,7 +103,7 @@ struct gcgt_graph {
     bool dir_opt_knob = true;
     uint32_t engine = 0;  // 0 = phase kernel; 1 = state-machine kernel (measured slower on C2: lone long tasks)  // BFS: all levels in one cooperative launch (measured slower on C2; GCGT_TUNE knob)
     uint32_t heavy_itv = 0xFFFFFFFFu, heavy_res = 1024, hub_segs = 8, wpb_max = 8;
-    uint32_t bu_alpha = 14, bu_beta = 24;  // Beamer-style switch thresholds on vertex counts
+    uint32_t bu_alpha = 4, bu_beta = 24;  // switch thresholds on vertex counts (C2/R-MAT/social sweep, r1)
     uint32_t* heavy_len = nullptr;
     unsigned long long* hub_ctr = nullptr;
     Stats* stats = nullptr;
@@ -119,6 +119,7 @@ struct gcgt_graph {
     cudaEvent_t kev0 = nullptr, kev1 = nullptr;
     double kernel_ms = 0;
     uint64_t kernel_launches = 0;
+    uint64_t launches = 0;  // kernels launched by the current call (gcgt_stats.launches)
 };
 
 namespace {
@@ -1169,9 +1170,14 @@ inline void launch_expand(const gcgt_params& P, bool staged, int grid, cudaStrea
 }
 
 // Heavy pass: the same engine over the level's heavy queue, 32 heavy vertices per warp batch.
+inline bool heavy_active(const gcgt_graph* g) {  // can any vertex be deferred to the heavy pass?
+    if (g->engine == 1) return false;                  // the state-machine kernel never defers
+    return g->heavy_itv != 0xFFFFFFFFu || (g->P.residual_segment_len == 0 && g->heavy_res != 0xFFFFFFFFu);
+}
+
 template <class App>
 inline void launch_heavy(const gcgt_graph* g, cudaStream_t s, const Ctx& c, const App& app) {
-    if (c.engine == 1) return;  // the state-machine kernel never defers
+    if (!heavy_active(g)) return;
     const HeavyFront fr{c.heavyq, c.heavy_len};
     launch_expand<App, HeavyFront, false>(g->P, g->staged, g->num_sms * 8, s, c, fr, app, 32);
 }
@@ -1296,6 +1302,7 @@ gcgt_status begin_call(gcgt_graph* g) {
     CU(cudaSetDevice(g->device));
     g->kernel_ms = 0;
     g->kernel_launches = 0;
+    g->launches = 0;
     CU(cudaMemsetAsync(g->stats, 0, sizeof(Stats), g->stream));
     CU(cudaEventRecord(g->ev0, g->stream));
     return GCGT_OK;
@@ -1317,6 +1324,7 @@ gcgt_status end_call(gcgt_graph* g, gcgt_stats* out, uint32_t iterations) {
         out->device_ms = ms;
         out->kernel_ms = g->kernel_ms;
         out->kernel_launches = g->kernel_launches;
+        out->launches = g->launches;
     }
     return GCGT_OK;
 }
@@ -1583,6 +1591,7 @@ extern "C" gcgt_status gcgt_bfs(gcgt_graph* g, uint32_t source, int32_t* levels,
     CU(cudaMemsetAsync(g->heavy_len, 0, 4, s));
     uint32_t* q[2] = {g->q, g->q + g->nw};
     bfs_seed<<<1, 1, 0, s>>>(source, g->V, g->F, q[0], g->ctr + 0, nullptr, g->levels, g->bstate);
+    g->launches = 1;
     Ctx c = make_ctx(g);
     if (g->dir_opt) c.dir = g->bstate;
     uint64_t qlen = 1;
@@ -1592,6 +1601,7 @@ extern "C" gcgt_status gcgt_bfs(gcgt_graph* g, uint32_t source, int32_t* levels,
         if ((st = kprof_begin(g))) return st;
         const cudaError_t e = launch_bfs_persistent(g, s, c, b);
         if (e == cudaSuccess) {
+            g->launches += 1;
             if ((st = kprof_end(g))) return st;
             CU(cudaMemcpyAsync(g->h_ctr + 6, g->ctr + 6, 4, cudaMemcpyDeviceToHost, s));
             CU(cudaStreamSynchronize(s));
@@ -1619,17 +1629,19 @@ extern "C" gcgt_status gcgt_bfs(gcgt_graph* g, uint32_t source, int32_t* levels,
             else wpb = 0;  // device-side sizing
             const QueueFront fr{q[cur], g->ctr + cur, g->F, nullptr};
             const BfsApp app{g->V, g->N, g->levels, (int32_t)level};
+            // profiled span = the level's expansion: top-down kernel (+ heavy pass + hub segments) or bottom-up
             if ((st = kprof_begin(g))) return st;
             launch_expand(g->P, g->staged, grid, s, c, fr, app, wpb);
-            if ((st = kprof_end(g))) return st;
             launch_heavy(g, s, c, app);
             launch_hub(g->P, g->staged, hub_grid(g), s, c, app);
             if (g->dir_opt) launch_bu(g, s);
+            if ((st = kprof_end(g))) return st;
             commit_dense<<<flat_grid(g, g->nw), kBlock, 0, s>>>(g->V, g->F, g->N, 0, g->nw, q[nxt], g->ctr + nxt,
                                                                  nullptr, g->ctr + cur, g->hub_ctr, g->heavy_len,
                                                                  g->levels, (int32_t)level + 1, g->bstate + 2);
             bfs_decide<<<1, 1, 0, s>>>(g->bstate, g->n, g->bu_alpha, g->bu_beta, g->dir_opt ? 1 : 0);
             count_level<<<1, 1, 0, s>>>(g->ctr + nxt, g->ctr + 6);
+            g->launches += 4 + (g->P.residual_segment_len ? 1 : 0) + (g->dir_opt ? 1 : 0) + (heavy_active(g) ? 1 : 0);
         }
         CU(cudaMemcpyAsync(g->h_ctr + 6, g->ctr + 6, 4, cudaMemcpyDeviceToHost, s));
         CU(cudaMemcpyAsync(g->h_ctr + (level & 1), g->ctr + (level & 1), 4, cudaMemcpyDeviceToHost, s));
