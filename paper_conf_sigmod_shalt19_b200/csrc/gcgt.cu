@@ -13,6 +13,7 @@
 // backward delta (Fig. 7(d), Brandes [9]).
 #include <cuda_runtime.h>
 #include <cooperative_groups.h>
+#include <cub/cub.cuh>
 #include <stdio.h>
 #include <string.h>
 
@@ -63,6 +64,16 @@ struct HubEntry {
     uint32_t seg_off;  // first flattened segment index of this entry (entries are ordered by seg_off)
 };
 
+// An interval chunk of a vertex with a long interval area: `count` intervals starting with the gap code at bit
+// `pos`, the previous interval having ended at `prev_end` (load-time checkpoint table, see build_checkpoints).
+struct ChunkEntry {
+    uint64_t pos;
+    uint32_t u;
+    uint32_t prev_end;
+    uint32_t count;
+    uint32_t pad;
+};
+
 struct HeavyEntry {
     uint64_t p;    // first bit after the itvNum field
     uint32_t u;
@@ -84,6 +95,11 @@ struct gcgt_graph {
     uint64_t* inOffs = nullptr;
     bool in_owned = false;       // inW / inOffs are separate allocations
     bool dir_opt = false;        // direction-optimizing BFS enabled (in-CGR available)
+    // interval checkpoint table (derived at load) + per-level chunk queue
+    uint32_t hv_n = 0, ck_c = 16;
+    uint32_t *hv_ids = nullptr, *hv_ptr = nullptr, *hv_rem = nullptr, *ck_prev = nullptr, *chunk_len = nullptr;
+    uint64_t *hv_after = nullptr, *ck_pos = nullptr;
+    ChunkEntry* chunkq = nullptr;
     uint32_t* bstate = nullptr;  // BFS direction state [8]: 0 dir (0 TD, 1 BU), 1 visited, 2 new-frontier count,
                                  // 3 previous frontier count
     // work
@@ -150,6 +166,16 @@ struct Ctx {
     uint32_t hub_segs;            // segment count above which a vertex's segments go to the hub queue
     uint32_t engine;              // 1 = state-machine kernel (sm_expand_kernel), 0 = phase kernel (expand_kernel)
     const uint32_t* dir;          // BFS direction gate: top-down kernels run only while *dir == 0 (nullptr: always)
+    // interval checkpoints (vertices with more than ck_c intervals; sorted ids, per-vertex checkpoint ranges)
+    uint32_t hv_n, ck_c;
+    const uint32_t* __restrict__ hv_ids;
+    const uint32_t* __restrict__ hv_ptr;
+    const uint64_t* __restrict__ hv_after;  // bit after the interval area
+    const uint32_t* __restrict__ hv_rem;    // unsegmented records: residual count
+    const uint64_t* __restrict__ ck_pos;
+    const uint32_t* __restrict__ ck_prev;
+    ChunkEntry* chunkq;
+    uint32_t* chunk_len;
 };
 
 __device__ __forceinline__ void add_stats(Stats* st, uint64_t v, uint64_t a, uint64_t b) {
@@ -348,8 +374,29 @@ __device__ __forceinline__ void expand_phase(const Ctx& c, const Front& fr, cons
                     c.heavyq[slot] = HeavyEntry{p, u, (uint32_t)itv, deg};
                 } else {
                     int64_t prev_end = 0;
-                    uint64_t in_itv = 0;
-                    for (uint64_t i = 0; i < itv; i++) {
+                    uint64_t in_itv = 0, nres_ck = 0;
+                    uint64_t itv_here = itv;
+                    bool ck = false;
+                    uint64_t after = 0;
+                    if (c.hv_n && itv > c.ck_c) {  // long interval area: chunks beyond the first go grid-wide
+                        uint32_t lo = 0, hi = c.hv_n - 1;
+                        while (lo < hi) {
+                            const uint32_t mid = (lo + hi) >> 1;
+                            if (c.hv_ids[mid] < u) lo = mid + 1; else hi = mid;
+                        }
+                        const uint32_t b0 = c.hv_ptr[lo], b1 = c.hv_ptr[lo + 1];
+                        const uint32_t slot = atomicAdd(c.chunk_len, b1 - b0);
+                        for (uint32_t k = b0; k < b1; k++) {
+                            const uint64_t first = (uint64_t)(k - b0 + 1) * c.ck_c;
+                            c.chunkq[slot + k - b0] = ChunkEntry{c.ck_pos[k], u, c.ck_prev[k],
+                                                                 (uint32_t)(itv - first < c.ck_c ? itv - first : c.ck_c), 0};
+                        }
+                        itv_here = c.ck_c;
+                        after = c.hv_after[lo];
+                        if (!SEG) nres_ck = c.hv_rem[lo];
+                        ck = true;
+                    }
+                    for (uint64_t i = 0; i < itv_here; i++) {
                         const uint64_t g = rs.template next<K>();
                         const uint64_t len = rs.template next<K>() - 1 + c.min_len;
                         const int64_t start = i == 0 ? unmap_first(u, g) : prev_end + (int64_t)g;
@@ -358,8 +405,9 @@ __device__ __forceinline__ void expand_phase(const Ctx& c, const Front& fr, cons
                         in_itv += len;
                     }
                     na += in_itv;
+                    if (ck) rs.init(c.W, after);
                     if (!SEG) {
-                        const uint64_t nres = deg - in_itv;
+                        const uint64_t nres = ck ? nres_ck : deg - in_itv;
                         int64_t cur = 0;
                         for (uint64_t i = 0; i < nres; i++) {
                             const uint64_t cd = rs.template next<K>();
@@ -672,6 +720,26 @@ __global__ void __launch_bounds__(kBlock, 4) sm_expand_kernel(Ctx c, Front fr, A
 // Hub segments of the level, flattened over the whole grid (one segment per thread at a time).
 template <int K, bool STAGED, class App>
 __device__ __forceinline__ void hub_phase(const Ctx& c, const App& app, uint64_t& na) {
+    if (c.chunk_len) {  // interval chunks of long interval areas: one chunk per thread
+        const uint32_t nck = *(volatile uint32_t*)c.chunk_len;
+        for (uint64_t j = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; j < nck;
+             j += (uint64_t)gridDim.x * blockDim.x) {
+            const ChunkEntry e = c.chunkq[j];
+            App t = app;
+            t.begin(e.u);
+            uint64_t p = e.pos;
+            uint32_t cur = e.prev_end;
+            for (uint32_t i = 0; i < e.count; i++) {
+                const uint32_t g = (uint32_t)decode<K>(c.W, p);
+                const uint32_t len = (uint32_t)(decode<K>(c.W, p) - 1) + c.min_len;
+                const uint32_t start = cur + g;
+                t.range(start, len);
+                cur = start + len - 1;
+                na += len;
+            }
+            t.end();
+        }
+    }
     const unsigned long long hc = *(volatile unsigned long long*)c.hub_ctr;
     const uint32_t nh = (uint32_t)(hc >> 32), S = (uint32_t)(hc & 0xffffffffu);
     for (uint64_t j = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; j < S; j += (uint64_t)gridDim.x * blockDim.x) {
@@ -907,12 +975,13 @@ __global__ void commit_dense(uint32_t* __restrict__ V, uint32_t* __restrict__ F,
                              uint32_t* __restrict__ qbits_out, uint32_t* __restrict__ reset_ctr,
                              unsigned long long* __restrict__ hub_ctr, uint32_t* __restrict__ heavy_len,
                              int32_t* __restrict__ levels = nullptr, int32_t new_level = 0,
-                             uint32_t* __restrict__ nf_count = nullptr) {
+                             uint32_t* __restrict__ nf_count = nullptr, uint32_t* __restrict__ chunk_len = nullptr) {
     commit_phase(V, F, N, w_lo, w_hi, qn, qn_len, qbits_out, levels, new_level, nf_count);
     if (blockIdx.x == 0 && threadIdx.x == 0) {
         if (reset_ctr) *reset_ctr = 0;
         if (hub_ctr) *hub_ctr = 0;
         if (heavy_len) *heavy_len = 0;
+        if (chunk_len) *chunk_len = 0;
     }
 }
 
@@ -1050,7 +1119,7 @@ __global__ void __launch_bounds__(kBlock, 4) bfs_persistent(Ctx c, BfsPersist b)
         const BfsApp app{b.V, b.N, b.levels, (int32_t)level};
         expand_phase<K, SEG, BfsApp, QueueFront, true, false>(c, fr, app, (uint32_t)wpb, smem, nv, na, nb);
         grid.sync();
-        if (SEG) {
+        if (SEG || c.hv_n) {
             hub_phase<K, false>(c, app, na);
             grid.sync();
         }
@@ -1058,6 +1127,7 @@ __global__ void __launch_bounds__(kBlock, 4) bfs_persistent(Ctx c, BfsPersist b)
         if (blockIdx.x == 0 && threadIdx.x == 0) {
             b.ctr[cur] = 0;
             *c.hub_ctr = 0;
+            if (c.chunk_len) *c.chunk_len = 0;
             c.cursor[0] = 0;
         }
         grid.sync();
@@ -1091,6 +1161,58 @@ __global__ void bfs_seed(uint32_t s, uint32_t* V, uint32_t* F, uint32_t* q, uint
 __global__ void bswap_words(uint64_t* w, uint64_t n) {
     for (uint64_t i = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; i < n; i += (uint64_t)gridDim.x * blockDim.x)
         w[i] = __byte_perm((uint32_t)(w[i] >> 32), 0, 0x0123) | ((uint64_t)__byte_perm((uint32_t)w[i], 0, 0x0123) << 32);
+}
+
+// ---- load-time interval checkpoint table ---------------------------------------------------------------------------
+// Vertices with more than C intervals get a checkpoint every C intervals: the bit position of the gap code of
+// interval kC and the end of interval kC-1.  Each chunk of C intervals then decodes on its own, so a long interval
+// area no longer forms one serial chain (the residual-segment idea of §5.2 applied to intervals, as a derived
+// device table; the CGR bytes are unchanged).
+template <int K, bool SEG>
+__global__ void ck_count(const uint64_t* __restrict__ W, const uint64_t* __restrict__ offs, uint64_t n, uint32_t C,
+                         uint8_t* __restrict__ flag, uint32_t* __restrict__ cnt) {
+    for (uint64_t u = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; u < n; u += (uint64_t)gridDim.x * blockDim.x) {
+        uint64_t p = ldg64(offs + u);
+        if (!SEG) decode<K>(W, p);
+        const uint64_t itv = decode<K>(W, p) - 1;
+        const bool h = itv > C;
+        flag[u] = h;
+        cnt[u] = h ? (uint32_t)((itv - 1) / C) : 0;
+    }
+}
+
+__global__ void ck_gather(const uint32_t* __restrict__ ids, const uint32_t* __restrict__ cnt, uint32_t H,
+                          uint32_t* __restrict__ out) {
+    for (uint64_t h = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; h <= H; h += (uint64_t)gridDim.x * blockDim.x)
+        out[h] = h < H ? cnt[ids[h]] : 0;
+}
+
+template <int K, bool SEG>
+__global__ void ck_fill(const uint64_t* __restrict__ W, const uint64_t* __restrict__ offs, uint32_t min_len,
+                        uint32_t C, const uint32_t* __restrict__ ids, const uint32_t* __restrict__ ptr, uint32_t H,
+                        uint64_t* __restrict__ ck_pos, uint32_t* __restrict__ ck_prev, uint64_t* __restrict__ after,
+                        uint32_t* __restrict__ rem) {
+    for (uint64_t h = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; h < H; h += (uint64_t)gridDim.x * blockDim.x) {
+        const uint32_t u = ids[h];
+        uint64_t p = ldg64(offs + u), deg = 0, sum = 0;
+        if (!SEG) deg = decode<K>(W, p) - 1;
+        const uint64_t itv = decode<K>(W, p) - 1;
+        int64_t prev_end = 0;
+        for (uint64_t i = 0; i < itv; i++) {
+            if (i && i % C == 0) {
+                const uint32_t k = ptr[h] + (uint32_t)(i / C) - 1;
+                ck_pos[k] = p;
+                ck_prev[k] = (uint32_t)prev_end;
+            }
+            const uint64_t g = decode<K>(W, p);
+            const uint64_t len = decode<K>(W, p) - 1 + min_len;
+            const int64_t start = i == 0 ? unmap_first(u, g) : prev_end + (int64_t)g;
+            prev_end = start + (int64_t)len - 1;
+            sum += len;
+        }
+        after[h] = p;
+        rem[h] = SEG ? 0 : (uint32_t)(deg - sum);
+    }
 }
 
 // Load-time pass: number of hub vertices (more than kHubSegs residual segments) and heavy vertices (long
@@ -1236,7 +1358,7 @@ inline void launch_bu(const gcgt_graph* g, cudaStream_t s) {
 
 template <class App>
 inline void launch_hub(const gcgt_params& P, bool staged, int grid, cudaStream_t s, const Ctx& c, const App& app) {
-    if (!P.residual_segment_len) return;
+    if (!P.residual_segment_len && !c.hv_n) return;
 #define GCGT_HUB(KK)                                                            \
     (staged ? hub_kernel<KK, true, App><<<grid, kBlock, 0, s>>>(c, app)         \
             : hub_kernel<KK, false, App><<<grid, kBlock, 0, s>>>(c, app))
@@ -1270,7 +1392,9 @@ inline int hub_grid(const gcgt_graph* g) { return g->num_sms * 4; }
 inline Ctx make_ctx(const gcgt_graph* g) {
     return Ctx{g->W,     g->offs,     g->P.min_interval_len, 8 * g->P.residual_segment_len,
                g->hubq, g->hub_ctr, g->stats,              g->cursor,
-               g->heavyq, g->heavy_len, g->heavy_itv, g->heavy_res, g->hub_segs, g->engine, nullptr};
+               g->heavyq, g->heavy_len, g->heavy_itv, g->heavy_res, g->hub_segs, g->engine, nullptr,
+               g->hv_n,  g->ck_c,      g->hv_ids,    g->hv_ptr,    g->hv_after, g->hv_rem, g->ck_pos, g->ck_prev,
+               g->chunkq, g->chunk_len};
 }
 
 gcgt_status copy_out(gcgt_graph* g, void* dst, const void* src, size_t bytes, int placement) {
@@ -1348,6 +1472,83 @@ gcgt_status galloc(const gcgt_graph* g, T** p, uint64_t count) {
 
 }  // namespace
 
+// Builds the interval checkpoint table (see ck_count / ck_fill) and the per-level chunk queue.
+gcgt_status build_checkpoints(gcgt_graph* g) {
+    gcgt_status st;
+    if ((st = galloc(g, &g->chunk_len, 1))) return st;
+    CU(cudaMemsetAsync(g->chunk_len, 0, 4, g->stream));
+    if (g->ck_c == 0xFFFFFFFFu || g->n == 0) return GCGT_OK;
+    cudaStream_t s = g->stream;
+    const bool seg = g->P.residual_segment_len != 0;
+    const uint32_t C = g->ck_c;
+    uint8_t* flag = nullptr;
+    uint32_t *cnt = nullptr, *ids = nullptr, *nsel = nullptr;
+    if ((st = galloc(g, &flag, g->n)) || (st = galloc(g, &cnt, g->n + 1)) || (st = galloc(g, &ids, g->n + 1)) ||
+        (st = galloc(g, &nsel, 1)))
+        return st;
+    const int gr = flat_grid(g, g->n);
+#define GCGT_CK(KK) (seg ? ck_count<KK, true><<<gr, kBlock, 0, s>>>(g->W, g->offs, g->n, C, flag, cnt)   \
+                         : ck_count<KK, false><<<gr, kBlock, 0, s>>>(g->W, g->offs, g->n, C, flag, cnt))
+    switch (g->P.zeta_k) {
+        case 1: GCGT_CK(1); break;
+        case 2: GCGT_CK(2); break;
+        case 3: GCGT_CK(3); break;
+        case 4: GCGT_CK(4); break;
+        default: GCGT_CK(5); break;
+    }
+#undef GCGT_CK
+    size_t tmp_bytes = 0;
+    cub::CountingInputIterator<uint32_t> iota(0);
+    CU(cub::DeviceSelect::Flagged(nullptr, tmp_bytes, iota, flag, ids, nsel, (int64_t)g->n, s));
+    void* tmp = nullptr;
+    size_t tmp2 = 0;
+    CU(cub::DeviceScan::ExclusiveSum(nullptr, tmp2, cnt, cnt, (int64_t)g->n + 1, s));
+    if ((st = galloc(g, (uint8_t**)&tmp, std::max(tmp_bytes, tmp2)))) return st;
+    CU(cub::DeviceSelect::Flagged(tmp, tmp_bytes, iota, flag, ids, nsel, (int64_t)g->n, s));
+    uint32_t H = 0;
+    CU(cudaMemcpyAsync(&H, nsel, 4, cudaMemcpyDeviceToHost, s));
+    CU(cudaStreamSynchronize(s));
+    if (H) {
+        if ((st = galloc(g, &g->hv_ids, H)) || (st = galloc(g, &g->hv_ptr, H + 1)) ||
+            (st = galloc(g, &g->hv_after, H)) || (st = galloc(g, &g->hv_rem, H)))
+            return st;
+        CU(cudaMemcpyAsync(g->hv_ids, ids, (uint64_t)H * 4, cudaMemcpyDeviceToDevice, s));
+        ck_gather<<<flat_grid(g, H + 1), kBlock, 0, s>>>(g->hv_ids, cnt, H, ids);
+        // ids now holds the per-heavy-vertex counts (+ a trailing 0); scan into hv_ptr
+        tmp2 = std::max(tmp_bytes, tmp2);
+        CU(cub::DeviceScan::ExclusiveSum(tmp, tmp2, ids, g->hv_ptr, (int64_t)H + 1, s));
+        uint32_t T = 0;
+        CU(cudaMemcpyAsync(&T, g->hv_ptr + H, 4, cudaMemcpyDeviceToHost, s));
+        CU(cudaStreamSynchronize(s));
+        if ((st = galloc(g, &g->ck_pos, (uint64_t)T + 1)) || (st = galloc(g, &g->ck_prev, (uint64_t)T + 1)) ||
+            (st = galloc(g, &g->chunkq, (uint64_t)T + 1)))
+            return st;
+        const int gh = flat_grid(g, H);
+#define GCGT_CF(KK)                                                                                                  \
+    (seg ? ck_fill<KK, true><<<gh, kBlock, 0, s>>>(g->W, g->offs, g->P.min_interval_len, C, g->hv_ids, g->hv_ptr, H, \
+                                                   g->ck_pos, g->ck_prev, g->hv_after, g->hv_rem)                      \
+         : ck_fill<KK, false><<<gh, kBlock, 0, s>>>(g->W, g->offs, g->P.min_interval_len, C, g->hv_ids, g->hv_ptr,  \
+                                                    H, g->ck_pos, g->ck_prev, g->hv_after, g->hv_rem))
+        switch (g->P.zeta_k) {
+            case 1: GCGT_CF(1); break;
+            case 2: GCGT_CF(2); break;
+            case 3: GCGT_CF(3); break;
+            case 4: GCGT_CF(4); break;
+            default: GCGT_CF(5); break;
+        }
+#undef GCGT_CF
+        g->hv_n = H;
+    }
+    cudaFreeAsync(flag, s);
+    cudaFreeAsync(cnt, s);
+    cudaFreeAsync(ids, s);
+    cudaFreeAsync(nsel, s);
+    cudaFreeAsync(tmp, s);
+    CU(cudaStreamSynchronize(s));
+    CU(cudaGetLastError());
+    return GCGT_OK;
+}
+
 // ------------------------------------------------------------------------------------------------------------------
 // C ABI
 // ------------------------------------------------------------------------------------------------------------------
@@ -1357,6 +1558,7 @@ extern "C" void gcgt_unload(gcgt_graph* g) {
     void* bufs[] = {g->W,      g->offs,    g->V,      g->F,         g->N,        g->q,      g->qbits,
                     g->ctr,    g->hubq,    g->hub_ctr, g->cursor,   g->heavyq,   g->heavy_len, g->stats,
                     g->levels, g->parent,  g->sigma,  g->delta,     g->bc,      g->bstate,
+                    g->hv_ids, g->hv_ptr,  g->hv_rem, g->ck_prev,   g->chunk_len, g->hv_after, g->ck_pos, g->chunkq,
                     g->in_owned ? g->inW : nullptr, g->in_owned ? g->inOffs : nullptr};
     if (g->stream) {
         for (void* b : bufs)
@@ -1418,6 +1620,7 @@ extern "C" gcgt_status gcgt_load(const gcgt_cgr* c, const gcgt_load_opts* opts, 
                 else if (k == "bu_alpha") g->bu_alpha = (uint32_t)v;
                 else if (k == "bu_beta") g->bu_beta = (uint32_t)v;
                 else if (k == "dir_opt") g->dir_opt_knob = v != 0;
+                else if (k == "ck_c") g->ck_c = (uint32_t)std::max(1ul, v);  // 0xFFFFFFFF disables checkpoints
                 else if (k == "heavy_itv") g->heavy_itv = (uint32_t)v;
                 else if (k == "heavy_res") g->heavy_res = (uint32_t)v;
                 else if (k == "hub_segs") g->hub_segs = (uint32_t)v;
@@ -1494,6 +1697,7 @@ extern "C" gcgt_status gcgt_load(const gcgt_cgr* c, const gcgt_load_opts* opts, 
     if ((st = galloc(g.get(), &g->heavyq, nheavy + 1)) || (st = galloc(g.get(), &g->heavy_len, 1))) return st;
     CU(cudaMemsetAsync(g->heavy_len, 0, 4, g->stream));
     if ((st = galloc(g.get(), &g->hubq, nhubs + nheavy + 1))) return st;
+    if ((st = build_checkpoints(g.get()))) return st;
     CU(cudaMemsetAsync(g->hub_ctr, 0, 8, g->stream));
     CU(cudaStreamSynchronize(g->stream));
     CU(cudaGetLastError());
@@ -1589,6 +1793,7 @@ extern "C" gcgt_status gcgt_bfs(gcgt_graph* g, uint32_t source, int32_t* levels,
     CU(cudaMemsetAsync(g->ctr, 0, 8 * 4, s));
     CU(cudaMemsetAsync(g->hub_ctr, 0, sizeof(unsigned long long), s));
     CU(cudaMemsetAsync(g->heavy_len, 0, 4, s));
+    CU(cudaMemsetAsync(g->chunk_len, 0, 4, s));
     uint32_t* q[2] = {g->q, g->q + g->nw};
     bfs_seed<<<1, 1, 0, s>>>(source, g->V, g->F, q[0], g->ctr + 0, nullptr, g->levels, g->bstate);
     g->launches = 1;
@@ -1638,7 +1843,8 @@ extern "C" gcgt_status gcgt_bfs(gcgt_graph* g, uint32_t source, int32_t* levels,
             if ((st = kprof_end(g))) return st;
             commit_dense<<<flat_grid(g, g->nw), kBlock, 0, s>>>(g->V, g->F, g->N, 0, g->nw, q[nxt], g->ctr + nxt,
                                                                  nullptr, g->ctr + cur, g->hub_ctr, g->heavy_len,
-                                                                 g->levels, (int32_t)level + 1, g->bstate + 2);
+                                                                 g->levels, (int32_t)level + 1, g->bstate + 2,
+                                                                 g->chunk_len);
             bfs_decide<<<1, 1, 0, s>>>(g->bstate, g->n, g->bu_alpha, g->bu_beta, g->dir_opt ? 1 : 0);
             count_level<<<1, 1, 0, s>>>(g->ctr + nxt, g->ctr + 6);
             g->launches += 4 + (g->P.residual_segment_len ? 1 : 0) + (g->dir_opt ? 1 : 0) + (heavy_active(g) ? 1 : 0);
@@ -1662,6 +1868,7 @@ extern "C" gcgt_status gcgt_cc(gcgt_graph* g, uint32_t* labels, int placement, g
     cudaStream_t s = g->stream;
     CU(cudaMemsetAsync(g->hub_ctr, 0, sizeof(unsigned long long), s));
     CU(cudaMemsetAsync(g->heavy_len, 0, 4, s));
+    CU(cudaMemsetAsync(g->chunk_len, 0, 4, s));
     cc_init<<<flat_grid(g, g->n), kBlock, 0, s>>>(g->parent, g->n);
     const Ctx c = make_ctx(g);
     const DenseFront fr{g->lo, g->hi};
@@ -1703,6 +1910,7 @@ extern "C" gcgt_status gcgt_bc(gcgt_graph* g, const uint32_t* sources, uint32_t 
     CU(cudaMemsetAsync(g->bc, 0, g->n * 8, s));
     CU(cudaMemsetAsync(g->hub_ctr, 0, sizeof(unsigned long long), s));
     CU(cudaMemsetAsync(g->heavy_len, 0, 4, s));
+    CU(cudaMemsetAsync(g->chunk_len, 0, 4, s));
     std::vector<uint32_t> lvl_off;
     for (uint32_t si = 0; si < k; si++) {
         const uint32_t src = sources[si];
@@ -1735,7 +1943,7 @@ extern "C" gcgt_status gcgt_bc(gcgt_graph* g, const uint32_t* sources, uint32_t 
             commit_dense<<<flat_grid(g, g->nw), kBlock, 0, s>>>(g->V, nullptr, g->N, 0, g->nw, g->q + total,
                                                                  g->ctr + 2 + ((level + 1) & 1), g->qbits + total,
                                                                  g->ctr + 2 + (level & 1), g->hub_ctr,
-                                                                 g->heavy_len);
+                                                                 g->heavy_len, nullptr, 0, nullptr, g->chunk_len);
             CU(cudaMemcpyAsync(g->h_ctr + 1, g->ctr + 2 + ((level + 1) & 1), 4, cudaMemcpyDeviceToHost, s));
             CU(cudaStreamSynchronize(s));
             if ((st = kprof_collect(g))) return st;
@@ -1756,6 +1964,7 @@ extern "C" gcgt_status gcgt_bc(gcgt_graph* g, const uint32_t* sources, uint32_t 
             launch_hub(g->P, g->staged, hub_grid(g), s, c, app);
             CU(cudaMemsetAsync(g->hub_ctr, 0, sizeof(unsigned long long), s));
             CU(cudaMemsetAsync(g->heavy_len, 0, 4, s));
+            CU(cudaMemsetAsync(g->chunk_len, 0, 4, s));
         }
     }
     if ((st = copy_out(g, bc, g->bc, g->n * 8, placement))) return st;
