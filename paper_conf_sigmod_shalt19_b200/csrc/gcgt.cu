@@ -96,7 +96,7 @@ struct gcgt_graph {
     bool in_owned = false;       // inW / inOffs are separate allocations
     bool dir_opt = false;        // direction-optimizing BFS enabled (in-CGR available)
     // interval checkpoint table (derived at load) + per-level chunk queue
-    uint32_t hv_n = 0, ck_c = 16;
+    uint32_t hv_n = 0, ck_c = 8;
     uint32_t *hv_ids = nullptr, *hv_ptr = nullptr, *hv_rem = nullptr, *ck_prev = nullptr, *chunk_len = nullptr;
     uint64_t *hv_after = nullptr, *ck_pos = nullptr;
     ChunkEntry* chunkq = nullptr;
