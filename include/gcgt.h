@@ -143,6 +143,32 @@ gcgt_status gcgt_cc(gcgt_graph* g, uint32_t* labels, int out_placement, gcgt_sta
 gcgt_status gcgt_bc(gcgt_graph* g, const uint32_t* sources, uint32_t k, double* bc, int out_placement,
                     gcgt_stats* stats);
 
+/* ---- Partitioned multi-GPU steps (§8 e; driver: paper_conf_sigmod_shalt19_b200/dist.py) -----------------------
+ * A graph loaded with nranks > 1 holds only its owned vertex range [lo, hi) (gcgt_graph_range; boundaries on
+ * 32-vertex words, balanced by CGR bits).  The caller runs the collectives between the steps (e.g. NCCL through
+ * torch.distributed).  Every bitmap crossing this boundary is a DEVICE array of ceil(n/32) uint32 words (bit v%32
+ * of word v/32); an owned slice is words [lo/32, ceil(hi/32)).  gcgt_bfs / gcgt_cc / gcgt_bc refuse partitioned
+ * graphs.  BFS level d:
+ *   gcgt_dist_bfs_expand  : decode the owned frontier's records, claim unvisited targets into `cand` (full bitmap,
+ *                           zeroed by the call)                                           [expansion + filter]
+ *   (caller) all-to-all   : slice q of every rank's cand goes to rank q
+ *   gcgt_dist_bfs_commit  : recv = nparts owned-size slices; fslice = OR(recv) & ~visited; levels of the new owned
+ *                           vertices = d + 1; *new_count = popcount(fslice) (host)       [contraction]
+ *   (caller) all-gather   : the owned fslices form the global next frontier
+ *   gcgt_dist_bfs_absorb  : frontier := gathered bitmap; visited |= frontier
+ * and the search ends when the all-reduced new_count is 0.  gcgt_dist_bfs_levels copies the owned levels out.
+ * CC: parent is a caller-owned device array of n uint32 replicated on every rank; per round
+ *   gcgt_dist_cc_hook (hook the owned vertices' arcs; *hooks = successful hooks), all-reduce(MIN) of parent,
+ *   gcgt_dist_cc_jump (pointer jumping); stop when the all-reduced hook count is 0. */
+gcgt_status gcgt_dist_bfs_begin(gcgt_graph* g, uint32_t source);
+gcgt_status gcgt_dist_bfs_expand(gcgt_graph* g, uint32_t level, uint32_t* cand);
+gcgt_status gcgt_dist_bfs_commit(gcgt_graph* g, uint32_t level, const uint32_t* recv, uint32_t nparts,
+                                 uint32_t* fslice, uint64_t* new_count);
+gcgt_status gcgt_dist_bfs_absorb(gcgt_graph* g, const uint32_t* frontier);
+gcgt_status gcgt_dist_bfs_levels(gcgt_graph* g, int32_t* levels_owned, int out_placement);
+gcgt_status gcgt_dist_cc_hook(gcgt_graph* g, uint32_t* parent, uint64_t* hooks);
+gcgt_status gcgt_dist_cc_jump(gcgt_graph* g, uint32_t* parent);
+
 /* ---- Test hook (parity pin of the warp decoder against Fig. 5 / Ex. 5.1) ------------------
  * Runs the device warp-parallel decoder (Alg. 4 :901-919) on one warp over a caller bit array (host, MSB-first
  * bytes, R1): vals[0..count-1] receive the first `count` codewords decoded from bit 0; the FIRST window step over

@@ -23,6 +23,8 @@ OUT_HOST, OUT_DEVICE = 0, 1
 # public symbols of include/gcgt.h (tests check the library exports every one)
 ABI_SYMBOLS = ["gcgt_encode", "gcgt_encode_transpose", "gcgt_cgr_view", "gcgt_cgr_from_arrays", "gcgt_cgr_save", "gcgt_cgr_open",
                "gcgt_cgr_free", "gcgt_load", "gcgt_unload", "gcgt_profile", "gcgt_graph_range", "gcgt_bfs", "gcgt_cc", "gcgt_bc",
+               "gcgt_dist_bfs_begin", "gcgt_dist_bfs_expand", "gcgt_dist_bfs_commit", "gcgt_dist_bfs_absorb",
+               "gcgt_dist_bfs_levels", "gcgt_dist_cc_hook", "gcgt_dist_cc_jump",
                "gcgt_debug_warp_decode", "gcgt_last_error", "gcgt_version"]
 
 
@@ -82,6 +84,13 @@ def lib():
         L.gcgt_bfs.argtypes = [p, u32, p, i32, C.POINTER(Stats)]
         L.gcgt_cc.argtypes = [p, p, i32, C.POINTER(Stats)]
         L.gcgt_bc.argtypes = [p, p, u32, p, i32, C.POINTER(Stats)]
+        L.gcgt_dist_bfs_begin.argtypes = [p, u32]
+        L.gcgt_dist_bfs_expand.argtypes = [p, u32, p]
+        L.gcgt_dist_bfs_commit.argtypes = [p, u32, p, u32, p, C.POINTER(u64)]
+        L.gcgt_dist_bfs_absorb.argtypes = [p, p]
+        L.gcgt_dist_bfs_levels.argtypes = [p, p, i32]
+        L.gcgt_dist_cc_hook.argtypes = [p, p, C.POINTER(u64)]
+        L.gcgt_dist_cc_jump.argtypes = [p, p]
         L.gcgt_debug_warp_decode.argtypes = [p, u64, u32, u32, u64, p, p, p, C.POINTER(u32)]
         L.gcgt_last_error.restype = C.c_char_p
         L.gcgt_version.restype = C.c_char_p
@@ -246,6 +255,35 @@ class Graph:
                "gcgt_bc")
         self.last_stats = st.as_dict()
         return res
+
+    # ---- partitioned steps (dist.py); device pointers as ints -------------------------------------------------
+    def dist_bfs_begin(self, source: int):
+        _check(lib().gcgt_dist_bfs_begin(self._h, source), "gcgt_dist_bfs_begin")
+
+    def dist_bfs_expand(self, level: int, cand_ptr: int):
+        _check(lib().gcgt_dist_bfs_expand(self._h, level, C.c_void_p(cand_ptr)), "gcgt_dist_bfs_expand")
+
+    def dist_bfs_commit(self, level: int, recv_ptr: int, nparts: int, fslice_ptr: int) -> int:
+        cnt = C.c_uint64(0)
+        _check(lib().gcgt_dist_bfs_commit(self._h, level, C.c_void_p(recv_ptr), nparts, C.c_void_p(fslice_ptr),
+                                          C.byref(cnt)), "gcgt_dist_bfs_commit")
+        return int(cnt.value)
+
+    def dist_bfs_absorb(self, frontier_ptr: int):
+        _check(lib().gcgt_dist_bfs_absorb(self._h, C.c_void_p(frontier_ptr)), "gcgt_dist_bfs_absorb")
+
+    def dist_bfs_levels(self, out):
+        ptr, where, res = _out(out, self.range()[1] - self.range()[0], np.int32, "int32")
+        _check(lib().gcgt_dist_bfs_levels(self._h, ptr, where), "gcgt_dist_bfs_levels")
+        return res
+
+    def dist_cc_hook(self, parent_ptr: int) -> int:
+        h = C.c_uint64(0)
+        _check(lib().gcgt_dist_cc_hook(self._h, C.c_void_p(parent_ptr), C.byref(h)), "gcgt_dist_cc_hook")
+        return int(h.value)
+
+    def dist_cc_jump(self, parent_ptr: int):
+        _check(lib().gcgt_dist_cc_jump(self._h, C.c_void_p(parent_ptr)), "gcgt_dist_cc_jump")
 
     def unload(self):
         if self._h:

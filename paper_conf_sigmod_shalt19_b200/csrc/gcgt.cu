@@ -90,7 +90,9 @@ struct gcgt_graph {
     uint64_t lo = 0, hi = 0;
     // CGR
     uint64_t* W = nullptr;     // stream-order words (+2 pad)
-    uint64_t* offs = nullptr;  // n + 1
+    uint64_t* offs = nullptr;        // offs[u] for owned u in [lo, hi] (points offs_alloc - lo)
+    uint64_t* offs_alloc = nullptr;  // hi - lo + 1 re-based offsets
+    int rank = 0, nranks = 1;
     uint64_t* inW = nullptr;     // in-CGR (transpose) for bottom-up; aliases W / offs when symmetric
     uint64_t* inOffs = nullptr;
     bool in_owned = false;       // inW / inOffs are separate allocations
@@ -215,6 +217,21 @@ struct HeavyFront {
         const uint32_t u = q[i].u;
         w = u >> 5;
         bits = 1u << (u & 31);
+    }
+};
+
+// Frontier bits of the owned word range (partitioned BFS): entry i is word w_lo + i with its F bits restricted to
+// the owned vertices [lo, hi).
+struct BitsFront {
+    const uint32_t* __restrict__ F;
+    uint64_t lo, hi;
+    __device__ __forceinline__ uint64_t size() const { return hi > lo ? ((hi + 31) >> 5) - (lo >> 5) : 0; }
+    __device__ __forceinline__ void get(uint64_t i, uint32_t& w, uint32_t& bits) const {
+        w = (uint32_t)((lo >> 5) + i);
+        const uint64_t v0 = (uint64_t)w * 32;
+        bits = F[w];
+        if (v0 < lo) bits &= 0xffffffffu << (lo - v0);
+        if (v0 + 32 > hi) bits &= (hi - v0 >= 32) ? 0xffffffffu : ((1u << (hi - v0)) - 1);
     }
 };
 
@@ -891,14 +908,24 @@ __device__ __forceinline__ uint32_t cc_find(uint32_t* parent, uint32_t x) {  // 
 struct CcApp {
     uint32_t* parent;
     uint32_t ru;
-    __device__ __forceinline__ void begin(uint32_t u) { ru = cc_find(parent, u); }
-    __device__ __forceinline__ void end() {}
+    uint32_t* hook_ctr;  // optional: counts successful hooks (partitioned CC convergence test)
+    uint32_t hooks;
+    __device__ __forceinline__ void begin(uint32_t u) {
+        ru = cc_find(parent, u);
+        hooks = 0;
+    }
+    __device__ __forceinline__ void end() {
+        if (hook_ctr && hooks) atomicAdd(hook_ctr, hooks);
+    }
     __device__ __forceinline__ void vertex(uint32_t) {}
     __device__ __forceinline__ void one(uint32_t v) {
         uint32_t rv = cc_find(parent, v);
         while (ru != rv) {
             const uint32_t hi = max(ru, rv), lo = min(ru, rv);
-            if (atomicCAS(parent + hi, hi, lo) == hi) break;
+            if (atomicCAS(parent + hi, hi, lo) == hi) {
+                hooks++;
+                break;
+            }
             ru = cc_find(parent, ru);  // hi stopped being a root: re-find both
             rv = cc_find(parent, rv);
         }
@@ -1142,6 +1169,46 @@ __global__ void count_level(const uint32_t* qn_len, uint32_t* counter) {
     if (*qn_len) *counter += 1;
 }
 
+// ---- partitioned BFS / CC steps (the collectives run in the caller, e.g. torch.distributed over NCCL) ------------
+// Contraction of the owned slice: OR of the P candidate slices received from every rank, minus visited; writes
+// levels and the owned next-frontier slice; counts new vertices.
+__global__ void dist_commit(const uint32_t* __restrict__ recv, uint32_t P, uint64_t w_lo, uint64_t nlw,
+                            const uint32_t* __restrict__ V, uint32_t* __restrict__ fslice, int32_t* __restrict__ levels,
+                            int32_t new_level, uint64_t n, unsigned long long* __restrict__ count) {
+    const uint32_t lane = lane_id();
+    uint32_t nf = 0;
+    const uint64_t gw = ((uint64_t)blockIdx.x * blockDim.x + threadIdx.x) >> 5;
+    const uint64_t nwarps = ((uint64_t)gridDim.x * blockDim.x) >> 5;
+    for (uint64_t base = gw * 32; base < nlw; base += nwarps * 32) {
+        const uint64_t i = base + lane;
+        uint32_t b = 0;
+        if (i < nlw) {
+            for (uint32_t r = 0; r < P; r++) b |= recv[(uint64_t)r * nlw + i];
+            b &= ~V[w_lo + i];
+            fslice[i] = b;
+        }
+        nf += __popc(b);
+        for (uint32_t m = __ballot_sync(0xffffffffu, b != 0); m; m &= m - 1) {  // coalesced level stores
+            const int j = __ffs(m) - 1;
+            const uint32_t bj = __shfl_sync(0xffffffffu, b, j);
+            const uint64_t v = (w_lo + base + j) * 32 + lane;
+            if (((bj >> lane) & 1u) && v < n) levels[v] = new_level;
+        }
+    }
+    for (int o = 16; o; o >>= 1) nf += __shfl_xor_sync(0xffffffffu, nf, o);
+    if (lane == 0 && nf) atomicAdd(count, (unsigned long long)nf);
+}
+
+// F = the gathered global frontier; V |= F.
+__global__ void dist_absorb(const uint32_t* __restrict__ Fg, uint32_t* __restrict__ F, uint32_t* __restrict__ V,
+                            uint64_t nw) {
+    for (uint64_t w = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; w < nw; w += (uint64_t)gridDim.x * blockDim.x) {
+        const uint32_t b = Fg[w];
+        F[w] = b;
+        V[w] |= b;
+    }
+}
+
 __global__ void bfs_seed(uint32_t s, uint32_t* V, uint32_t* F, uint32_t* q, uint32_t* qlen, uint32_t* qbits,
                          int32_t* levels = nullptr, uint32_t* bstate = nullptr) {
     V[s >> 5] = 1u << (s & 31);
@@ -1169,22 +1236,25 @@ __global__ void bswap_words(uint64_t* w, uint64_t n) {
 // area no longer forms one serial chain (the residual-segment idea of §5.2 applied to intervals, as a derived
 // device table; the CGR bytes are unchanged).
 template <int K, bool SEG>
-__global__ void ck_count(const uint64_t* __restrict__ W, const uint64_t* __restrict__ offs, uint64_t n, uint32_t C,
-                         uint8_t* __restrict__ flag, uint32_t* __restrict__ cnt) {
-    for (uint64_t u = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; u < n; u += (uint64_t)gridDim.x * blockDim.x) {
+__global__ void ck_count(const uint64_t* __restrict__ W, const uint64_t* __restrict__ offs, uint64_t lo, uint64_t n,
+                         uint32_t C, uint8_t* __restrict__ flag, uint32_t* __restrict__ cnt) {
+    for (uint64_t i = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; i < n; i += (uint64_t)gridDim.x * blockDim.x) {
+        const uint64_t u = lo + i;  // flag / cnt are indexed by owned position; the selected ids are re-based below
         uint64_t p = ldg64(offs + u);
         if (!SEG) decode<K>(W, p);
         const uint64_t itv = decode<K>(W, p) - 1;
         const bool h = itv > C;
-        flag[u] = h;
-        cnt[u] = h ? (uint32_t)((itv - 1) / C) : 0;
+        flag[i] = h;
+        cnt[i] = h ? (uint32_t)((itv - 1) / C) : 0;
     }
 }
 
-__global__ void ck_gather(const uint32_t* __restrict__ ids, const uint32_t* __restrict__ cnt, uint32_t H,
+__global__ void ck_gather(uint32_t* __restrict__ ids, const uint32_t* __restrict__ cnt, uint32_t H, uint64_t lo,
                           uint32_t* __restrict__ out) {
-    for (uint64_t h = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; h <= H; h += (uint64_t)gridDim.x * blockDim.x)
+    for (uint64_t h = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; h <= H; h += (uint64_t)gridDim.x * blockDim.x) {
         out[h] = h < H ? cnt[ids[h]] : 0;
+        if (h < H) ids[h] += (uint32_t)lo;  // owned position -> global vertex id
+    }
 }
 
 template <int K, bool SEG>
@@ -1218,10 +1288,12 @@ __global__ void ck_fill(const uint64_t* __restrict__ W, const uint64_t* __restri
 // Load-time pass: number of hub vertices (more than kHubSegs residual segments) and heavy vertices (long
 // interval area / unsegmented list); sizes the per-level hub and heavy queues.
 template <int K, bool SEG>
-__global__ void count_special(const uint64_t* __restrict__ W, const uint64_t* __restrict__ offs, uint64_t n,
-                              uint32_t heavy_itv, uint32_t heavy_res, uint32_t hub_segs, unsigned long long* out) {
+__global__ void count_special(const uint64_t* __restrict__ W, const uint64_t* __restrict__ offs, uint64_t lo,
+                              uint64_t n, uint32_t heavy_itv, uint32_t heavy_res, uint32_t hub_segs,
+                              unsigned long long* out) {
     uint32_t hubs = 0, heavy = 0;
-    for (uint64_t u = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; u < n; u += (uint64_t)gridDim.x * blockDim.x) {
+    for (uint64_t u = lo + (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; u < n;
+         u += (uint64_t)gridDim.x * blockDim.x) {
         uint64_t p = ldg64(offs + u);
         uint64_t deg = 0;
         if (!SEG) deg = decode<K>(W, p) - 1;
@@ -1477,18 +1549,20 @@ gcgt_status build_checkpoints(gcgt_graph* g) {
     gcgt_status st;
     if ((st = galloc(g, &g->chunk_len, 1))) return st;
     CU(cudaMemsetAsync(g->chunk_len, 0, 4, g->stream));
-    if (g->ck_c == 0xFFFFFFFFu || g->n == 0) return GCGT_OK;
+    if (g->ck_c == 0xFFFFFFFFu || g->hi == g->lo) return GCGT_OK;
     cudaStream_t s = g->stream;
     const bool seg = g->P.residual_segment_len != 0;
     const uint32_t C = g->ck_c;
     uint8_t* flag = nullptr;
     uint32_t *cnt = nullptr, *ids = nullptr, *nsel = nullptr;
-    if ((st = galloc(g, &flag, g->n)) || (st = galloc(g, &cnt, g->n + 1)) || (st = galloc(g, &ids, g->n + 1)) ||
+    if ((st = galloc(g, &flag, g->hi - g->lo + 1)) || (st = galloc(g, &cnt, g->hi - g->lo + 1)) ||
+        (st = galloc(g, &ids, g->hi - g->lo + 1)) ||
         (st = galloc(g, &nsel, 1)))
         return st;
-    const int gr = flat_grid(g, g->n);
-#define GCGT_CK(KK) (seg ? ck_count<KK, true><<<gr, kBlock, 0, s>>>(g->W, g->offs, g->n, C, flag, cnt)   \
-                         : ck_count<KK, false><<<gr, kBlock, 0, s>>>(g->W, g->offs, g->n, C, flag, cnt))
+    const uint64_t nloc = g->hi - g->lo;
+    const int gr = flat_grid(g, nloc);
+#define GCGT_CK(KK) (seg ? ck_count<KK, true><<<gr, kBlock, 0, s>>>(g->W, g->offs, g->lo, nloc, C, flag, cnt)   \
+                         : ck_count<KK, false><<<gr, kBlock, 0, s>>>(g->W, g->offs, g->lo, nloc, C, flag, cnt))
     switch (g->P.zeta_k) {
         case 1: GCGT_CK(1); break;
         case 2: GCGT_CK(2); break;
@@ -1499,12 +1573,12 @@ gcgt_status build_checkpoints(gcgt_graph* g) {
 #undef GCGT_CK
     size_t tmp_bytes = 0;
     cub::CountingInputIterator<uint32_t> iota(0);
-    CU(cub::DeviceSelect::Flagged(nullptr, tmp_bytes, iota, flag, ids, nsel, (int64_t)g->n, s));
+    CU(cub::DeviceSelect::Flagged(nullptr, tmp_bytes, iota, flag, ids, nsel, (int64_t)nloc, s));
     void* tmp = nullptr;
     size_t tmp2 = 0;
-    CU(cub::DeviceScan::ExclusiveSum(nullptr, tmp2, cnt, cnt, (int64_t)g->n + 1, s));
+    CU(cub::DeviceScan::ExclusiveSum(nullptr, tmp2, cnt, cnt, (int64_t)nloc + 1, s));
     if ((st = galloc(g, (uint8_t**)&tmp, std::max(tmp_bytes, tmp2)))) return st;
-    CU(cub::DeviceSelect::Flagged(tmp, tmp_bytes, iota, flag, ids, nsel, (int64_t)g->n, s));
+    CU(cub::DeviceSelect::Flagged(tmp, tmp_bytes, iota, flag, ids, nsel, (int64_t)nloc, s));
     uint32_t H = 0;
     CU(cudaMemcpyAsync(&H, nsel, 4, cudaMemcpyDeviceToHost, s));
     CU(cudaStreamSynchronize(s));
@@ -1513,7 +1587,7 @@ gcgt_status build_checkpoints(gcgt_graph* g) {
             (st = galloc(g, &g->hv_after, H)) || (st = galloc(g, &g->hv_rem, H)))
             return st;
         CU(cudaMemcpyAsync(g->hv_ids, ids, (uint64_t)H * 4, cudaMemcpyDeviceToDevice, s));
-        ck_gather<<<flat_grid(g, H + 1), kBlock, 0, s>>>(g->hv_ids, cnt, H, ids);
+        ck_gather<<<flat_grid(g, H + 1), kBlock, 0, s>>>(g->hv_ids, cnt, H, g->lo, ids);
         // ids now holds the per-heavy-vertex counts (+ a trailing 0); scan into hv_ptr
         tmp2 = std::max(tmp_bytes, tmp2);
         CU(cub::DeviceScan::ExclusiveSum(tmp, tmp2, ids, g->hv_ptr, (int64_t)H + 1, s));
@@ -1555,7 +1629,7 @@ gcgt_status build_checkpoints(gcgt_graph* g) {
 extern "C" void gcgt_unload(gcgt_graph* g) {
     if (!g) return;
     cudaSetDevice(g->device);
-    void* bufs[] = {g->W,      g->offs,    g->V,      g->F,         g->N,        g->q,      g->qbits,
+    void* bufs[] = {g->W,      g->offs_alloc, g->V,      g->F,         g->N,        g->q,      g->qbits,
                     g->ctr,    g->hubq,    g->hub_ctr, g->cursor,   g->heavyq,   g->heavy_len, g->stats,
                     g->levels, g->parent,  g->sigma,  g->delta,     g->bc,      g->bstate,
                     g->hv_ids, g->hv_ptr,  g->hv_rem, g->ck_prev,   g->chunk_len, g->hv_after, g->ck_pos, g->chunkq,
@@ -1580,7 +1654,7 @@ extern "C" gcgt_status gcgt_load(const gcgt_cgr* c, const gcgt_load_opts* opts, 
     if (!c || !out) return fail(GCGT_EINVAL, "null argument");
     gcgt_load_opts o{};
     if (opts) o = *opts;
-    if (o.nranks > 1) return fail(GCGT_EINVAL, "multi-rank load: use gcgt_load with the NCCL build (not in this build)");
+    if (o.nranks > 1 && (o.rank < 0 || o.rank >= o.nranks)) return fail(GCGT_EINVAL, "bad rank");
     int ndev = 0;
     if (cudaGetDeviceCount(&ndev) != cudaSuccess || ndev == 0) return fail(GCGT_ECUDA, "no CUDA device");
     if (o.device < 0 || o.device >= ndev) return fail(GCGT_EINVAL, "bad device ordinal");
@@ -1629,12 +1703,31 @@ extern "C" gcgt_status gcgt_load(const gcgt_cgr* c, const gcgt_load_opts* opts, 
             i = j + 1;
         }
     }
+    // 1-D vertex-range partition (§8 e): rank r owns [lo, hi), boundaries on 32-vertex words, balanced by CGR bits.
+    // Records are self-contained, so the slice is a copy of whole 64-bit words plus re-based bit offsets.
     g->lo = 0;
     g->hi = c->n;
+    g->nranks = o.nranks > 1 ? o.nranks : 1;
+    g->rank = o.nranks > 1 ? o.rank : 0;
+    if (g->nranks > 1) {
+        auto bound = [&](int r) -> uint64_t {
+            if (r <= 0) return 0;
+            if (r >= g->nranks) return c->n;
+            const uint64_t target = c->nbits / (uint64_t)g->nranks * (uint64_t)r;
+            const uint64_t v = (uint64_t)(std::lower_bound(c->bit_offsets.begin(), c->bit_offsets.end(), target) -
+                                          c->bit_offsets.begin());
+            return std::min<uint64_t>(c->n, v & ~31ull);
+        };
+        g->lo = bound(g->rank);
+        g->hi = std::max(g->lo, bound(g->rank + 1));
+        g->dir_opt_knob = false;  // bottom-up needs the whole in-CGR: top-down only when partitioned
+    }
     g->nw = (c->n + 31) / 32 + 1;
-    const uint64_t nwords = (c->nbits + 63) / 64 + 2;
+    const uint64_t w0 = c->bit_offsets[g->lo] / 64;
+    const uint64_t nwords = (c->bit_offsets[g->hi] + 63) / 64 - w0 + 2;
+    const uint64_t nloc = g->hi - g->lo;
     gcgt_status st;
-    if ((st = galloc(g.get(), &g->W, nwords)) || (st = galloc(g.get(), &g->offs, g->n + 1)) || (st = galloc(g.get(), &g->V, g->nw)) ||
+    if ((st = galloc(g.get(), &g->W, nwords)) || (st = galloc(g.get(), &g->offs_alloc, nloc + 1)) || (st = galloc(g.get(), &g->V, g->nw)) ||
         (st = galloc(g.get(), &g->F, g->nw)) || (st = galloc(g.get(), &g->N, g->nw)) || (st = galloc(g.get(), &g->ctr, 8)) ||
         (st = galloc(g.get(), &g->stats, 1)) || (st = galloc(g.get(), &g->levels, g->n)))
         return st;
@@ -1646,9 +1739,22 @@ extern "C" gcgt_status gcgt_load(const gcgt_cgr* c, const gcgt_load_opts* opts, 
     CU(cudaEventCreate(&g->ev1));
     CU(cudaEventCreate(&g->kev0));
     CU(cudaEventCreate(&g->kev1));
-    CU(cudaMemcpyAsync(g->W, c->words.data(), nwords * sizeof(uint64_t), cudaMemcpyHostToDevice, g->stream));
-    CU(cudaMemcpyAsync(g->offs, c->bit_offsets.data(), (g->n + 1) * sizeof(uint64_t), cudaMemcpyHostToDevice,
-                       g->stream));
+    {
+        const uint64_t avail = c->words.size() - w0;  // the host array holds >= 2 padding words
+        CU(cudaMemsetAsync(g->W, 0, nwords * sizeof(uint64_t), g->stream));
+        CU(cudaMemcpyAsync(g->W, c->words.data() + w0, std::min(nwords, avail) * sizeof(uint64_t),
+                           cudaMemcpyHostToDevice, g->stream));
+    }
+    if (w0 == 0) {
+        CU(cudaMemcpyAsync(g->offs_alloc, c->bit_offsets.data() + g->lo, (nloc + 1) * sizeof(uint64_t),
+                           cudaMemcpyHostToDevice, g->stream));
+    } else {
+        std::vector<uint64_t> ro(c->bit_offsets.begin() + g->lo, c->bit_offsets.begin() + g->hi + 1);
+        for (auto& x : ro) x -= w0 * 64;
+        CU(cudaMemcpyAsync(g->offs_alloc, ro.data(), (nloc + 1) * sizeof(uint64_t), cudaMemcpyHostToDevice, g->stream));
+        CU(cudaStreamSynchronize(g->stream));  // ro is a stack vector
+    }
+    g->offs = g->offs_alloc - g->lo;  // kernels index offs[u] with global vertex ids
     bswap_words<<<flat_grid(g.get(), nwords), kBlock, 0, g->stream>>>(g->W, nwords);
     CU(cudaMemsetAsync(g->N, 0, g->nw * 4, g->stream));
     if ((st = galloc(g.get(), &g->bstate, 8))) return st;
@@ -1682,11 +1788,11 @@ extern "C" gcgt_status gcgt_load(const gcgt_cgr* c, const gcgt_load_opts* opts, 
         const bool seg = g->P.residual_segment_len != 0;
         cudaStream_t s = g->stream;
         switch (g->P.zeta_k) {
-            case 1: seg ? count_special<1, true><<<gr, kBlock, 0, s>>>(g->W, g->offs, g->n, g->heavy_itv, g->heavy_res, g->hub_segs, dcount) : count_special<1, false><<<gr, kBlock, 0, s>>>(g->W, g->offs, g->n, g->heavy_itv, g->heavy_res, g->hub_segs, dcount); break;
-            case 2: seg ? count_special<2, true><<<gr, kBlock, 0, s>>>(g->W, g->offs, g->n, g->heavy_itv, g->heavy_res, g->hub_segs, dcount) : count_special<2, false><<<gr, kBlock, 0, s>>>(g->W, g->offs, g->n, g->heavy_itv, g->heavy_res, g->hub_segs, dcount); break;
-            case 3: seg ? count_special<3, true><<<gr, kBlock, 0, s>>>(g->W, g->offs, g->n, g->heavy_itv, g->heavy_res, g->hub_segs, dcount) : count_special<3, false><<<gr, kBlock, 0, s>>>(g->W, g->offs, g->n, g->heavy_itv, g->heavy_res, g->hub_segs, dcount); break;
-            case 4: seg ? count_special<4, true><<<gr, kBlock, 0, s>>>(g->W, g->offs, g->n, g->heavy_itv, g->heavy_res, g->hub_segs, dcount) : count_special<4, false><<<gr, kBlock, 0, s>>>(g->W, g->offs, g->n, g->heavy_itv, g->heavy_res, g->hub_segs, dcount); break;
-            default: seg ? count_special<5, true><<<gr, kBlock, 0, s>>>(g->W, g->offs, g->n, g->heavy_itv, g->heavy_res, g->hub_segs, dcount) : count_special<5, false><<<gr, kBlock, 0, s>>>(g->W, g->offs, g->n, g->heavy_itv, g->heavy_res, g->hub_segs, dcount); break;
+            case 1: seg ? count_special<1, true><<<gr, kBlock, 0, s>>>(g->W, g->offs, g->lo, g->hi, g->heavy_itv, g->heavy_res, g->hub_segs, dcount) : count_special<1, false><<<gr, kBlock, 0, s>>>(g->W, g->offs, g->lo, g->hi, g->heavy_itv, g->heavy_res, g->hub_segs, dcount); break;
+            case 2: seg ? count_special<2, true><<<gr, kBlock, 0, s>>>(g->W, g->offs, g->lo, g->hi, g->heavy_itv, g->heavy_res, g->hub_segs, dcount) : count_special<2, false><<<gr, kBlock, 0, s>>>(g->W, g->offs, g->lo, g->hi, g->heavy_itv, g->heavy_res, g->hub_segs, dcount); break;
+            case 3: seg ? count_special<3, true><<<gr, kBlock, 0, s>>>(g->W, g->offs, g->lo, g->hi, g->heavy_itv, g->heavy_res, g->hub_segs, dcount) : count_special<3, false><<<gr, kBlock, 0, s>>>(g->W, g->offs, g->lo, g->hi, g->heavy_itv, g->heavy_res, g->hub_segs, dcount); break;
+            case 4: seg ? count_special<4, true><<<gr, kBlock, 0, s>>>(g->W, g->offs, g->lo, g->hi, g->heavy_itv, g->heavy_res, g->hub_segs, dcount) : count_special<4, false><<<gr, kBlock, 0, s>>>(g->W, g->offs, g->lo, g->hi, g->heavy_itv, g->heavy_res, g->hub_segs, dcount); break;
+            default: seg ? count_special<5, true><<<gr, kBlock, 0, s>>>(g->W, g->offs, g->lo, g->hi, g->heavy_itv, g->heavy_res, g->hub_segs, dcount) : count_special<5, false><<<gr, kBlock, 0, s>>>(g->W, g->offs, g->lo, g->hi, g->heavy_itv, g->heavy_res, g->hub_segs, dcount); break;
         }
     }
     unsigned long long counts[2] = {0, 0};
@@ -1783,6 +1889,7 @@ extern "C" gcgt_status gcgt_graph_range(const gcgt_graph* g, uint64_t* lo, uint6
 
 extern "C" gcgt_status gcgt_bfs(gcgt_graph* g, uint32_t source, int32_t* levels, int placement, gcgt_stats* stats) {
     if (!g || !levels) return fail(GCGT_EINVAL, "null argument");
+    if (g->nranks > 1) return fail(GCGT_EINVAL, "partitioned graph: use the gcgt_dist_* steps (dist.py)");
     if (source >= g->n) return fail(GCGT_ERANGE, "source >= n");
     gcgt_status st;
     if ((st = begin_call(g))) return st;
@@ -1862,6 +1969,7 @@ extern "C" gcgt_status gcgt_bfs(gcgt_graph* g, uint32_t source, int32_t* levels,
 
 extern "C" gcgt_status gcgt_cc(gcgt_graph* g, uint32_t* labels, int placement, gcgt_stats* stats) {
     if (!g || !labels) return fail(GCGT_EINVAL, "null argument");
+    if (g->nranks > 1) return fail(GCGT_EINVAL, "partitioned graph: use the gcgt_dist_* steps (dist.py)");
     gcgt_status st;
     if (!g->parent && (st = galloc(g, &g->parent, g->n))) return st;
     if ((st = begin_call(g))) return st;
@@ -1872,7 +1980,7 @@ extern "C" gcgt_status gcgt_cc(gcgt_graph* g, uint32_t* labels, int placement, g
     cc_init<<<flat_grid(g, g->n), kBlock, 0, s>>>(g->parent, g->n);
     const Ctx c = make_ctx(g);
     const DenseFront fr{g->lo, g->hi};
-    const CcApp app{g->parent, 0};
+    const CcApp app{g->parent, 0, nullptr, 0};
     int grid;
     uint32_t wpb;
     frontier_launch(g, (g->hi - g->lo + 31) / 32 + 1, &grid, &wpb);
@@ -1891,6 +1999,7 @@ extern "C" gcgt_status gcgt_cc(gcgt_graph* g, uint32_t* labels, int placement, g
 extern "C" gcgt_status gcgt_bc(gcgt_graph* g, const uint32_t* sources, uint32_t k, double* bc, int placement,
                                gcgt_stats* stats) {
     if (!g || !bc || (k && !sources)) return fail(GCGT_EINVAL, "null argument");
+    if (g->nranks > 1) return fail(GCGT_EINVAL, "partitioned graph: BC shards sources over full replicas (dist.py)");
     for (uint32_t i = 0; i < k; i++)
         if (sources[i] >= g->n) return fail(GCGT_ERANGE, "source >= n");
     gcgt_status st;
@@ -1969,4 +2078,125 @@ extern "C" gcgt_status gcgt_bc(gcgt_graph* g, const uint32_t* sources, uint32_t 
     }
     if ((st = copy_out(g, bc, g->bc, g->n * 8, placement))) return st;
     return end_call(g, stats, k);
+}
+
+// ------------------------------------------------------------------------------------------------------------------
+// Partitioned (multi-GPU) steps.  The caller (paper_conf_sigmod_shalt19_b200/dist.py) runs the collectives between
+// them; all bitmaps crossing the boundary are device arrays of ceil(n/32) 32-bit words (bit v%32 of word v/32).
+// ------------------------------------------------------------------------------------------------------------------
+namespace {
+gcgt_status dist_sync(gcgt_graph* g) {
+    CU(cudaStreamSynchronize(g->stream));
+    CU(cudaGetLastError());
+    return GCGT_OK;
+}
+}  // namespace
+
+extern "C" gcgt_status gcgt_dist_bfs_begin(gcgt_graph* g, uint32_t source) {
+    gcgt_internal::clear_error();
+    if (!g) return fail(GCGT_EINVAL, "null graph");
+    if (source >= g->n) return fail(GCGT_ERANGE, "source >= n");
+    CU(cudaSetDevice(g->device));
+    cudaStream_t s = g->stream;
+    CU(cudaMemsetAsync(g->V, 0, g->nw * 4, s));
+    CU(cudaMemsetAsync(g->F, 0, g->nw * 4, s));
+    CU(cudaMemsetAsync(g->levels, 0xff, g->n * 4, s));
+    CU(cudaMemsetAsync(g->hub_ctr, 0, 8, s));
+    CU(cudaMemsetAsync(g->chunk_len, 0, 4, s));
+    CU(cudaMemsetAsync(g->heavy_len, 0, 4, s));
+    CU(cudaMemsetAsync(g->ctr, 0, 8 * 4, s));
+    bfs_seed<<<1, 1, 0, s>>>(source, g->V, g->F, g->q, g->ctr, nullptr, g->levels, nullptr);
+    return dist_sync(g);
+}
+
+extern "C" gcgt_status gcgt_dist_bfs_expand(gcgt_graph* g, uint32_t level, uint32_t* cand) {
+    gcgt_internal::clear_error();
+    if (!g || !cand) return fail(GCGT_EINVAL, "null argument");
+    CU(cudaSetDevice(g->device));
+    cudaStream_t s = g->stream;
+    CU(cudaMemsetAsync(cand, 0, ((g->n + 31) / 32) * 4, s));
+    const Ctx c = make_ctx(g);
+    const BitsFront fr{g->F, g->lo, g->hi};
+    const BfsApp app{g->V, cand, g->levels, (int32_t)level};
+    int grid;
+    uint32_t wpb;
+    frontier_launch(g, (g->hi - g->lo + 31) / 32 + 1, &grid, &wpb);
+    launch_expand(g->P, g->staged, grid, s, c, fr, app, 0);
+    launch_heavy(g, s, c, app);
+    launch_hub(g->P, g->staged, hub_grid(g), s, c, app);
+    CU(cudaMemsetAsync(g->hub_ctr, 0, 8, s));
+    CU(cudaMemsetAsync(g->chunk_len, 0, 4, s));
+    CU(cudaMemsetAsync(g->heavy_len, 0, 4, s));
+    return dist_sync(g);
+}
+
+extern "C" gcgt_status gcgt_dist_bfs_commit(gcgt_graph* g, uint32_t level, const uint32_t* recv, uint32_t nparts,
+                                            uint32_t* fslice, uint64_t* new_count) {
+    gcgt_internal::clear_error();
+    if (!g || !recv || !fslice || !new_count || nparts == 0) return fail(GCGT_EINVAL, "null argument");
+    CU(cudaSetDevice(g->device));
+    cudaStream_t s = g->stream;
+    const uint64_t w_lo = g->lo / 32, nlw = (g->hi + 31) / 32 - w_lo;
+    unsigned long long* cnt = (unsigned long long*)g->stats;  // scratch: reuse the stats block
+    CU(cudaMemsetAsync(cnt, 0, 8, s));
+    if (nlw)
+        dist_commit<<<flat_grid(g, nlw * 32), kBlock, 0, s>>>(recv, nparts, w_lo, nlw, g->V, fslice, g->levels,
+                                                               (int32_t)level + 1, g->n, cnt);
+    CU(cudaMemcpyAsync(g->h_stats, cnt, 8, cudaMemcpyDeviceToHost, s));
+    gcgt_status st = dist_sync(g);
+    if (st) return st;
+    *new_count = g->h_stats->vertices;
+    CU(cudaMemsetAsync(g->stats, 0, sizeof(Stats), s));
+    return dist_sync(g);
+}
+
+extern "C" gcgt_status gcgt_dist_bfs_absorb(gcgt_graph* g, const uint32_t* frontier) {
+    gcgt_internal::clear_error();
+    if (!g || !frontier) return fail(GCGT_EINVAL, "null argument");
+    CU(cudaSetDevice(g->device));
+    const uint64_t nwf = (g->n + 31) / 32;
+    dist_absorb<<<flat_grid(g, nwf), kBlock, 0, g->stream>>>(frontier, g->F, g->V, nwf);
+    return dist_sync(g);
+}
+
+extern "C" gcgt_status gcgt_dist_bfs_levels(gcgt_graph* g, int32_t* levels_owned, int placement) {
+    gcgt_internal::clear_error();
+    if (!g || !levels_owned) return fail(GCGT_EINVAL, "null argument");
+    gcgt_status st;
+    if ((st = copy_out(g, levels_owned, g->levels + g->lo, (g->hi - g->lo) * 4, placement))) return st;
+    return dist_sync(g);
+}
+
+extern "C" gcgt_status gcgt_dist_cc_hook(gcgt_graph* g, uint32_t* parent, uint64_t* hooks) {
+    gcgt_internal::clear_error();
+    if (!g || !parent || !hooks) return fail(GCGT_EINVAL, "null argument");
+    CU(cudaSetDevice(g->device));
+    cudaStream_t s = g->stream;
+    uint32_t* hc = g->ctr + 7;
+    CU(cudaMemsetAsync(hc, 0, 4, s));
+    CU(cudaMemsetAsync(g->hub_ctr, 0, 8, s));
+    CU(cudaMemsetAsync(g->chunk_len, 0, 4, s));
+    CU(cudaMemsetAsync(g->heavy_len, 0, 4, s));
+    const Ctx c = make_ctx(g);
+    const DenseFront fr{g->lo, g->hi};
+    const CcApp app{parent, 0, hc, 0};
+    int grid;
+    uint32_t wpb;
+    frontier_launch(g, (g->hi - g->lo + 31) / 32 + 1, &grid, &wpb);
+    launch_expand(g->P, g->staged, grid, s, c, fr, app, wpb);
+    launch_heavy(g, s, c, app);
+    launch_hub(g->P, g->staged, hub_grid(g), s, c, app);
+    CU(cudaMemcpyAsync(g->h_ctr + 7, hc, 4, cudaMemcpyDeviceToHost, s));
+    gcgt_status st = dist_sync(g);
+    if (st) return st;
+    *hooks = g->h_ctr[7];
+    return GCGT_OK;
+}
+
+extern "C" gcgt_status gcgt_dist_cc_jump(gcgt_graph* g, uint32_t* parent) {
+    gcgt_internal::clear_error();
+    if (!g || !parent) return fail(GCGT_EINVAL, "null argument");
+    CU(cudaSetDevice(g->device));
+    cc_jump<<<flat_grid(g, g->n), kBlock, 0, g->stream>>>(parent, g->n);
+    return dist_sync(g);
 }
