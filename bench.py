@@ -6,8 +6,9 @@
 A step is one BFS query (the whole §8(a) path: frontier management, header / interval / residual-segment decode,
 filter, contraction) from a seeded root over the device-resident CGR of the configuration's synthetic graph.
 Default workload = BASELINE.json configs[1] (uk-2002-like web graph, 18.5M vertices) on 1 B200.
-With N > 1 ranks every rank runs its own stream of BFS queries on a full replica ("weak" scaling over independent
-queries; no data-path collective); value = all ranks' traversed edges / max-over-ranks time.
+With N > 1 ranks (torchrun, NCCL) the graph is 1-D vertex-range partitioned: rank 0 builds and caches
+the CGR, every rank loads only its slice, and each BFS exchanges the next-frontier bitmap per level (all-to-all +
+all-gather over NVLink); "strong" scaling (the same graph and queries at every N); time = max over ranks.
 `--impl reference` times the oracle (oracle/, plain C, 1 thread) on the same workload (rank 0 only).
 Prints ONE JSON line on rank 0.
 """
@@ -40,6 +41,8 @@ def parse():
     ap.add_argument("--roots", type=int, default=16)
     ap.add_argument("--no-cpu-baseline", action="store_true")
     ap.add_argument("--no-e2e", action="store_true")
+    ap.add_argument("--dist-backend", default="nccl", choices=["nccl", "gloo"],
+                    help="gloo (+ host-staged exchange) only to smoke-test the N>1 path with ranks sharing one GPU")
     return ap.parse_args()
 
 
@@ -176,10 +179,14 @@ def main():
 
     if ws > 1:
         os.environ.setdefault("MASTER_ADDR", "127.0.0.1")
+        local = local % torch.cuda.device_count()
         torch.cuda.set_device(local)
-        dist.init_process_group("nccl", device_id=torch.device("cuda", local))
-    else:
-        torch.cuda.set_device(local)
+        if args.dist_backend == "nccl":
+            dist.init_process_group("nccl", device_id=torch.device("cuda", local))
+        else:
+            dist.init_process_group("gloo")
+        return run_partitioned(args, cfg, ws, rank, local)
+    torch.cuda.set_device(local)
     dev = torch.device("cuda", local)
 
     ro, co, tgen = make_graph(cfg)
@@ -288,6 +295,86 @@ def main():
     g.unload()
     if ws > 1:
         dist.destroy_process_group()
+
+
+def run_partitioned(args, cfg, ws, rank, local):
+    """N > 1: partitioned BFS (§8(e)); one JSON line from rank 0."""
+    import torch
+    import torch.distributed as dist
+    import paper_conf_sigmod_shalt19_b200 as G
+    from paper_conf_sigmod_shalt19_b200.dist import DistBFS, GraphOps
+    dev = torch.device("cuda", local)
+    path = os.path.join("/tmp", f"gcgt_bench_{cfg.name}.cgr")
+    meta = [None]
+    t0 = time.time()
+    if rank == 0:
+        ro, co, tgen = make_graph(cfg)
+        cgr = G.encode(ro, co, cfg.min_interval_len, cfg.residual_segment_len, cfg.zeta_k)
+        if args.dist_backend != "nccl":
+            path = path + f".{os.getpid()}"
+        cgr.save(path)
+        roots = choose_roots(ro, args.roots)
+        deg = np.diff(ro.astype(np.int64))
+        meta = [{"roots": roots, "m": int(ro[-1]), "deg_path": path + ".deg.npy", "path": path}]
+        np.save(meta[0]["deg_path"], deg)
+        del ro, co
+    dist.broadcast_object_list(meta, src=0)
+    meta = meta[0]
+    path = meta["path"]
+    cgr = G.open_cgr(path)
+    _, nbits, _, n, _ = cgr.view()
+    g = G.load(cgr, device=local, stream="torch", rank=rank, nranks=ws)
+    del cgr
+    deg = np.load(meta["deg_path"])
+    d = DistBFS(GraphOps(g, dev), exchange_on_host=args.dist_backend != "nccl")
+    roots = meta["roots"]
+    tprep = time.time() - t0
+    edges_of_root = {}
+    for r in sorted(set(roots)):
+        lv, _ = d.bfs(r)
+        edges_of_root[r] = edges_of(cfg, int(deg[lv >= 0].sum()))
+    for i in range(args.warmup):
+        d.bfs(roots[i % len(roots)])
+    stream = torch.cuda.current_stream(dev)
+    evs = [(torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)) for _ in range(args.steps)]
+    clocks = ClockSampler(local)
+    dist.barrier()
+    torch.cuda.synchronize()
+    clocks.start()
+    edges, levels = 0.0, 0
+    for i in range(args.steps):
+        r = roots[(args.warmup + i) % len(roots)]
+        evs[i][0].record(stream)
+        _, nlev = d.bfs(r)
+        evs[i][1].record(stream)
+        edges += edges_of_root[r]
+        levels += nlev
+    torch.cuda.synchronize()
+    dist.barrier()
+    ck = clocks.stop()
+    t_ms = sum(a.elapsed_time(b) for a, b in evs)
+    tt = torch.tensor([t_ms], dtype=torch.float64, device=dev)
+    dist.all_reduce(tt, op=dist.ReduceOp.MAX)
+    t_ms = float(tt.item())
+    lo, hi = g.range()
+    if rank == 0:
+        line = {"metric": METRIC, "value": edges / (t_ms * 1e-3) / 1e9, "unit": "GTEPS", "n_gpus": ws,
+                "steps": args.steps, "warmup": args.warmup, "ms_per_step": t_ms / args.steps,
+                "higher_is_better": True, "scaling": "strong", "vs_baseline": None, "dtype": "u32",
+                "data": "synthetic",
+                "config": {"workload": cfg.name + ": " + cfg.desc, "n": int(n), "m": meta["m"],
+                           "bits_per_arc": nbits / max(1, meta["m"]), "parallelism": f"{ws}-way 1-D vertex-range "
+                           "partition, per-level all-to-all + all-gather of frontier bitmaps (NCCL)",
+                           "levels_per_bfs": levels / args.steps, "rank0_range": [lo, hi],
+                           "edges_per_bfs": edges / args.steps, "prep_s": round(tprep, 1),
+                           "l2": "inputs (CGR slices) resident; bitmaps L2-resident; no flush"},
+                "roofline": None, "cpu_baseline": None, "e2e": None,
+                "note": "roofline / e2e are reported on the 1-GPU line; per level each rank launches expand, hub, "
+                        "commit and absorb kernels (+ NCCL collectives)",
+                "gpu_launches": int(4 * levels + 2 * args.steps), "clocks": ck}
+        print(json.dumps(line), flush=True)
+    g.unload()
+    dist.destroy_process_group()
 
 
 def measure_e2e(G, cgr, incgr, roots, edges_of_root, cfg, n, nbits, dev, local, steps=3):
