@@ -119,6 +119,10 @@ void gcgt_unload(gcgt_graph* g);
  * Adds one event pair per launch; results are unchanged. */
 gcgt_status gcgt_profile(gcgt_graph* g, int enable);
 
+/* With profiling on, the last gcgt_bfs call's device time split into spans (ms): [0] top-down expansion kernel(s),
+ * [1] hub segments / interval chunks, [2] bottom-up kernel, [3] contraction + direction choice.  count <= 4. */
+gcgt_status gcgt_profile_spans(const gcgt_graph* g, double* ms, int count);
+
 /* Owned vertex range [*lo, *hi) of this rank (whole [0, n) on a single GPU). */
 gcgt_status gcgt_graph_range(const gcgt_graph* g, uint64_t* lo, uint64_t* hi);
 

@@ -22,7 +22,7 @@ OUT_HOST, OUT_DEVICE = 0, 1
 
 # public symbols of include/gcgt.h (tests check the library exports every one)
 ABI_SYMBOLS = ["gcgt_encode", "gcgt_encode_transpose", "gcgt_cgr_view", "gcgt_cgr_from_arrays", "gcgt_cgr_save", "gcgt_cgr_open",
-               "gcgt_cgr_free", "gcgt_load", "gcgt_unload", "gcgt_profile", "gcgt_graph_range", "gcgt_bfs", "gcgt_cc", "gcgt_bc",
+               "gcgt_cgr_free", "gcgt_load", "gcgt_unload", "gcgt_profile", "gcgt_profile_spans", "gcgt_graph_range", "gcgt_bfs", "gcgt_cc", "gcgt_bc",
                "gcgt_dist_bfs_begin", "gcgt_dist_bfs_expand", "gcgt_dist_bfs_commit", "gcgt_dist_bfs_absorb",
                "gcgt_dist_bfs_levels", "gcgt_dist_cc_hook", "gcgt_dist_cc_jump",
                "gcgt_debug_warp_decode", "gcgt_last_error", "gcgt_version"]
@@ -80,6 +80,7 @@ def lib():
         L.gcgt_unload.argtypes = [p]
         L.gcgt_unload.restype = None
         L.gcgt_profile.argtypes = [p, i32]
+        L.gcgt_profile_spans.argtypes = [p, p, i32]
         L.gcgt_graph_range.argtypes = [p, C.POINTER(u64), C.POINTER(u64)]
         L.gcgt_bfs.argtypes = [p, u32, p, i32, C.POINTER(Stats)]
         L.gcgt_cc.argtypes = [p, p, i32, C.POINTER(Stats)]
@@ -227,6 +228,12 @@ class Graph:
 
     def profile(self, enable: bool = True):
         _check(lib().gcgt_profile(self._h, 1 if enable else 0), "gcgt_profile")
+
+    def profile_spans(self):
+        """Last profiled gcgt_bfs split into spans (ms): expand, hub, bottom-up, contraction."""
+        a = np.zeros(4, dtype=np.float64)
+        _check(lib().gcgt_profile_spans(self._h, _np_ptr(a), 4), "gcgt_profile_spans")
+        return dict(zip(["expand", "hub", "bottom_up", "contract"], [float(x) for x in a]))
 
     def range(self):
         lo, hi = C.c_uint64(), C.c_uint64()

@@ -135,6 +135,8 @@ struct gcgt_graph {
     // profiling of the dominant kernel
     bool profile = false;
     cudaEvent_t kev0 = nullptr, kev1 = nullptr;
+    cudaEvent_t sev[5] = {nullptr, nullptr, nullptr, nullptr, nullptr};  // span marks within a BFS level
+    double span_ms[4] = {0, 0, 0, 0};  // expand(+heavy), hub, bottom-up, contraction (+decide)
     double kernel_ms = 0;
     uint64_t kernel_launches = 0;
     uint64_t launches = 0;  // kernels launched by the current call (gcgt_stats.launches)
@@ -1499,6 +1501,7 @@ gcgt_status begin_call(gcgt_graph* g) {
     g->kernel_ms = 0;
     g->kernel_launches = 0;
     g->launches = 0;
+    for (double& x : g->span_ms) x = 0;
     CU(cudaMemsetAsync(g->stats, 0, sizeof(Stats), g->stream));
     CU(cudaEventRecord(g->ev0, g->stream));
     return GCGT_OK;
@@ -1645,6 +1648,8 @@ extern "C" void gcgt_unload(gcgt_graph* g) {
     if (g->ev1) cudaEventDestroy(g->ev1);
     if (g->kev0) cudaEventDestroy(g->kev0);
     if (g->kev1) cudaEventDestroy(g->kev1);
+    for (auto& e : g->sev)
+        if (e) cudaEventDestroy(e);
     if (g->own_stream && g->stream) cudaStreamDestroy(g->stream);
     delete g;
 }
@@ -1880,6 +1885,12 @@ extern "C" gcgt_status gcgt_profile(gcgt_graph* g, int enable) {
     return GCGT_OK;
 }
 
+extern "C" gcgt_status gcgt_profile_spans(const gcgt_graph* g, double* ms, int count) {
+    if (!g || !ms) return fail(GCGT_EINVAL, "null argument");
+    for (int k = 0; k < count && k < 4; k++) ms[k] = g->span_ms[k];
+    return GCGT_OK;
+}
+
 extern "C" gcgt_status gcgt_graph_range(const gcgt_graph* g, uint64_t* lo, uint64_t* hi) {
     if (!g) return fail(GCGT_EINVAL, "null graph");
     if (lo) *lo = g->lo;
@@ -1943,10 +1954,14 @@ extern "C" gcgt_status gcgt_bfs(gcgt_graph* g, uint32_t source, int32_t* levels,
             const BfsApp app{g->V, g->N, g->levels, (int32_t)level};
             // profiled span = the level's expansion: top-down kernel (+ heavy pass + hub segments) or bottom-up
             if ((st = kprof_begin(g))) return st;
+            if (g->profile) CU(cudaEventRecord(g->sev[0], s));
             launch_expand(g->P, g->staged, grid, s, c, fr, app, wpb);
             launch_heavy(g, s, c, app);
+            if (g->profile) CU(cudaEventRecord(g->sev[1], s));
             launch_hub(g->P, g->staged, hub_grid(g), s, c, app);
+            if (g->profile) CU(cudaEventRecord(g->sev[2], s));
             if (g->dir_opt) launch_bu(g, s);
+            if (g->profile) CU(cudaEventRecord(g->sev[3], s));
             if ((st = kprof_end(g))) return st;
             commit_dense<<<flat_grid(g, g->nw), kBlock, 0, s>>>(g->V, g->F, g->N, 0, g->nw, q[nxt], g->ctr + nxt,
                                                                  nullptr, g->ctr + cur, g->hub_ctr, g->heavy_len,
@@ -1954,6 +1969,15 @@ extern "C" gcgt_status gcgt_bfs(gcgt_graph* g, uint32_t source, int32_t* levels,
                                                                  g->chunk_len);
             bfs_decide<<<1, 1, 0, s>>>(g->bstate, g->n, g->bu_alpha, g->bu_beta, g->dir_opt ? 1 : 0);
             count_level<<<1, 1, 0, s>>>(g->ctr + nxt, g->ctr + 6);
+            if (g->profile) {  // profiling waits per level anyway (nlev = 1)
+                CU(cudaEventRecord(g->sev[4], s));
+                CU(cudaEventSynchronize(g->sev[4]));
+                for (int k = 0; k < 4; k++) {
+                    float ms = 0;
+                    CU(cudaEventElapsedTime(&ms, g->sev[k], g->sev[k + 1]));
+                    g->span_ms[k] += ms;
+                }
+            }
             g->launches += 4 + (g->P.residual_segment_len ? 1 : 0) + (g->dir_opt ? 1 : 0) + (heavy_active(g) ? 1 : 0);
         }
         CU(cudaMemcpyAsync(g->h_ctr + 6, g->ctr + 6, 4, cudaMemcpyDeviceToHost, s));

@@ -25,10 +25,13 @@ for tune in tunes:
     g.profile(True)
     t = 0.0
     k = 0.0
+    spans = {}
     for r in roots:
         g.bfs(r, out=out)
         t += g.last_stats["device_ms"]
         k += g.last_stats["kernel_ms"]
+        for kk, vv in g.profile_spans().items():
+            spans[kk] = spans.get(kk, 0.0) + vv / len(roots)
     g.profile(False)
     t2 = 0.0
     for r in roots:
@@ -36,5 +39,5 @@ for tune in tunes:
         t2 += g.last_stats["device_ms"]
     arcs = g.last_stats["arcs_decoded"]
     print(f"{tune:45s} bfs {t2 / len(roots):7.3f} ms (profiled {t / len(roots):7.3f})  expand {k / len(roots):7.3f} ms"
-          f"  ~{arcs / (t2 / len(roots)) / 1e6:6.1f} GTEPS", flush=True)
+          f"  spans {{{', '.join(f'{a}: {b:.2f}' for a, b in spans.items())}}}", flush=True)
     g.unload()
