@@ -1744,6 +1744,7 @@ extern "C" gcgt_status gcgt_load(const gcgt_cgr* c, const gcgt_load_opts* opts, 
     CU(cudaEventCreate(&g->ev1));
     CU(cudaEventCreate(&g->kev0));
     CU(cudaEventCreate(&g->kev1));
+    for (auto& e : g->sev) CU(cudaEventCreate(&e));
     {
         const uint64_t avail = c->words.size() - w0;  // the host array holds >= 2 padding words
         CU(cudaMemsetAsync(g->W, 0, nwords * sizeof(uint64_t), g->stream));
