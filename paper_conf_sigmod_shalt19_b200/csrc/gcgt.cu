@@ -325,6 +325,7 @@ struct WarpSmem {
     uint32_t w[32], b[32], pre[33];
     uint32_t u[32], spre[33];
     uint64_t base[32];
+    uint32_t ckb[32], nck[32], itv[32];  // interval-chunk tasks of long interval areas (checkpoint table)
 };
 
 // DEFER = true: the level's frontier pass (heavy vertices are queued); false: the heavy pass over that queue
@@ -362,7 +363,7 @@ __device__ __forceinline__ void expand_phase(const Ctx& c, const Front& fr, cons
         for (uint32_t t0 = 0; t0 < total; t0 += 32) {
             // ---- phase A
             const uint32_t j = t0 + lane;
-            uint32_t nseg = 0, u = 0;
+            uint32_t nseg = 0, u = 0, ckb = 0, nck = 0, itv_all = 0;
             uint64_t segbase = 0;
             if (j < total) {
                 uint32_t lo = 0, hi = 31;  // owner lane: largest o with pre[o] <= j
@@ -403,13 +404,9 @@ __device__ __forceinline__ void expand_phase(const Ctx& c, const Front& fr, cons
                             const uint32_t mid = (lo + hi) >> 1;
                             if (c.hv_ids[mid] < u) lo = mid + 1; else hi = mid;
                         }
-                        const uint32_t b0 = c.hv_ptr[lo], b1 = c.hv_ptr[lo + 1];
-                        const uint32_t slot = atomicAdd(c.chunk_len, b1 - b0);
-                        for (uint32_t k = b0; k < b1; k++) {
-                            const uint64_t first = (uint64_t)(k - b0 + 1) * c.ck_c;
-                            c.chunkq[slot + k - b0] = ChunkEntry{c.ck_pos[k], u, c.ck_prev[k],
-                                                                 (uint32_t)(itv - first < c.ck_c ? itv - first : c.ck_c), 0};
-                        }
+                        ckb = c.hv_ptr[lo];  // chunks 1.. become phase-B tasks of this batch
+                        nck = c.hv_ptr[lo + 1] - ckb;
+                        itv_all = (uint32_t)itv;
                         itv_here = c.ck_c;
                         after = c.hv_after[lo];
                         if (!SEG) nres_ck = c.hv_rem[lo];
@@ -447,15 +444,18 @@ __device__ __forceinline__ void expand_phase(const Ctx& c, const Front& fr, cons
                     t.end();
                 }
             }
-            if (SEG) {
-                // ---- phase B: flatten the batch's segments and decode one per lane
-                uint32_t sincl = nseg;
+            if (SEG || c.hv_n) {
+                // ---- phase B: flatten the batch's tasks (interval chunks, then residual segments), one per lane
+                uint32_t sincl = nck + nseg;
                 for (int o = 1; o < 32; o <<= 1) {
                     const uint32_t tt = __shfl_up_sync(0xffffffffu, sincl, o);
                     if (lane >= (uint32_t)o) sincl += tt;
                 }
                 sm.u[lane] = u;
                 sm.base[lane] = segbase;
+                sm.ckb[lane] = ckb;
+                sm.nck[lane] = nck;
+                sm.itv[lane] = itv_all;
                 sm.spre[lane + 1] = sincl;
                 if (lane == 0) sm.spre[0] = 0;
                 __syncwarp();
@@ -468,10 +468,26 @@ __device__ __forceinline__ void expand_phase(const Ctx& c, const Front& fr, cons
                             const uint32_t mid = (lo + hi + 1) >> 1;
                             if (sm.spre[mid] <= sj) lo = mid; else hi = mid - 1;
                         }
-                        const uint32_t su = sm.u[lo];
+                        const uint32_t su = sm.u[lo], idx = sj - sm.spre[lo], snck = sm.nck[lo];
                         App t = app;
                         t.begin(su);
-                        na += decode_segment<K, STAGED>(c.W, sm.base[lo] + (uint64_t)(sj - sm.spre[lo]) * c.seg_bits, su, t);
+                        if (idx < snck) {  // interval chunk idx+1 of su: up to ck_c intervals from a checkpoint
+                            const uint32_t k = sm.ckb[lo] + idx;
+                            const uint32_t left = sm.itv[lo] - (idx + 1) * c.ck_c;
+                            const uint32_t cnt = left < c.ck_c ? left : c.ck_c;
+                            uint64_t p = c.ck_pos[k];
+                            uint32_t cur = c.ck_prev[k];
+                            for (uint32_t i = 0; i < cnt; i++) {
+                                const uint32_t g = (uint32_t)decode<K>(c.W, p);
+                                const uint32_t len = (uint32_t)(decode<K>(c.W, p) - 1) + c.min_len;
+                                t.range(cur + g, len);
+                                cur += g + len - 1;
+                                na += len;
+                            }
+                        } else {
+                            na += decode_segment<K, STAGED>(c.W, sm.base[lo] + (uint64_t)(idx - snck) * c.seg_bits,
+                                                            su, t);
+                        }
                         t.end();
                     }
                 }
@@ -1017,7 +1033,9 @@ __global__ void commit_dense(uint32_t* __restrict__ V, uint32_t* __restrict__ F,
 // Direction choice for the next BFS level (one thread; Beamer et al.'s heuristic on vertex counts): switch to
 // bottom-up when the new frontier is large against the unvisited set and growing, back to top-down when it is
 // small against n and shrinking.  st: [0] dir, [1] visited, [2] new-frontier count (consumed), [3] previous.
-__global__ void bfs_decide(uint32_t* st, uint64_t n, uint32_t alpha, uint32_t beta, int enabled) {
+__global__ void bfs_decide(uint32_t* st, uint64_t n, uint32_t alpha, uint32_t beta, int enabled,
+                           const uint32_t* qn_len, uint32_t* level_counter) {
+    if (*qn_len) *level_counter += 1;  // levels that produced a non-empty next frontier
     const uint64_t nf = st[2];
     st[2] = 0;
     const uint64_t visited = (uint64_t)st[1] + nf;
@@ -1164,51 +1182,6 @@ __global__ void __launch_bounds__(kBlock, 4) bfs_persistent(Ctx c, BfsPersist b)
     }
     add_stats(c.st, nv, na, nb);
     if (blockIdx.x == 0 && threadIdx.x == 0) b.ctr[6] = level + 1;
-}
-
-// Counts expanded levels on the device: a level that produced a non-empty next queue adds one.
-__global__ void count_level(const uint32_t* qn_len, uint32_t* counter) {
-    if (*qn_len) *counter += 1;
-}
-
-// ---- partitioned BFS / CC steps (the collectives run in the caller, e.g. torch.distributed over NCCL) ------------
-// Contraction of the owned slice: OR of the P candidate slices received from every rank, minus visited; writes
-// levels and the owned next-frontier slice; counts new vertices.
-__global__ void dist_commit(const uint32_t* __restrict__ recv, uint32_t P, uint64_t w_lo, uint64_t nlw,
-                            const uint32_t* __restrict__ V, uint32_t* __restrict__ fslice, int32_t* __restrict__ levels,
-                            int32_t new_level, uint64_t n, unsigned long long* __restrict__ count) {
-    const uint32_t lane = lane_id();
-    uint32_t nf = 0;
-    const uint64_t gw = ((uint64_t)blockIdx.x * blockDim.x + threadIdx.x) >> 5;
-    const uint64_t nwarps = ((uint64_t)gridDim.x * blockDim.x) >> 5;
-    for (uint64_t base = gw * 32; base < nlw; base += nwarps * 32) {
-        const uint64_t i = base + lane;
-        uint32_t b = 0;
-        if (i < nlw) {
-            for (uint32_t r = 0; r < P; r++) b |= recv[(uint64_t)r * nlw + i];
-            b &= ~V[w_lo + i];
-            fslice[i] = b;
-        }
-        nf += __popc(b);
-        for (uint32_t m = __ballot_sync(0xffffffffu, b != 0); m; m &= m - 1) {  // coalesced level stores
-            const int j = __ffs(m) - 1;
-            const uint32_t bj = __shfl_sync(0xffffffffu, b, j);
-            const uint64_t v = (w_lo + base + j) * 32 + lane;
-            if (((bj >> lane) & 1u) && v < n) levels[v] = new_level;
-        }
-    }
-    for (int o = 16; o; o >>= 1) nf += __shfl_xor_sync(0xffffffffu, nf, o);
-    if (lane == 0 && nf) atomicAdd(count, (unsigned long long)nf);
-}
-
-// F = the gathered global frontier; V |= F.
-__global__ void dist_absorb(const uint32_t* __restrict__ Fg, uint32_t* __restrict__ F, uint32_t* __restrict__ V,
-                            uint64_t nw) {
-    for (uint64_t w = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; w < nw; w += (uint64_t)gridDim.x * blockDim.x) {
-        const uint32_t b = Fg[w];
-        F[w] = b;
-        V[w] |= b;
-    }
 }
 
 __global__ void bfs_seed(uint32_t s, uint32_t* V, uint32_t* F, uint32_t* q, uint32_t* qlen, uint32_t* qbits,
@@ -1968,8 +1941,8 @@ extern "C" gcgt_status gcgt_bfs(gcgt_graph* g, uint32_t source, int32_t* levels,
                                                                  nullptr, g->ctr + cur, g->hub_ctr, g->heavy_len,
                                                                  g->levels, (int32_t)level + 1, g->bstate + 2,
                                                                  g->chunk_len);
-            bfs_decide<<<1, 1, 0, s>>>(g->bstate, g->n, g->bu_alpha, g->bu_beta, g->dir_opt ? 1 : 0);
-            count_level<<<1, 1, 0, s>>>(g->ctr + nxt, g->ctr + 6);
+            bfs_decide<<<1, 1, 0, s>>>(g->bstate, g->n, g->bu_alpha, g->bu_beta, g->dir_opt ? 1 : 0, g->ctr + nxt,
+                                       g->ctr + 6);
             if (g->profile) {  // profiling waits per level anyway (nlev = 1)
                 CU(cudaEventRecord(g->sev[4], s));
                 CU(cudaEventSynchronize(g->sev[4]));
@@ -1979,7 +1952,7 @@ extern "C" gcgt_status gcgt_bfs(gcgt_graph* g, uint32_t source, int32_t* levels,
                     g->span_ms[k] += ms;
                 }
             }
-            g->launches += 4 + (g->P.residual_segment_len ? 1 : 0) + (g->dir_opt ? 1 : 0) + (heavy_active(g) ? 1 : 0);
+            g->launches += 3 + (g->P.residual_segment_len ? 1 : 0) + (g->dir_opt ? 1 : 0) + (heavy_active(g) ? 1 : 0);
         }
         CU(cudaMemcpyAsync(g->h_ctr + 6, g->ctr + 6, 4, cudaMemcpyDeviceToHost, s));
         CU(cudaMemcpyAsync(g->h_ctr + (level & 1), g->ctr + (level & 1), 4, cudaMemcpyDeviceToHost, s));
