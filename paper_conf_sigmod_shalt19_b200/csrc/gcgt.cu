@@ -98,7 +98,7 @@ struct gcgt_graph {
     bool in_owned = false;       // inW / inOffs are separate allocations
     bool dir_opt = false;        // direction-optimizing BFS enabled (in-CGR available)
     // interval checkpoint table (derived at load) + per-level chunk queue
-    uint32_t hv_n = 0, ck_c = 8;
+    uint32_t hv_n = 0, ck_c = 4;
     uint32_t *hv_ids = nullptr, *hv_ptr = nullptr, *hv_rem = nullptr, *ck_prev = nullptr, *chunk_len = nullptr;
     uint64_t *hv_after = nullptr, *ck_pos = nullptr;
     ChunkEntry* chunkq = nullptr;
@@ -1182,6 +1182,46 @@ __global__ void __launch_bounds__(kBlock, 4) bfs_persistent(Ctx c, BfsPersist b)
     }
     add_stats(c.st, nv, na, nb);
     if (blockIdx.x == 0 && threadIdx.x == 0) b.ctr[6] = level + 1;
+}
+
+// ---- partitioned BFS / CC steps (the collectives run in the caller, e.g. torch.distributed over NCCL) ------------
+// Contraction of the owned slice: OR of the P candidate slices received from every rank, minus visited; writes
+// levels and the owned next-frontier slice; counts new vertices.
+__global__ void dist_commit(const uint32_t* __restrict__ recv, uint32_t P, uint64_t w_lo, uint64_t nlw,
+                            const uint32_t* __restrict__ V, uint32_t* __restrict__ fslice, int32_t* __restrict__ levels,
+                            int32_t new_level, uint64_t n, unsigned long long* __restrict__ count) {
+    const uint32_t lane = lane_id();
+    uint32_t nf = 0;
+    const uint64_t gw = ((uint64_t)blockIdx.x * blockDim.x + threadIdx.x) >> 5;
+    const uint64_t nwarps = ((uint64_t)gridDim.x * blockDim.x) >> 5;
+    for (uint64_t base = gw * 32; base < nlw; base += nwarps * 32) {
+        const uint64_t i = base + lane;
+        uint32_t b = 0;
+        if (i < nlw) {
+            for (uint32_t r = 0; r < P; r++) b |= recv[(uint64_t)r * nlw + i];
+            b &= ~V[w_lo + i];
+            fslice[i] = b;
+        }
+        nf += __popc(b);
+        for (uint32_t m = __ballot_sync(0xffffffffu, b != 0); m; m &= m - 1) {  // coalesced level stores
+            const int j = __ffs(m) - 1;
+            const uint32_t bj = __shfl_sync(0xffffffffu, b, j);
+            const uint64_t v = (w_lo + base + j) * 32 + lane;
+            if (((bj >> lane) & 1u) && v < n) levels[v] = new_level;
+        }
+    }
+    for (int o = 16; o; o >>= 1) nf += __shfl_xor_sync(0xffffffffu, nf, o);
+    if (lane == 0 && nf) atomicAdd(count, (unsigned long long)nf);
+}
+
+// F = the gathered global frontier; V |= F.
+__global__ void dist_absorb(const uint32_t* __restrict__ Fg, uint32_t* __restrict__ F, uint32_t* __restrict__ V,
+                            uint64_t nw) {
+    for (uint64_t w = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; w < nw; w += (uint64_t)gridDim.x * blockDim.x) {
+        const uint32_t b = Fg[w];
+        F[w] = b;
+        V[w] |= b;
+    }
 }
 
 __global__ void bfs_seed(uint32_t s, uint32_t* V, uint32_t* F, uint32_t* q, uint32_t* qlen, uint32_t* qbits,
