@@ -1081,50 +1081,58 @@ __global__ void __launch_bounds__(kBlock) bu_kernel(const uint64_t* __restrict__
         if (!unv) continue;
         bool found = false;
         if ((unv >> lane) & 1u) {
+            // BitBuf decoding: this kernel is instruction-bound (long in-record scans at high lane utilisation), so
+            // the cheaper 32-bit refill decoder pays off here (unlike the latency-bound top-down kernel)
             const uint32_t v = (uint32_t)(v0 + lane);
             const uint64_t p0 = ldg64(offs + v);
-            uint64_t p = p0;
+            BitBuf bb;
+            bb.init(W, p0);
             nv++;
-            uint64_t deg = 0, got = 0;
-            if (!SEG) deg = decode<K>(W, p) - 1;
-            const uint64_t itv = decode<K>(W, p) - 1;
-            int64_t prev_end = 0;
+            uint64_t deg = 0, got = 0, pend = p0;
+            if (!SEG) deg = bb.template next<K>(W) - 1;
+            const uint64_t itv = bb.template next<K>(W) - 1;
+            uint32_t prev_end = 0;
             for (uint64_t i = 0; i < itv && !found; i++) {
-                const uint64_t g = decode<K>(W, p);
-                const uint64_t len = decode<K>(W, p) - 1 + min_len;
-                const int64_t start = i == 0 ? unmap_first(v, g) : prev_end + (int64_t)g;
-                found = frontier_range(F, (uint32_t)start, (uint32_t)len);
-                prev_end = start + (int64_t)len - 1;
+                const uint64_t g = bb.template next<K>(W);
+                const uint32_t len = (uint32_t)(bb.template next<K>(W) - 1) + min_len;
+                const uint32_t start = i == 0 ? (uint32_t)unmap_first(v, g) : prev_end + (uint32_t)g;
+                found = frontier_range(F, start, len);
+                prev_end = start + len - 1;
                 got += len;
             }
             if (!found) {
                 if (!SEG) {
                     const uint64_t nres = deg - got;
-                    int64_t cur = 0;
+                    uint32_t cur = 0;
                     for (uint64_t i = 0; i < nres && !found; i++) {
-                        const uint64_t c = decode<K>(W, p);
-                        cur = i == 0 ? unmap_first(v, c) : cur + (int64_t)c;
+                        const uint64_t c = bb.template next<K>(W);
+                        cur = i == 0 ? (uint32_t)unmap_first(v, c) : cur + (uint32_t)c;
                         found = (__ldg(F + (cur >> 5)) >> (cur & 31)) & 1u;
                         got++;
                     }
+                    pend = bb.pos();
                 } else {
-                    const uint64_t nseg = decode<K>(W, p) - 1;
-                    const uint64_t base = p;
+                    const uint64_t nseg = bb.template next<K>(W) - 1;
+                    const uint64_t base = bb.pos();
+                    pend = base;
                     for (uint64_t sg = 0; sg < nseg && !found; sg++) {
-                        p = base + sg * seg_bits;
-                        const uint64_t cnt = decode<K>(W, p) - 1;
-                        int64_t cur = 0;
-                        for (uint64_t i = 0; i < cnt && !found; i++) {
-                            const uint64_t c = decode<K>(W, p);
-                            cur = i == 0 ? unmap_first(v, c) : cur + (int64_t)c;
+                        bb.init(W, base + sg * seg_bits);
+                        const uint32_t cnt = (uint32_t)(bb.template next<K>(W) - 1);
+                        uint32_t cur = 0;
+                        for (uint32_t i = 0; i < cnt && !found; i++) {
+                            const uint64_t c = bb.template next<K>(W);
+                            cur = i == 0 ? (uint32_t)unmap_first(v, c) : cur + (uint32_t)c;
                             found = (__ldg(F + (cur >> 5)) >> (cur & 31)) & 1u;
                             got++;
                         }
+                        pend = bb.pos();
                     }
                 }
+            } else {
+                pend = bb.pos();
             }
             na += got;
-            nb += p - p0;
+            nb += pend - p0;
         }
         const uint32_t fb = __ballot_sync(0xffffffffu, found);
         if (lane == 0 && fb) N[w] = fb;
