@@ -13,6 +13,7 @@
 // backward delta (Fig. 7(d), Brandes [9]).
 #include <cuda_runtime.h>
 #include <cooperative_groups.h>
+#include <cooperative_groups/reduce.h>
 #include <cub/cub.cuh>
 #include <stdio.h>
 #include <string.h>
@@ -899,9 +900,14 @@ struct BcBwdApp {
         for (uint32_t t = 0; t < len; t++) one(s + t);
     }
     __device__ __forceinline__ void end() {
-        if (acc != 0.0) {
-            atomicAdd(delta + u, acc);
-            if (u != source) atomicAdd(bc + u, acc);
+        // lanes finishing tasks of the same vertex (a hub's segments sit side by side in the hub queue) first sum
+        // their partials, so a vertex with 10^5 segments does not serialise 10^5 fp64 atomics on one address
+        cg::coalesced_group act = cg::coalesced_threads();
+        cg::coalesced_group same = cg::labeled_partition(act, u);
+        const double sum = cg::reduce(same, acc, cg::plus<double>());
+        if (same.thread_rank() == 0 && sum != 0.0) {
+            atomicAdd(delta + u, sum);
+            if (u != source) atomicAdd(bc + u, sum);
         }
     }
 };
