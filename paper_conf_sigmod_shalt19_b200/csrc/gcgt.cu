@@ -65,14 +65,11 @@ struct HubEntry {
     uint32_t seg_off;  // first flattened segment index of this entry (entries are ordered by seg_off)
 };
 
-// An interval chunk of a vertex with a long interval area: `count` intervals starting with the gap code at bit
-// `pos`, the previous interval having ended at `prev_end` (load-time checkpoint table, see build_checkpoints).
-struct ChunkEntry {
-    uint64_t pos;
-    uint32_t u;
-    uint32_t prev_end;
-    uint32_t count;
-    uint32_t pad;
+// A long interval (more than long_len ids) deferred to the level's long-range queue and expanded grid-wide in chunks
+// of lr_chunk ids: the Two-Phase Traversal's "long interval expanded by the whole thread group" (Alg. 2 l.23-32,
+// PAPER.md:667-688) at grid scale.  Entries are ordered by chunk_off (one packed atomic hands out both indices).
+struct LongRange {
+    uint32_t u, start, len, chunk_off;
 };
 
 struct HeavyEntry {
@@ -100,9 +97,11 @@ struct gcgt_graph {
     bool dir_opt = false;        // direction-optimizing BFS enabled (in-CGR available)
     // interval checkpoint table (derived at load) + per-level chunk queue
     uint32_t hv_n = 0, ck_c = 4;
-    uint32_t *hv_ids = nullptr, *hv_ptr = nullptr, *hv_rem = nullptr, *ck_prev = nullptr, *chunk_len = nullptr;
+    uint32_t *hv_ids = nullptr, *hv_ptr = nullptr, *hv_rem = nullptr, *ck_prev = nullptr;
     uint64_t *hv_after = nullptr, *ck_pos = nullptr;
-    ChunkEntry* chunkq = nullptr;
+    LongRange* lrq = nullptr;              // per-level long-range queue
+    unsigned long long* lr_ctr = nullptr;  // (entries << 32) | chunks
+    uint32_t long_len = 1024, lr_chunk = 256;
     uint32_t* bstate = nullptr;  // BFS direction state [8]: 0 dir (0 TD, 1 BU), 1 visited, 2 new-frontier count,
                                  // 3 previous frontier count
     // work
@@ -179,8 +178,9 @@ struct Ctx {
     const uint32_t* __restrict__ hv_rem;    // unsegmented records: residual count
     const uint64_t* __restrict__ ck_pos;
     const uint32_t* __restrict__ ck_prev;
-    ChunkEntry* chunkq;
-    uint32_t* chunk_len;
+    LongRange* lrq;
+    unsigned long long* lr_ctr;
+    uint32_t long_len, lr_chunk;
 };
 
 __device__ __forceinline__ void add_stats(Stats* st, uint64_t v, uint64_t a, uint64_t b) {
@@ -255,6 +255,18 @@ struct DenseFront {
 // One residual segment (FORMAT.md R17): count, first residual anchored at u, then gaps.  Returns the count.
 // The segment's bits are staged in registers (RegStream) and the neighbour ids are handed to the filter four at a
 // time (App::many), so their visited-bitmap probes are in flight together.
+// Interval hand-off: short intervals go to the filter directly; long ones to the level's long-range queue.
+template <class App>
+__device__ __forceinline__ void range_or_defer(const Ctx& c, App& t, uint32_t u, uint32_t start, uint32_t len) {
+    if (len <= c.long_len || !c.lr_ctr) {
+        t.range(start, len);
+        return;
+    }
+    const uint32_t nch = (len + c.lr_chunk - 1) / c.lr_chunk;
+    const unsigned long long old = atomicAdd(c.lr_ctr, (1ull << 32) | (unsigned long long)nch);
+    c.lrq[old >> 32] = LongRange{u, start, len, (uint32_t)(old & 0xffffffffu)};
+}
+
 // Per-codeword global-window reader (the unstaged alternative to RegStream; same interface).
 struct WinStream {
     const uint64_t* __restrict__ W;
@@ -417,7 +429,7 @@ __device__ __forceinline__ void expand_phase(const Ctx& c, const Front& fr, cons
                         const uint64_t g = rs.template next<K>();
                         const uint64_t len = rs.template next<K>() - 1 + c.min_len;
                         const int64_t start = i == 0 ? unmap_first(u, g) : prev_end + (int64_t)g;
-                        t.range((uint32_t)start, (uint32_t)len);
+                        range_or_defer(c, t, u, (uint32_t)start, (uint32_t)len);
                         prev_end = start + (int64_t)len - 1;
                         in_itv += len;
                     }
@@ -481,7 +493,7 @@ __device__ __forceinline__ void expand_phase(const Ctx& c, const Front& fr, cons
                             for (uint32_t i = 0; i < cnt; i++) {
                                 const uint32_t g = (uint32_t)decode<K>(c.W, p);
                                 const uint32_t len = (uint32_t)(decode<K>(c.W, p) - 1) + c.min_len;
-                                t.range(cur + g, len);
+                                range_or_defer(c, t, su, cur + g, len);
                                 cur += g + len - 1;
                                 na += len;
                             }
@@ -756,23 +768,21 @@ __global__ void __launch_bounds__(kBlock, 4) sm_expand_kernel(Ctx c, Front fr, A
 // Hub segments of the level, flattened over the whole grid (one segment per thread at a time).
 template <int K, bool STAGED, class App>
 __device__ __forceinline__ void hub_phase(const Ctx& c, const App& app, uint64_t& na) {
-    if (c.chunk_len) {  // interval chunks of long interval areas: one chunk per thread
-        const uint32_t nck = *(volatile uint32_t*)c.chunk_len;
-        for (uint64_t j = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; j < nck;
+    if (c.lr_ctr) {  // long intervals: one lr_chunk-id piece per thread
+        const unsigned long long lc = *(volatile unsigned long long*)c.lr_ctr;
+        const uint32_t ne = (uint32_t)(lc >> 32), nchunks = (uint32_t)(lc & 0xffffffffu);
+        for (uint64_t j = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; j < nchunks;
              j += (uint64_t)gridDim.x * blockDim.x) {
-            const ChunkEntry e = c.chunkq[j];
+            uint32_t lo = 0, hi = ne - 1;
+            while (lo < hi) {
+                const uint32_t mid = (lo + hi + 1) >> 1;
+                if (c.lrq[mid].chunk_off <= j) lo = mid; else hi = mid - 1;
+            }
+            const LongRange e = c.lrq[lo];
+            const uint32_t off = (uint32_t)(j - e.chunk_off) * c.lr_chunk;
             App t = app;
             t.begin(e.u);
-            uint64_t p = e.pos;
-            uint32_t cur = e.prev_end;
-            for (uint32_t i = 0; i < e.count; i++) {
-                const uint32_t g = (uint32_t)decode<K>(c.W, p);
-                const uint32_t len = (uint32_t)(decode<K>(c.W, p) - 1) + c.min_len;
-                const uint32_t start = cur + g;
-                t.range(start, len);
-                cur = start + len - 1;
-                na += len;
-            }
+            t.range(e.start + off, min(c.lr_chunk, e.len - off));
             t.end();
         }
     }
@@ -1026,13 +1036,14 @@ __global__ void commit_dense(uint32_t* __restrict__ V, uint32_t* __restrict__ F,
                              uint32_t* __restrict__ qbits_out, uint32_t* __restrict__ reset_ctr,
                              unsigned long long* __restrict__ hub_ctr, uint32_t* __restrict__ heavy_len,
                              int32_t* __restrict__ levels = nullptr, int32_t new_level = 0,
-                             uint32_t* __restrict__ nf_count = nullptr, uint32_t* __restrict__ chunk_len = nullptr) {
+                             uint32_t* __restrict__ nf_count = nullptr,
+                             unsigned long long* __restrict__ lr_ctr = nullptr) {
     commit_phase(V, F, N, w_lo, w_hi, qn, qn_len, qbits_out, levels, new_level, nf_count);
     if (blockIdx.x == 0 && threadIdx.x == 0) {
         if (reset_ctr) *reset_ctr = 0;
         if (hub_ctr) *hub_ctr = 0;
         if (heavy_len) *heavy_len = 0;
-        if (chunk_len) *chunk_len = 0;
+        if (lr_ctr) *lr_ctr = 0;
     }
 }
 
@@ -1180,7 +1191,7 @@ __global__ void __launch_bounds__(kBlock, 4) bfs_persistent(Ctx c, BfsPersist b)
         const BfsApp app{b.V, b.N, b.levels, (int32_t)level};
         expand_phase<K, SEG, BfsApp, QueueFront, true, false>(c, fr, app, (uint32_t)wpb, smem, nv, na, nb);
         grid.sync();
-        if (SEG || c.hv_n) {
+        if (SEG || c.hv_n || c.lr_ctr) {
             hub_phase<K, false>(c, app, na);
             grid.sync();
         }
@@ -1188,7 +1199,7 @@ __global__ void __launch_bounds__(kBlock, 4) bfs_persistent(Ctx c, BfsPersist b)
         if (blockIdx.x == 0 && threadIdx.x == 0) {
             b.ctr[cur] = 0;
             *c.hub_ctr = 0;
-            if (c.chunk_len) *c.chunk_len = 0;
+            if (c.lr_ctr) *c.lr_ctr = 0;
             c.cursor[0] = 0;
         }
         grid.sync();
@@ -1319,8 +1330,8 @@ __global__ void ck_fill(const uint64_t* __restrict__ W, const uint64_t* __restri
 template <int K, bool SEG>
 __global__ void count_special(const uint64_t* __restrict__ W, const uint64_t* __restrict__ offs, uint64_t lo,
                               uint64_t n, uint32_t heavy_itv, uint32_t heavy_res, uint32_t hub_segs,
-                              unsigned long long* out) {
-    uint32_t hubs = 0, heavy = 0;
+                              uint32_t min_len, uint32_t long_len, unsigned long long* out) {
+    uint32_t hubs = 0, heavy = 0, longs = 0;
     for (uint64_t u = lo + (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; u < n;
          u += (uint64_t)gridDim.x * blockDim.x) {
         uint64_t p = ldg64(offs + u);
@@ -1328,18 +1339,21 @@ __global__ void count_special(const uint64_t* __restrict__ W, const uint64_t* __
         if (!SEG) deg = decode<K>(W, p) - 1;
         const uint64_t itv = decode<K>(W, p) - 1;
         if (itv > heavy_itv || (!SEG && deg > heavy_res)) heavy++;
-        if (SEG) {
-            for (uint64_t i = 0; i < 2 * itv; i++) decode<K>(W, p);
-            if (decode<K>(W, p) - 1 > hub_segs) hubs++;
+        for (uint64_t i = 0; i < itv; i++) {
+            decode<K>(W, p);
+            if (decode<K>(W, p) - 1 + min_len > long_len) longs++;
         }
+        if (SEG && decode<K>(W, p) - 1 > hub_segs) hubs++;
     }
     for (int o = 16; o; o >>= 1) {
         hubs += __shfl_xor_sync(0xffffffffu, hubs, o);
         heavy += __shfl_xor_sync(0xffffffffu, heavy, o);
+        longs += __shfl_xor_sync(0xffffffffu, longs, o);
     }
     if (lane_id() == 0) {
         if (hubs) atomicAdd(out, (unsigned long long)hubs);
         if (heavy) atomicAdd(out + 1, (unsigned long long)heavy);
+        if (longs) atomicAdd(out + 2, (unsigned long long)longs);
     }
 }
 
@@ -1459,7 +1473,7 @@ inline void launch_bu(const gcgt_graph* g, cudaStream_t s) {
 
 template <class App>
 inline void launch_hub(const gcgt_params& P, bool staged, int grid, cudaStream_t s, const Ctx& c, const App& app) {
-    if (!P.residual_segment_len && !c.hv_n) return;
+    if (!P.residual_segment_len && !c.hv_n && !c.lr_ctr) return;
 #define GCGT_HUB(KK)                                                            \
     (staged ? hub_kernel<KK, true, App><<<grid, kBlock, 0, s>>>(c, app)         \
             : hub_kernel<KK, false, App><<<grid, kBlock, 0, s>>>(c, app))
@@ -1495,7 +1509,7 @@ inline Ctx make_ctx(const gcgt_graph* g) {
                g->hubq, g->hub_ctr, g->stats,              g->cursor,
                g->heavyq, g->heavy_len, g->heavy_itv, g->heavy_res, g->hub_segs, g->engine, nullptr,
                g->hv_n,  g->ck_c,      g->hv_ids,    g->hv_ptr,    g->hv_after, g->hv_rem, g->ck_pos, g->ck_prev,
-               g->chunkq, g->chunk_len};
+               g->lrq,   g->lr_ctr,    g->long_len,  g->lr_chunk};
 }
 
 gcgt_status copy_out(gcgt_graph* g, void* dst, const void* src, size_t bytes, int placement) {
@@ -1577,8 +1591,8 @@ gcgt_status galloc(const gcgt_graph* g, T** p, uint64_t count) {
 // Builds the interval checkpoint table (see ck_count / ck_fill) and the per-level chunk queue.
 gcgt_status build_checkpoints(gcgt_graph* g) {
     gcgt_status st;
-    if ((st = galloc(g, &g->chunk_len, 1))) return st;
-    CU(cudaMemsetAsync(g->chunk_len, 0, 4, g->stream));
+    if ((st = galloc(g, &g->lr_ctr, 1))) return st;
+    CU(cudaMemsetAsync(g->lr_ctr, 0, 8, g->stream));
     if (g->ck_c == 0xFFFFFFFFu || g->hi == g->lo) return GCGT_OK;
     cudaStream_t s = g->stream;
     const bool seg = g->P.residual_segment_len != 0;
@@ -1624,8 +1638,7 @@ gcgt_status build_checkpoints(gcgt_graph* g) {
         uint32_t T = 0;
         CU(cudaMemcpyAsync(&T, g->hv_ptr + H, 4, cudaMemcpyDeviceToHost, s));
         CU(cudaStreamSynchronize(s));
-        if ((st = galloc(g, &g->ck_pos, (uint64_t)T + 1)) || (st = galloc(g, &g->ck_prev, (uint64_t)T + 1)) ||
-            (st = galloc(g, &g->chunkq, (uint64_t)T + 1)))
+        if ((st = galloc(g, &g->ck_pos, (uint64_t)T + 1)) || (st = galloc(g, &g->ck_prev, (uint64_t)T + 1)))
             return st;
         const int gh = flat_grid(g, H);
 #define GCGT_CF(KK)                                                                                                  \
@@ -1662,7 +1675,7 @@ extern "C" void gcgt_unload(gcgt_graph* g) {
     void* bufs[] = {g->W,      g->offs_alloc, g->V,      g->F,         g->N,        g->q,      g->qbits,
                     g->ctr,    g->hubq,    g->hub_ctr, g->cursor,   g->heavyq,   g->heavy_len, g->stats,
                     g->levels, g->parent,  g->sigma,  g->delta,     g->bc,      g->bstate,
-                    g->hv_ids, g->hv_ptr,  g->hv_rem, g->ck_prev,   g->chunk_len, g->hv_after, g->ck_pos, g->chunkq,
+                    g->hv_ids, g->hv_ptr,  g->hv_rem, g->ck_prev,   g->lr_ctr, g->hv_after, g->ck_pos, g->lrq,
                     g->in_owned ? g->inW : nullptr, g->in_owned ? g->inOffs : nullptr};
     if (g->stream) {
         for (void* b : bufs)
@@ -1730,6 +1743,7 @@ extern "C" gcgt_status gcgt_load(const gcgt_cgr* c, const gcgt_load_opts* opts, 
                 else if (k == "heavy_itv") g->heavy_itv = (uint32_t)v;
                 else if (k == "heavy_res") g->heavy_res = (uint32_t)v;
                 else if (k == "hub_segs") g->hub_segs = (uint32_t)v;
+                else if (k == "long_len") g->long_len = (uint32_t)std::max(32ul, v);
                 else if (k == "wpb_max") g->wpb_max = (uint32_t)std::max(1ul, std::min(32ul, v));
             }
             i = j + 1;
@@ -1814,29 +1828,30 @@ extern "C" gcgt_status gcgt_load(const gcgt_cgr* c, const gcgt_load_opts* opts, 
     if ((st = galloc(g.get(), &g->hub_ctr, 1)) || (st = galloc(g.get(), &g->cursor, 2))) return st;
     CU(cudaMemsetAsync(g->cursor, 0, 16, g->stream));
     unsigned long long* dcount = nullptr;
-    if ((st = galloc(g.get(), &dcount, 2))) return st;
-    CU(cudaMemsetAsync(dcount, 0, 16, g->stream));
+    if ((st = galloc(g.get(), &dcount, 3))) return st;
+    CU(cudaMemsetAsync(dcount, 0, 24, g->stream));
     {
         const int gr = flat_grid(g.get(), g->n);
         const bool seg = g->P.residual_segment_len != 0;
         cudaStream_t s = g->stream;
         switch (g->P.zeta_k) {
-            case 1: seg ? count_special<1, true><<<gr, kBlock, 0, s>>>(g->W, g->offs, g->lo, g->hi, g->heavy_itv, g->heavy_res, g->hub_segs, dcount) : count_special<1, false><<<gr, kBlock, 0, s>>>(g->W, g->offs, g->lo, g->hi, g->heavy_itv, g->heavy_res, g->hub_segs, dcount); break;
-            case 2: seg ? count_special<2, true><<<gr, kBlock, 0, s>>>(g->W, g->offs, g->lo, g->hi, g->heavy_itv, g->heavy_res, g->hub_segs, dcount) : count_special<2, false><<<gr, kBlock, 0, s>>>(g->W, g->offs, g->lo, g->hi, g->heavy_itv, g->heavy_res, g->hub_segs, dcount); break;
-            case 3: seg ? count_special<3, true><<<gr, kBlock, 0, s>>>(g->W, g->offs, g->lo, g->hi, g->heavy_itv, g->heavy_res, g->hub_segs, dcount) : count_special<3, false><<<gr, kBlock, 0, s>>>(g->W, g->offs, g->lo, g->hi, g->heavy_itv, g->heavy_res, g->hub_segs, dcount); break;
-            case 4: seg ? count_special<4, true><<<gr, kBlock, 0, s>>>(g->W, g->offs, g->lo, g->hi, g->heavy_itv, g->heavy_res, g->hub_segs, dcount) : count_special<4, false><<<gr, kBlock, 0, s>>>(g->W, g->offs, g->lo, g->hi, g->heavy_itv, g->heavy_res, g->hub_segs, dcount); break;
-            default: seg ? count_special<5, true><<<gr, kBlock, 0, s>>>(g->W, g->offs, g->lo, g->hi, g->heavy_itv, g->heavy_res, g->hub_segs, dcount) : count_special<5, false><<<gr, kBlock, 0, s>>>(g->W, g->offs, g->lo, g->hi, g->heavy_itv, g->heavy_res, g->hub_segs, dcount); break;
+            case 1: seg ? count_special<1, true><<<gr, kBlock, 0, s>>>(g->W, g->offs, g->lo, g->hi, g->heavy_itv, g->heavy_res, g->hub_segs, g->P.min_interval_len, g->long_len, dcount) : count_special<1, false><<<gr, kBlock, 0, s>>>(g->W, g->offs, g->lo, g->hi, g->heavy_itv, g->heavy_res, g->hub_segs, g->P.min_interval_len, g->long_len, dcount); break;
+            case 2: seg ? count_special<2, true><<<gr, kBlock, 0, s>>>(g->W, g->offs, g->lo, g->hi, g->heavy_itv, g->heavy_res, g->hub_segs, g->P.min_interval_len, g->long_len, dcount) : count_special<2, false><<<gr, kBlock, 0, s>>>(g->W, g->offs, g->lo, g->hi, g->heavy_itv, g->heavy_res, g->hub_segs, g->P.min_interval_len, g->long_len, dcount); break;
+            case 3: seg ? count_special<3, true><<<gr, kBlock, 0, s>>>(g->W, g->offs, g->lo, g->hi, g->heavy_itv, g->heavy_res, g->hub_segs, g->P.min_interval_len, g->long_len, dcount) : count_special<3, false><<<gr, kBlock, 0, s>>>(g->W, g->offs, g->lo, g->hi, g->heavy_itv, g->heavy_res, g->hub_segs, g->P.min_interval_len, g->long_len, dcount); break;
+            case 4: seg ? count_special<4, true><<<gr, kBlock, 0, s>>>(g->W, g->offs, g->lo, g->hi, g->heavy_itv, g->heavy_res, g->hub_segs, g->P.min_interval_len, g->long_len, dcount) : count_special<4, false><<<gr, kBlock, 0, s>>>(g->W, g->offs, g->lo, g->hi, g->heavy_itv, g->heavy_res, g->hub_segs, g->P.min_interval_len, g->long_len, dcount); break;
+            default: seg ? count_special<5, true><<<gr, kBlock, 0, s>>>(g->W, g->offs, g->lo, g->hi, g->heavy_itv, g->heavy_res, g->hub_segs, g->P.min_interval_len, g->long_len, dcount) : count_special<5, false><<<gr, kBlock, 0, s>>>(g->W, g->offs, g->lo, g->hi, g->heavy_itv, g->heavy_res, g->hub_segs, g->P.min_interval_len, g->long_len, dcount); break;
         }
     }
-    unsigned long long counts[2] = {0, 0};
-    CU(cudaMemcpyAsync(counts, dcount, 16, cudaMemcpyDeviceToHost, g->stream));
+    unsigned long long counts[3] = {0, 0, 0};
+    CU(cudaMemcpyAsync(counts, dcount, 24, cudaMemcpyDeviceToHost, g->stream));
     CU(cudaStreamSynchronize(g->stream));
     cudaFreeAsync(dcount, g->stream);
-    const uint64_t nhubs = counts[0], nheavy = counts[1];
+    const uint64_t nhubs = counts[0], nheavy = counts[1], nlong = counts[2];
     if ((st = galloc(g.get(), &g->heavyq, nheavy + 1)) || (st = galloc(g.get(), &g->heavy_len, 1))) return st;
     CU(cudaMemsetAsync(g->heavy_len, 0, 4, g->stream));
     if ((st = galloc(g.get(), &g->hubq, nhubs + nheavy + 1))) return st;
     if ((st = build_checkpoints(g.get()))) return st;
+    if ((st = galloc(g.get(), &g->lrq, nlong + 1))) return st;
     CU(cudaMemsetAsync(g->hub_ctr, 0, 8, g->stream));
     CU(cudaStreamSynchronize(g->stream));
     CU(cudaGetLastError());
@@ -1939,7 +1954,7 @@ extern "C" gcgt_status gcgt_bfs(gcgt_graph* g, uint32_t source, int32_t* levels,
     CU(cudaMemsetAsync(g->ctr, 0, 8 * 4, s));
     CU(cudaMemsetAsync(g->hub_ctr, 0, sizeof(unsigned long long), s));
     CU(cudaMemsetAsync(g->heavy_len, 0, 4, s));
-    CU(cudaMemsetAsync(g->chunk_len, 0, 4, s));
+    CU(cudaMemsetAsync(g->lr_ctr, 0, 8, s));
     uint32_t* q[2] = {g->q, g->q + g->nw};
     bfs_seed<<<1, 1, 0, s>>>(source, g->V, g->F, q[0], g->ctr + 0, nullptr, g->levels, g->bstate);
     g->launches = 1;
@@ -1994,7 +2009,7 @@ extern "C" gcgt_status gcgt_bfs(gcgt_graph* g, uint32_t source, int32_t* levels,
             commit_dense<<<flat_grid(g, g->nw), kBlock, 0, s>>>(g->V, g->F, g->N, 0, g->nw, q[nxt], g->ctr + nxt,
                                                                  nullptr, g->ctr + cur, g->hub_ctr, g->heavy_len,
                                                                  g->levels, (int32_t)level + 1, g->bstate + 2,
-                                                                 g->chunk_len);
+                                                                 g->lr_ctr);
             bfs_decide<<<1, 1, 0, s>>>(g->bstate, g->n, g->bu_alpha, g->bu_beta, g->dir_opt ? 1 : 0, g->ctr + nxt,
                                        g->ctr + 6);
             if (g->profile) {  // profiling waits per level anyway (nlev = 1)
@@ -2028,7 +2043,7 @@ extern "C" gcgt_status gcgt_cc(gcgt_graph* g, uint32_t* labels, int placement, g
     cudaStream_t s = g->stream;
     CU(cudaMemsetAsync(g->hub_ctr, 0, sizeof(unsigned long long), s));
     CU(cudaMemsetAsync(g->heavy_len, 0, 4, s));
-    CU(cudaMemsetAsync(g->chunk_len, 0, 4, s));
+    CU(cudaMemsetAsync(g->lr_ctr, 0, 8, s));
     cc_init<<<flat_grid(g, g->n), kBlock, 0, s>>>(g->parent, g->n);
     const Ctx c = make_ctx(g);
     const DenseFront fr{g->lo, g->hi};
@@ -2071,7 +2086,7 @@ extern "C" gcgt_status gcgt_bc(gcgt_graph* g, const uint32_t* sources, uint32_t 
     CU(cudaMemsetAsync(g->bc, 0, g->n * 8, s));
     CU(cudaMemsetAsync(g->hub_ctr, 0, sizeof(unsigned long long), s));
     CU(cudaMemsetAsync(g->heavy_len, 0, 4, s));
-    CU(cudaMemsetAsync(g->chunk_len, 0, 4, s));
+    CU(cudaMemsetAsync(g->lr_ctr, 0, 8, s));
     std::vector<uint32_t> lvl_off;
     for (uint32_t si = 0; si < k; si++) {
         const uint32_t src = sources[si];
@@ -2104,7 +2119,7 @@ extern "C" gcgt_status gcgt_bc(gcgt_graph* g, const uint32_t* sources, uint32_t 
             commit_dense<<<flat_grid(g, g->nw), kBlock, 0, s>>>(g->V, nullptr, g->N, 0, g->nw, g->q + total,
                                                                  g->ctr + 2 + ((level + 1) & 1), g->qbits + total,
                                                                  g->ctr + 2 + (level & 1), g->hub_ctr,
-                                                                 g->heavy_len, nullptr, 0, nullptr, g->chunk_len);
+                                                                 g->heavy_len, nullptr, 0, nullptr, g->lr_ctr);
             CU(cudaMemcpyAsync(g->h_ctr + 1, g->ctr + 2 + ((level + 1) & 1), 4, cudaMemcpyDeviceToHost, s));
             CU(cudaStreamSynchronize(s));
             if ((st = kprof_collect(g))) return st;
@@ -2125,7 +2140,7 @@ extern "C" gcgt_status gcgt_bc(gcgt_graph* g, const uint32_t* sources, uint32_t 
             launch_hub(g->P, g->staged, hub_grid(g), s, c, app);
             CU(cudaMemsetAsync(g->hub_ctr, 0, sizeof(unsigned long long), s));
             CU(cudaMemsetAsync(g->heavy_len, 0, 4, s));
-            CU(cudaMemsetAsync(g->chunk_len, 0, 4, s));
+            CU(cudaMemsetAsync(g->lr_ctr, 0, 8, s));
         }
     }
     if ((st = copy_out(g, bc, g->bc, g->n * 8, placement))) return st;
@@ -2154,7 +2169,7 @@ extern "C" gcgt_status gcgt_dist_bfs_begin(gcgt_graph* g, uint32_t source) {
     CU(cudaMemsetAsync(g->F, 0, g->nw * 4, s));
     CU(cudaMemsetAsync(g->levels, 0xff, g->n * 4, s));
     CU(cudaMemsetAsync(g->hub_ctr, 0, 8, s));
-    CU(cudaMemsetAsync(g->chunk_len, 0, 4, s));
+    CU(cudaMemsetAsync(g->lr_ctr, 0, 8, s));
     CU(cudaMemsetAsync(g->heavy_len, 0, 4, s));
     CU(cudaMemsetAsync(g->ctr, 0, 8 * 4, s));
     bfs_seed<<<1, 1, 0, s>>>(source, g->V, g->F, g->q, g->ctr, nullptr, g->levels, nullptr);
@@ -2177,7 +2192,7 @@ extern "C" gcgt_status gcgt_dist_bfs_expand(gcgt_graph* g, uint32_t level, uint3
     launch_heavy(g, s, c, app);
     launch_hub(g->P, g->staged, hub_grid(g), s, c, app);
     CU(cudaMemsetAsync(g->hub_ctr, 0, 8, s));
-    CU(cudaMemsetAsync(g->chunk_len, 0, 4, s));
+    CU(cudaMemsetAsync(g->lr_ctr, 0, 8, s));
     CU(cudaMemsetAsync(g->heavy_len, 0, 4, s));
     return dist_sync(g);
 }
@@ -2227,7 +2242,7 @@ extern "C" gcgt_status gcgt_dist_cc_hook(gcgt_graph* g, uint32_t* parent, uint64
     uint32_t* hc = g->ctr + 7;
     CU(cudaMemsetAsync(hc, 0, 4, s));
     CU(cudaMemsetAsync(g->hub_ctr, 0, 8, s));
-    CU(cudaMemsetAsync(g->chunk_len, 0, 4, s));
+    CU(cudaMemsetAsync(g->lr_ctr, 0, 8, s));
     CU(cudaMemsetAsync(g->heavy_len, 0, 4, s));
     const Ctx c = make_ctx(g);
     const DenseFront fr{g->lo, g->hi};
