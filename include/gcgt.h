@@ -113,6 +113,15 @@ typedef struct {
  * each rank keeps only the records of its owned vertex range (balanced by CGR bits; records are self-contained,
  * so slicing is a bit copy) plus replicated n-bit bitmaps.  opts may be NULL (device 0, own stream). */
 gcgt_status gcgt_load(const gcgt_cgr* cgr, const gcgt_load_opts* opts, gcgt_graph** out);
+
+/* Uncompressed baseline (§8 f3; the paper's GPUCSR comparison, Fig. 8 :1571-1578): copies a
+ * plain CSR (host, caller-owned; rows need not be sorted; ids < n < 2^32) to the device.  gcgt_bfs on the result
+ * runs the same frontier / filter / contraction / direction machinery as the CGR path with expansion reading
+ * col[] instead of decoding, so the time ratio is the decoding overhead.  With direction_optimizing the bottom-up
+ * in-lists are the transpose (built on the host) or, when `symmetric`, the CSR itself; opts->in_cgr is ignored.
+ * Single GPU only (nranks <= 1).  gcgt_cc / gcgt_bc / gcgt_dist_* return EINVAL on such a graph.
+ * stats->cgr_bits_decoded counts 32 bits per col[] entry read.  Errors: EINVAL, ERANGE (id >= n), ENOMEM, ECUDA. */
+gcgt_status gcgt_load_csr(const gcgt_csr* csr, const gcgt_load_opts* opts, gcgt_graph** out);
 void gcgt_unload(gcgt_graph* g);
 
 /* Enables (1) / disables (0) per-launch CUDA-event timing of the dominant kernel (fills gcgt_stats.kernel_ms).

@@ -22,7 +22,7 @@ OUT_HOST, OUT_DEVICE = 0, 1
 
 # public symbols of include/gcgt.h (tests check the library exports every one)
 ABI_SYMBOLS = ["gcgt_encode", "gcgt_encode_transpose", "gcgt_cgr_view", "gcgt_cgr_from_arrays", "gcgt_cgr_save", "gcgt_cgr_open",
-               "gcgt_cgr_free", "gcgt_load", "gcgt_unload", "gcgt_profile", "gcgt_profile_spans", "gcgt_graph_range", "gcgt_bfs", "gcgt_cc", "gcgt_bc",
+               "gcgt_cgr_free", "gcgt_load", "gcgt_load_csr", "gcgt_unload", "gcgt_profile", "gcgt_profile_spans", "gcgt_graph_range", "gcgt_bfs", "gcgt_cc", "gcgt_bc",
                "gcgt_dist_bfs_begin", "gcgt_dist_bfs_expand", "gcgt_dist_bfs_commit", "gcgt_dist_bfs_absorb",
                "gcgt_dist_bfs_levels", "gcgt_dist_cc_hook", "gcgt_dist_cc_jump",
                "gcgt_debug_warp_decode", "gcgt_last_error", "gcgt_version"]
@@ -77,6 +77,7 @@ def lib():
         L.gcgt_cgr_free.argtypes = [p]
         L.gcgt_cgr_free.restype = None
         L.gcgt_load.argtypes = [p, C.POINTER(LoadOpts), C.POINTER(p)]
+        L.gcgt_load_csr.argtypes = [C.POINTER(Csr), C.POINTER(LoadOpts), C.POINTER(p)]
         L.gcgt_unload.argtypes = [p]
         L.gcgt_unload.restype = None
         L.gcgt_profile.argtypes = [p, i32]
@@ -312,6 +313,30 @@ def cgr_n(cgr: CGR) -> int:
 
 def load(cgr: CGR, device: int = 0, stream=None, **kw) -> Graph:
     return Graph(cgr, device, stream, **kw)
+
+
+def load_csr(row_offsets: np.ndarray, cols: np.ndarray, device: int = 0, stream=None, symmetric: bool = False,
+             direction_optimizing: bool = True) -> Graph:
+    """Uncompressed baseline (gcgt_load_csr, §8 f3): the same BFS machinery reading col[] instead of the CGR.
+    Only ``bfs`` is supported on the returned graph."""
+    ro = np.ascontiguousarray(row_offsets, dtype=np.uint64)
+    co = np.ascontiguousarray(cols, dtype=np.uint32)
+    if co.size == 0:
+        co = np.zeros(1, dtype=np.uint32)
+    if stream == "torch":
+        import torch
+        stream = torch.cuda.current_stream(device).cuda_stream
+    csr = Csr(ro.size - 1, ro.ctypes.data, co.ctypes.data)
+    opts = LoadOpts(device, C.c_void_p(stream) if stream else None, 0, 1, None, None, 1 if symmetric else 0,
+                    1 if direction_optimizing else 0)
+    h = C.c_void_p()
+    _check(lib().gcgt_load_csr(C.byref(csr), C.byref(opts), C.byref(h)), "gcgt_load_csr")
+    g = Graph.__new__(Graph)
+    g._in_cgr = None
+    g._h = h
+    g.n = int(ro.size - 1)
+    g.last_stats = {}
+    return g
 
 
 def debug_warp_decode(bytes_: np.ndarray, nbits: int, zeta_k: int, window: int, count: int):

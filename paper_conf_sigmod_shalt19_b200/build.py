@@ -18,7 +18,7 @@ NCCL_INC = "/usr/include"
 
 SOURCES_CU = ["gcgt.cu"]
 SOURCES_CPP = ["encode.cpp"]
-HEADERS = ["internal.h", "decode.cuh"]
+HEADERS = ["internal.h", "decode.cuh", "csr_bfs.cuh"]
 
 
 def _newer(target, deps):

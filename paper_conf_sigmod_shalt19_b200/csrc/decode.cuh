@@ -38,18 +38,41 @@ __device__ __noinline__ uint64_t decode_slow(const uint64_t* __restrict__ W, uin
 }
 
 // decodeNum (Alg. 1 l.6): one VLC codeword at p; advances p.
+// Fast path in 32-bit arithmetic: the top 32 bits of the window (one funnel shift of the two words holding it) hold
+// every codeword of at most 32 bits (zeta_3: values < 2^24; gamma: < 2^15), i.e. nearly all gaps and counts; longer
+// codewords take the 64-bit window, then the bit-serial slow path.
 template <int K>
 __device__ __forceinline__ uint64_t decode(const uint64_t* __restrict__ W, uint64_t& p) {
-    const uint64_t win = window(W, p);
-    const uint32_t z = (uint32_t)__clzll((long long)win);
+    const uint64_t i = p >> 6;
+    const uint32_t s = (uint32_t)(p & 63);
+    const uint64_t a = ldg64(W + i), b = ldg64(W + i + 1);
+    const uint32_t x = s < 32 ? (uint32_t)(a >> 32) : (uint32_t)a;
+    const uint32_t y = s < 32 ? (uint32_t)a : (uint32_t)(b >> 32);
+    const uint32_t hi = __funnelshift_l(y, x, s & 31);  // window bits 0..31
+    const uint32_t z = __clz(hi);
     if (K == 1) {
-        if (z < 32) {
+        if (z < 16) {
             const uint32_t L = 2 * z + 1;
+            p += L;
+            return hi >> (32 - L);
+        }
+    } else {
+        const uint32_t h = z + 1, L = h * (K + 1);
+        if (L <= 32) {
+            p += L;
+            return (hi << h) >> (32 - K * h);
+        }
+    }
+    const uint64_t win = s ? (a << s) | (b >> (64 - s)) : a;
+    const uint32_t zz = (uint32_t)__clzll((long long)win);
+    if (K == 1) {
+        if (zz < 32) {
+            const uint32_t L = 2 * zz + 1;
             p += L;
             return win >> (64 - L);
         }
     } else {
-        const uint32_t h = z + 1, L = h * (K + 1);
+        const uint32_t h = zz + 1, L = h * (K + 1);
         if (L <= 64) {
             p += L;
             return (win << h) >> (64 - K * h);
@@ -296,6 +319,24 @@ struct BitBuf {
             buf |= (uint64_t)ld32(W, nxt) << (32 - avail);
             avail += 32;
             nxt++;
+        }
+        // fast path (32-bit arithmetic): after the refill avail > 32, so a codeword of <= 32 bits is complete
+        const uint32_t hi = (uint32_t)(buf >> 32);
+        const uint32_t z32 = __clz(hi);
+        if (K == 1) {
+            if (z32 < 16) {
+                const uint32_t L = 2 * z32 + 1;
+                buf <<= L;
+                avail -= L;
+                return hi >> (32 - L);
+            }
+        } else {
+            const uint32_t h = z32 + 1, L = h * (K + 1);
+            if (L <= 32) {
+                buf <<= L;
+                avail -= L;
+                return (hi << h) >> (32 - K * h);
+            }
         }
         const uint32_t z = (uint32_t)__clzll((long long)buf);
         uint32_t L, h = 0;

@@ -102,6 +102,19 @@ struct gcgt_graph {
     LongRange* lrq = nullptr;              // per-level long-range queue
     unsigned long long* lr_ctr = nullptr;  // (entries << 32) | chunks
     uint32_t long_len = 1024, lr_chunk = 256;
+    // uncompressed baseline (gcgt_load_csr, §8 f3): device CSR (+ in-lists for bottom-up) instead of the CGR
+    bool is_csr = false;
+    uint64_t* crow = nullptr;
+    uint32_t* ccol = nullptr;
+    uint64_t* crow_in = nullptr;
+    uint32_t* ccol_in = nullptr;
+    bool csr_in_owned = false;
+    void* csr_hubq = nullptr;
+    unsigned long long* mf = nullptr;  // record bits (CSR: arcs) of the new frontier, for bfs_decide
+    // direction test: record bits (Beamer's edge form) on symmetric graphs, vertex counts on directed ones (sweep of
+    // round 1: R-MAT 1.39 -> 0.60 ms with bits; the directed web / social recipes are faster with vertex counts)
+    bool dir_bits = false;
+    uint32_t alpha_bits = 30;
     uint32_t* bstate = nullptr;  // BFS direction state [8]: 0 dir (0 TD, 1 BU), 1 visited, 2 new-frontier count,
                                  // 3 previous frontier count
     // work
@@ -354,12 +367,14 @@ __device__ __forceinline__ void expand_phase(const Ctx& c, const Front& fr, cons
         const uint64_t b = qlen / ((uint64_t)gridDim.x * kWarps * 4);
         wpb = b < 1 ? 1 : (b > 8 ? 8 : (uint32_t)b);
     }
-    unsigned long long next = 0;  // the next batch's cursor value is fetched one batch ahead (latency hidden)
-    if (lane == 0) next = atomicAdd(c.cursor, (unsigned long long)wpb);
+    // Every warp's first batch is static (its global warp index), so a small frontier costs no cursor atomics; later
+    // batches come from the atomic cursor, numbered after the static ones and fetched one batch ahead.
+    const uint64_t nstatic = (uint64_t)gridDim.x * kWarps * wpb;
+    unsigned long long next = ((uint64_t)blockIdx.x * kWarps + wid) * wpb;
     for (;;) {
         const uint64_t base = __shfl_sync(0xffffffffu, next, 0);
         if (base >= qlen) break;
-        if (lane == 0) next = atomicAdd(c.cursor, (unsigned long long)wpb);
+        if (lane == 0) next = nstatic + atomicAdd(c.cursor, (unsigned long long)wpb);
         uint32_t w = 0, bits = 0;
         if (lane < wpb && base + lane < qlen) fr.get(base + lane, w, bits);
         uint32_t incl = __popc(bits);
@@ -514,13 +529,14 @@ __device__ __forceinline__ void expand_phase(const Ctx& c, const Front& fr, cons
 template <int K, bool SEG, class App, class Front, bool DEFER, bool STAGED>
 __global__ void __launch_bounds__(kBlock, 4) expand_kernel(Ctx c, Front fr, App app, uint32_t wpb) {
     __shared__ WarpSmem smem[kWarps];
+    if (c.dir && *c.dir) return;  // this BFS level runs bottom-up: no work, cursor untouched
     uint64_t nv = 0, na = 0, nb = 0;
     expand_phase<K, SEG, App, Front, DEFER, STAGED>(c, fr, app, wpb, smem, nv, na, nb);
     add_stats(c.st, nv, na, nb);
-    // the last warp out resets the work cursor for the next launch
-    if (lane_id() == 0) {
-        const unsigned long long nw = (unsigned long long)gridDim.x * kWarps;
-        if (atomicAdd(c.cursor + 1, 1ull) == nw - 1) {
+    // the last block out resets the work cursor for the next launch
+    __syncthreads();
+    if (threadIdx.x == 0) {
+        if (atomicAdd(c.cursor + 1, 1ull) == gridDim.x - 1) {
             c.cursor[0] = 0;
             c.cursor[1] = 0;
         }
@@ -804,6 +820,8 @@ __device__ __forceinline__ void hub_phase(const Ctx& c, const App& app, uint64_t
 
 template <int K, bool STAGED, class App>
 __global__ void __launch_bounds__(kBlock) hub_kernel(Ctx c, App app) {
+    if (*(volatile unsigned long long*)c.hub_ctr == 0 && (!c.lr_ctr || *(volatile unsigned long long*)c.lr_ctr == 0))
+        return;  // no hub segments / long intervals this level
     uint64_t na = 0;
     hub_phase<K, STAGED>(c, app, na);
     add_stats(c.st, 0, na, 0);
@@ -983,6 +1001,45 @@ __global__ void cc_init(uint32_t* parent, uint64_t n) {
         parent[v] = (uint32_t)v;
 }
 
+// Direction choice for the next BFS level (Beamer et al.'s heuristic): switch to bottom-up when the new frontier is
+// large against the unvisited set and growing, back to top-down when it is small against n and shrinking.
+// st: [0] dir, [1] visited, [2] new-frontier count (consumed), [3] previous.  With mf_bits (record bits of the new
+// frontier, summed by the contraction) the top-down -> bottom-up test is Beamer's edge form with CGR bits as the
+// work measure: mf * alpha_bits > (unvisited vertices) * (mean record bits).
+struct DecideArgs {
+    uint32_t* st;
+    uint64_t n;
+    uint32_t alpha, beta;
+    int enabled;
+    const uint32_t* qn_len;
+    uint32_t* level_counter;
+    unsigned long long* mf_bits;
+    double bits_per_vertex;
+    uint32_t alpha_bits;
+    uint32_t* done;  // blocks of commit_dense finished (the last one decides)
+};
+
+__device__ __forceinline__ void decide_body(const DecideArgs& d) {
+    uint32_t* st = d.st;
+    if (*(volatile const uint32_t*)d.qn_len) *d.level_counter += 1;  // levels that produced a non-empty frontier
+    const uint64_t nf = *(volatile uint32_t*)(st + 2);
+    st[2] = 0;
+    const uint64_t visited = (uint64_t)st[1] + nf;
+    st[1] = (uint32_t)visited;
+    const uint64_t nu = d.n - visited, prev = st[3];
+    uint32_t dir = st[0];
+    bool to_bu = nf * d.alpha > nu;
+    if (d.mf_bits) {
+        to_bu = (double)*(volatile unsigned long long*)d.mf_bits * d.alpha_bits > (double)nu * d.bits_per_vertex;
+        *d.mf_bits = 0;
+    }
+    if (!d.enabled || nf == 0) dir = 0;
+    else if (dir == 0 && to_bu && nf > prev) dir = 1;
+    else if (dir == 1 && nf * d.beta < d.n && nf < prev) dir = 0;
+    st[0] = dir;
+    st[3] = (uint32_t)nf;
+}
+
 // ---- contraction ---------------------------------------------------------------------------------------------------
 // Dense scan of N over words [w_lo, w_hi): every non-zero word is folded into V (and F), cleared, and appended to
 // the next queue (one atomic per warp).  Also resets the hub counter and the consumed queue's length.
@@ -990,11 +1047,14 @@ __device__ __forceinline__ void commit_phase(uint32_t* __restrict__ V, uint32_t*
                                              uint32_t* __restrict__ N, uint64_t w_lo, uint64_t w_hi,
                                              uint32_t* __restrict__ qn, uint32_t* __restrict__ qn_len,
                                              uint32_t* __restrict__ qbits_out, int32_t* __restrict__ levels = nullptr,
-                                             int32_t new_level = 0, uint32_t* __restrict__ nf_count = nullptr) {
+                                             int32_t new_level = 0, uint32_t* __restrict__ nf_count = nullptr,
+                                             const uint64_t* __restrict__ offs = nullptr,
+                                             unsigned long long* __restrict__ mf_bits = nullptr) {
     const uint32_t lane = lane_id();
     const uint64_t gw = ((uint64_t)blockIdx.x * blockDim.x + threadIdx.x) >> 5;
     const uint64_t nwarps = ((uint64_t)gridDim.x * blockDim.x) >> 5;
     uint32_t nf = 0;
+    uint64_t mf = 0;
     for (uint64_t base = w_lo + gw * 32; base < w_hi; base += nwarps * 32) {
         const uint64_t w = base + lane;
         uint32_t b = 0;
@@ -1007,6 +1067,17 @@ __device__ __forceinline__ void commit_phase(uint32_t* __restrict__ V, uint32_t*
             if (F && F[w] != b) F[w] = b;  // F = exactly the new frontier
         }
         nf += __popc(b);
+        if (mf_bits && b) {  // record bits of the new frontier (the top-down work estimate of bfs_decide)
+            const uint64_t v0 = w * 32;
+            if (b == 0xffffffffu) {
+                mf += ldg64(offs + v0 + 32) - ldg64(offs + v0);
+            } else {
+                for (uint32_t m = b; m; m &= m - 1) {
+                    const uint64_t v = v0 + __ffs(m) - 1;
+                    mf += ldg64(offs + v + 1) - ldg64(offs + v);
+                }
+            }
+        }
         const uint32_t bal = __ballot_sync(0xffffffffu, b != 0);
         if (bal) {
             uint32_t pos = 0;
@@ -1029,6 +1100,10 @@ __device__ __forceinline__ void commit_phase(uint32_t* __restrict__ V, uint32_t*
         for (int o = 16; o; o >>= 1) nf += __shfl_xor_sync(0xffffffffu, nf, o);
         if (lane == 0 && nf) atomicAdd(nf_count, nf);
     }
+    if (mf_bits) {
+        for (int o = 16; o; o >>= 1) mf += __shfl_xor_sync(0xffffffffu, mf, o);
+        if (lane == 0 && mf) atomicAdd(mf_bits, (unsigned long long)mf);
+    }
 }
 
 __global__ void commit_dense(uint32_t* __restrict__ V, uint32_t* __restrict__ F, uint32_t* __restrict__ N,
@@ -1037,33 +1112,27 @@ __global__ void commit_dense(uint32_t* __restrict__ V, uint32_t* __restrict__ F,
                              unsigned long long* __restrict__ hub_ctr, uint32_t* __restrict__ heavy_len,
                              int32_t* __restrict__ levels = nullptr, int32_t new_level = 0,
                              uint32_t* __restrict__ nf_count = nullptr,
-                             unsigned long long* __restrict__ lr_ctr = nullptr) {
-    commit_phase(V, F, N, w_lo, w_hi, qn, qn_len, qbits_out, levels, new_level, nf_count);
+                             unsigned long long* __restrict__ lr_ctr = nullptr,
+                             const uint64_t* __restrict__ offs = nullptr,
+                             unsigned long long* __restrict__ mf_bits = nullptr, DecideArgs dec = DecideArgs{}) {
+    commit_phase(V, F, N, w_lo, w_hi, qn, qn_len, qbits_out, levels, new_level, nf_count, offs, mf_bits);
     if (blockIdx.x == 0 && threadIdx.x == 0) {
         if (reset_ctr) *reset_ctr = 0;
         if (hub_ctr) *hub_ctr = 0;
         if (heavy_len) *heavy_len = 0;
         if (lr_ctr) *lr_ctr = 0;
     }
-}
-
-// Direction choice for the next BFS level (one thread; Beamer et al.'s heuristic on vertex counts): switch to
-// bottom-up when the new frontier is large against the unvisited set and growing, back to top-down when it is
-// small against n and shrinking.  st: [0] dir, [1] visited, [2] new-frontier count (consumed), [3] previous.
-__global__ void bfs_decide(uint32_t* st, uint64_t n, uint32_t alpha, uint32_t beta, int enabled,
-                           const uint32_t* qn_len, uint32_t* level_counter) {
-    if (*qn_len) *level_counter += 1;  // levels that produced a non-empty next frontier
-    const uint64_t nf = st[2];
-    st[2] = 0;
-    const uint64_t visited = (uint64_t)st[1] + nf;
-    st[1] = (uint32_t)visited;
-    const uint64_t nu = n - visited, prev = st[3];
-    uint32_t dir = st[0];
-    if (!enabled || nf == 0) dir = 0;
-    else if (dir == 0 && nf * alpha > nu && nf > prev) dir = 1;
-    else if (dir == 1 && nf * beta < n && nf < prev) dir = 0;
-    st[0] = dir;
-    st[3] = (uint32_t)nf;
+    if (dec.st) {  // BFS: the last block out takes the direction decision for the next level
+        __syncthreads();
+        if (threadIdx.x == 0) {
+            __threadfence();
+            if (atomicAdd(dec.done, 1u) == gridDim.x - 1) {
+                __threadfence();
+                decide_body(dec);
+                *dec.done = 0;
+            }
+        }
+    }
 }
 
 // ---- bottom-up step (north_star addition; §8 a9) -----------------------------------------------------------------
@@ -1518,6 +1587,8 @@ gcgt_status copy_out(gcgt_graph* g, void* dst, const void* src, size_t bytes, in
     return GCGT_OK;
 }
 
+#include "csr_bfs.cuh"
+
 // Brackets one launch of the dominant kernel when profiling (the caller syncs before reading).
 inline gcgt_status kprof_begin(gcgt_graph* g) {
     if (g->profile) CU(cudaEventRecord(g->kev0, g->stream));
@@ -1676,7 +1747,9 @@ extern "C" void gcgt_unload(gcgt_graph* g) {
                     g->ctr,    g->hubq,    g->hub_ctr, g->cursor,   g->heavyq,   g->heavy_len, g->stats,
                     g->levels, g->parent,  g->sigma,  g->delta,     g->bc,      g->bstate,
                     g->hv_ids, g->hv_ptr,  g->hv_rem, g->ck_prev,   g->lr_ctr, g->hv_after, g->ck_pos, g->lrq,
-                    g->in_owned ? g->inW : nullptr, g->in_owned ? g->inOffs : nullptr};
+                    g->in_owned ? g->inW : nullptr, g->in_owned ? g->inOffs : nullptr,
+                    g->crow,   g->ccol,    g->csr_hubq, g->mf,
+                    g->csr_in_owned ? g->crow_in : nullptr, g->csr_in_owned ? g->ccol_in : nullptr};
     if (g->stream) {
         for (void* b : bufs)
             if (b) cudaFreeAsync(b, g->stream);
@@ -1722,6 +1795,7 @@ extern "C" gcgt_status gcgt_load(const gcgt_cgr* c, const gcgt_load_opts* opts, 
     g->n = c->n;
     g->nbits = c->nbits;
     g->P = c->params;
+    g->dir_bits = o.symmetric != 0 && !o.in_cgr;
     if (const char* tune = getenv("GCGT_TUNE")) {  // development knob: key=value,... (results never change)
         std::string t(tune);
         size_t i = 0;
@@ -1738,6 +1812,8 @@ extern "C" gcgt_status gcgt_load(const gcgt_cgr* c, const gcgt_load_opts* opts, 
                 else if (k == "engine") g->engine = (uint32_t)v;
                 else if (k == "bu_alpha") g->bu_alpha = (uint32_t)v;
                 else if (k == "bu_beta") g->bu_beta = (uint32_t)v;
+                else if (k == "dir_bits") g->dir_bits = v != 0;
+                else if (k == "alpha_bits") g->alpha_bits = (uint32_t)v;
                 else if (k == "dir_opt") g->dir_opt_knob = v != 0;
                 else if (k == "ck_c") g->ck_c = (uint32_t)std::max(1ul, v);  // 0xFFFFFFFF disables checkpoints
                 else if (k == "heavy_itv") g->heavy_itv = (uint32_t)v;
@@ -1804,7 +1880,8 @@ extern "C" gcgt_status gcgt_load(const gcgt_cgr* c, const gcgt_load_opts* opts, 
     g->offs = g->offs_alloc - g->lo;  // kernels index offs[u] with global vertex ids
     bswap_words<<<flat_grid(g.get(), nwords), kBlock, 0, g->stream>>>(g->W, nwords);
     CU(cudaMemsetAsync(g->N, 0, g->nw * 4, g->stream));
-    if ((st = galloc(g.get(), &g->bstate, 8))) return st;
+    if ((st = galloc(g.get(), &g->bstate, 8)) || (st = galloc(g.get(), &g->mf, 1))) return st;
+    CU(cudaMemsetAsync(g->mf, 0, 8, g->stream));
     // in-CGR for bottom-up levels: the transpose if given, else the out-CGR itself on symmetric graphs
     if (o.in_cgr) {
         const gcgt_cgr* ic = o.in_cgr;
@@ -1854,6 +1931,112 @@ extern "C" gcgt_status gcgt_load(const gcgt_cgr* c, const gcgt_load_opts* opts, 
     if ((st = galloc(g.get(), &g->lrq, nlong + 1))) return st;
     CU(cudaMemsetAsync(g->hub_ctr, 0, 8, g->stream));
     CU(cudaStreamSynchronize(g->stream));
+    CU(cudaGetLastError());
+    *out = g.release();
+    return GCGT_OK;
+}
+
+
+// Uncompressed baseline load (§8 f3): plain CSR on the device; in-lists = the host transpose (counting sort) or the
+// CSR itself when symmetric.  Shares the frontier buffers and counters with the CGR path.
+extern "C" gcgt_status gcgt_load_csr(const gcgt_csr* csr, const gcgt_load_opts* opts, gcgt_graph** out) {
+    gcgt_internal::clear_error();
+    if (!csr || !out || (csr->n && !csr->row_offsets)) return fail(GCGT_EINVAL, "null argument");
+    gcgt_load_opts o{};
+    if (opts) o = *opts;
+    if (o.nranks > 1) return fail(GCGT_EINVAL, "CSR baseline: single GPU only");
+    const uint64_t n = csr->n, m = n ? csr->row_offsets[n] : 0;
+    if (n >= 0xFFFFFFFFull) return fail(GCGT_ERANGE, "n must fit 32-bit ids");
+    if (m && !csr->cols) return fail(GCGT_EINVAL, "null cols");
+    for (uint64_t v = 0; v < n; v++)
+        if (csr->row_offsets[v + 1] < csr->row_offsets[v]) return fail(GCGT_EINVAL, "row_offsets not monotone");
+    for (uint64_t e = 0; e < m; e++)
+        if (csr->cols[e] >= n) return fail(GCGT_ERANGE, "column id >= n");
+    int ndev = 0;
+    if (cudaGetDeviceCount(&ndev) != cudaSuccess || ndev == 0) return fail(GCGT_ECUDA, "no CUDA device");
+    if (o.device < 0 || o.device >= ndev) return fail(GCGT_EINVAL, "bad device ordinal");
+    std::unique_ptr<gcgt_graph, void (*)(gcgt_graph*)> g(new gcgt_graph(), gcgt_unload);
+    g->device = o.device;
+    g->is_csr = true;
+    CU(cudaSetDevice(o.device));
+    CU(cudaDeviceGetAttribute(&g->num_sms, cudaDevAttrMultiProcessorCount, o.device));
+    if (o.stream) g->stream = (cudaStream_t)o.stream;
+    else {
+        CU(cudaStreamCreateWithFlags(&g->stream, cudaStreamNonBlocking));
+        g->own_stream = true;
+    }
+    g->dir_bits = o.symmetric != 0;
+    if (const char* tune = getenv("GCGT_TUNE")) {  // the direction-switch knobs apply here too
+        std::string t(tune);
+        for (const char* k : {"bu_alpha=", "bu_beta=", "alpha_bits=", "dir_bits="}) {
+            const size_t i = t.find(k);
+            if (i != std::string::npos && (i == 0 || t[i - 1] == ',')) {
+                const uint32_t v = (uint32_t)strtoul(t.c_str() + i + strlen(k), nullptr, 10);
+                if (k[0] == 'b' && k[3] == 'a') g->bu_alpha = v;
+                else if (k[0] == 'b') g->bu_beta = v;
+                else if (k[0] == 'a') g->alpha_bits = v;
+                else g->dir_bits = v != 0;
+            }
+        }
+    }
+    g->n = n;
+    g->lo = 0;
+    g->hi = n;
+    g->nw = (n + 31) / 32 + 1;
+    cudaStream_t s = g->stream;
+    gcgt_status st;
+    if ((st = galloc(g.get(), &g->crow, n + 1)) || (st = galloc(g.get(), &g->ccol, m)) ||
+        (st = galloc(g.get(), &g->V, g->nw)) || (st = galloc(g.get(), &g->F, g->nw)) ||
+        (st = galloc(g.get(), &g->N, g->nw)) || (st = galloc(g.get(), &g->ctr, 8)) ||
+        (st = galloc(g.get(), &g->stats, 1)) || (st = galloc(g.get(), &g->levels, n)) ||
+        (st = galloc(g.get(), &g->bstate, 8)) || (st = galloc(g.get(), &g->hub_ctr, 1)) ||
+        (st = galloc(g.get(), &g->mf, 1)) ||
+        (st = galloc(g.get(), &g->cursor, 2)))
+        return st;
+    g->qcap = 2 * g->nw;
+    if ((st = galloc(g.get(), &g->q, g->qcap))) return st;
+    CU(cudaMallocHost((void**)&g->h_ctr, 8 * sizeof(uint32_t)));
+    CU(cudaMallocHost((void**)&g->h_stats, sizeof(Stats)));
+    CU(cudaEventCreate(&g->ev0));
+    CU(cudaEventCreate(&g->ev1));
+    CU(cudaEventCreate(&g->kev0));
+    CU(cudaEventCreate(&g->kev1));
+    for (auto& e : g->sev) CU(cudaEventCreate(&e));
+    CU(cudaMemcpyAsync(g->crow, csr->row_offsets, (n + 1) * 8, cudaMemcpyHostToDevice, s));
+    if (m) CU(cudaMemcpyAsync(g->ccol, csr->cols, m * 4, cudaMemcpyHostToDevice, s));
+    CU(cudaMemsetAsync(g->N, 0, g->nw * 4, s));
+    CU(cudaMemsetAsync(g->cursor, 0, 16, s));
+    CU(cudaMemsetAsync(g->hub_ctr, 0, 8, s));
+    CU(cudaMemsetAsync(g->mf, 0, 8, s));
+    g->nbits = m;  // the CSR's "record bits" for the direction test: arcs
+    uint64_t nhub = 0;
+    for (uint64_t v = 0; v < n; v++) nhub += csr->row_offsets[v + 1] - csr->row_offsets[v] > kCsrHub;
+    CsrHubEntry* hubq = nullptr;
+    if ((st = galloc(g.get(), &hubq, nhub + 1))) return st;
+    g->csr_hubq = hubq;
+    if (o.direction_optimizing) {
+        if (o.symmetric) {
+            g->crow_in = g->crow;
+            g->ccol_in = g->ccol;
+            g->dir_opt = true;
+        } else {
+            std::vector<uint64_t> tro(n + 1, 0);
+            std::vector<uint32_t> tco(m);
+            for (uint64_t e = 0; e < m; e++) tro[csr->cols[e] + 1]++;
+            for (uint64_t v = 0; v < n; v++) tro[v + 1] += tro[v];
+            std::vector<uint64_t> pos(tro.begin(), tro.end() - 1);
+            for (uint64_t u = 0; u < n; u++)
+                for (uint64_t e = csr->row_offsets[u]; e < csr->row_offsets[u + 1]; e++)
+                    tco[pos[csr->cols[e]]++] = (uint32_t)u;
+            if ((st = galloc(g.get(), &g->crow_in, n + 1)) || (st = galloc(g.get(), &g->ccol_in, m))) return st;
+            g->csr_in_owned = true;
+            CU(cudaMemcpyAsync(g->crow_in, tro.data(), (n + 1) * 8, cudaMemcpyHostToDevice, s));
+            if (m) CU(cudaMemcpyAsync(g->ccol_in, tco.data(), m * 4, cudaMemcpyHostToDevice, s));
+            CU(cudaStreamSynchronize(s));  // tro / tco are host vectors
+            g->dir_opt = true;
+        }
+    }
+    CU(cudaStreamSynchronize(s));
     CU(cudaGetLastError());
     *out = g.release();
     return GCGT_OK;
@@ -1941,12 +2124,91 @@ extern "C" gcgt_status gcgt_graph_range(const gcgt_graph* g, uint64_t* lo, uint6
     return GCGT_OK;
 }
 
+
+// ---- uncompressed-CSR baseline (§8 f3, csr_bfs.cuh) -------------------------------------------------------------
+gcgt_status csr_bfs(gcgt_graph* g, uint32_t source, int32_t* levels, int placement, gcgt_stats* stats) {
+    cudaStream_t s = g->stream;
+    CU(cudaMemsetAsync(g->V, 0, g->nw * 4, s));
+    CU(cudaMemsetAsync(g->F, 0, g->nw * 4, s));
+    CU(cudaMemsetAsync(g->levels, 0xff, g->n * 4, s));
+    CU(cudaMemsetAsync(g->ctr, 0, 8 * 4, s));
+    CU(cudaMemsetAsync(g->hub_ctr, 0, sizeof(unsigned long long), s));
+    uint32_t* q[2] = {g->q, g->q + g->nw};
+    bfs_seed<<<1, 1, 0, s>>>(source, g->V, g->F, q[0], g->ctr + 0, nullptr, g->levels, g->bstate);
+    g->launches = 1;
+    static int per_sm = 0;
+    if (!per_sm) {
+        cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per_sm, csr_expand_kernel<QueueFront>, kBlock, 0);
+        if (per_sm < 1) per_sm = 1;
+    }
+    static int per_sm_bu = 0;
+    if (!per_sm_bu) {
+        cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per_sm_bu, csr_bu_kernel, kBlock, 0);
+        if (per_sm_bu < 1) per_sm_bu = 1;
+    }
+    const int egrid = per_sm * g->num_sms;
+    const int bgrid = (int)std::max<uint64_t>(1, std::min<uint64_t>((g->nw + kWarps - 1) / kWarps,
+                                                                    (uint64_t)per_sm_bu * g->num_sms));
+    CsrHubEntry* hubq = (CsrHubEntry*)g->csr_hubq;
+    uint64_t qlen = 1;
+    uint32_t level = 0;
+    gcgt_status st;
+    constexpr uint32_t kChunk = 4;
+    while (qlen) {
+        const uint32_t nlev = g->profile ? 1 : kChunk;
+        for (uint32_t i = 0; i < nlev; i++, level++) {
+            const int cur = level & 1, nxt = cur ^ 1;
+            const QueueFront fr{q[cur], g->ctr + cur, g->F, nullptr};
+            const BfsApp app{g->V, g->N, g->levels, (int32_t)level};
+            if ((st = kprof_begin(g))) return st;
+            if (g->profile) CU(cudaEventRecord(g->sev[0], s));
+            csr_expand_kernel<QueueFront><<<egrid, kBlock, 0, s>>>(g->crow, g->ccol, fr, app, g->cursor, hubq,
+                                                                    g->hub_ctr, g->dir_opt ? g->bstate : nullptr,
+                                                                    g->stats);
+            if (g->profile) CU(cudaEventRecord(g->sev[1], s));
+            csr_hub_kernel<<<hub_grid(g), kBlock, 0, s>>>(g->ccol, hubq, g->hub_ctr, app, g->stats);
+            if (g->profile) CU(cudaEventRecord(g->sev[2], s));
+            if (g->dir_opt)
+                csr_bu_kernel<<<bgrid, kBlock, 0, s>>>(g->crow_in, g->ccol_in, g->V, g->F, g->N, g->n, g->bstate,
+                                                        g->stats);
+            if (g->profile) CU(cudaEventRecord(g->sev[3], s));
+            if ((st = kprof_end(g))) return st;
+            commit_dense<<<flat_grid(g, g->nw), kBlock, 0, s>>>(g->V, g->F, g->N, 0, g->nw, q[nxt], g->ctr + nxt,
+                                                                 nullptr, g->ctr + cur, g->hub_ctr, nullptr,
+                                                                 g->levels, (int32_t)level + 1, g->bstate + 2,
+                                                                 nullptr, g->dir_bits && g->dir_opt ? g->crow : nullptr,
+                                                                 g->dir_bits && g->dir_opt ? g->mf : nullptr,
+                DecideArgs{g->bstate, g->n, g->bu_alpha, g->bu_beta, g->dir_opt ? 1 : 0, g->ctr + nxt, g->ctr + 6,
+                           g->dir_bits && g->dir_opt ? g->mf : nullptr,
+                           (double)g->nbits / (double)std::max<uint64_t>(1, g->n), g->alpha_bits, g->ctr + 7});
+            g->launches += 3 + (g->dir_opt ? 1 : 0);
+            if (g->profile) {
+                CU(cudaEventRecord(g->sev[4], s));
+                CU(cudaEventSynchronize(g->sev[4]));
+                for (int k = 0; k < 4; k++) {
+                    float ms = 0;
+                    CU(cudaEventElapsedTime(&ms, g->sev[k], g->sev[k + 1]));
+                    g->span_ms[k] += ms;
+                }
+            }
+        }
+        CU(cudaMemcpyAsync(g->h_ctr + 6, g->ctr + 6, 4, cudaMemcpyDeviceToHost, s));
+        CU(cudaMemcpyAsync(g->h_ctr + (level & 1), g->ctr + (level & 1), 4, cudaMemcpyDeviceToHost, s));
+        CU(cudaStreamSynchronize(s));
+        if ((st = kprof_collect(g))) return st;
+        qlen = g->h_ctr[level & 1];
+    }
+    if ((st = copy_out(g, levels, g->levels, g->n * 4, placement))) return st;
+    return end_call(g, stats, g->h_ctr[6] + 1);
+}
+
 extern "C" gcgt_status gcgt_bfs(gcgt_graph* g, uint32_t source, int32_t* levels, int placement, gcgt_stats* stats) {
     if (!g || !levels) return fail(GCGT_EINVAL, "null argument");
     if (g->nranks > 1) return fail(GCGT_EINVAL, "partitioned graph: use the gcgt_dist_* steps (dist.py)");
     if (source >= g->n) return fail(GCGT_ERANGE, "source >= n");
     gcgt_status st;
     if ((st = begin_call(g))) return st;
+    if (g->is_csr) return csr_bfs(g, source, levels, placement, stats);
     cudaStream_t s = g->stream;
     CU(cudaMemsetAsync(g->V, 0, g->nw * 4, s));
     CU(cudaMemsetAsync(g->F, 0, g->nw * 4, s));
@@ -2009,19 +2271,28 @@ extern "C" gcgt_status gcgt_bfs(gcgt_graph* g, uint32_t source, int32_t* levels,
             commit_dense<<<flat_grid(g, g->nw), kBlock, 0, s>>>(g->V, g->F, g->N, 0, g->nw, q[nxt], g->ctr + nxt,
                                                                  nullptr, g->ctr + cur, g->hub_ctr, g->heavy_len,
                                                                  g->levels, (int32_t)level + 1, g->bstate + 2,
-                                                                 g->lr_ctr);
-            bfs_decide<<<1, 1, 0, s>>>(g->bstate, g->n, g->bu_alpha, g->bu_beta, g->dir_opt ? 1 : 0, g->ctr + nxt,
-                                       g->ctr + 6);
+                                                                 g->lr_ctr, g->dir_bits && g->dir_opt ? g->offs : nullptr,
+                                                                 g->dir_bits && g->dir_opt ? g->mf : nullptr,
+                DecideArgs{g->bstate, g->n, g->bu_alpha, g->bu_beta, g->dir_opt ? 1 : 0, g->ctr + nxt, g->ctr + 6,
+                           g->dir_bits && g->dir_opt ? g->mf : nullptr,
+                           (double)g->nbits / (double)std::max<uint64_t>(1, g->n), g->alpha_bits, g->ctr + 7});
             if (g->profile) {  // profiling waits per level anyway (nlev = 1)
                 CU(cudaEventRecord(g->sev[4], s));
                 CU(cudaEventSynchronize(g->sev[4]));
+                float lms[4];
                 for (int k = 0; k < 4; k++) {
-                    float ms = 0;
-                    CU(cudaEventElapsedTime(&ms, g->sev[k], g->sev[k + 1]));
-                    g->span_ms[k] += ms;
+                    CU(cudaEventElapsedTime(&lms[k], g->sev[k], g->sev[k + 1]));
+                    g->span_ms[k] += lms[k];
+                }
+                if (getenv("GCGT_TRACE")) {  // development aid (tools/trace_bfs.py): one line per level on stderr
+                    uint32_t hb[4], hq = 0;
+                    CU(cudaMemcpy(hb, g->bstate, 16, cudaMemcpyDeviceToHost));
+                    CU(cudaMemcpy(&hq, g->ctr + nxt, 4, cudaMemcpyDeviceToHost));
+                    fprintf(stderr, "level %3u next_dir %u visited %10u new %9u next_words %8u | exp %.4f hub %.4f "
+                            "bu %.4f commit %.4f ms\n", level, hb[0], hb[1], hb[3], hq, lms[0], lms[1], lms[2], lms[3]);
                 }
             }
-            g->launches += 3 + (g->P.residual_segment_len ? 1 : 0) + (g->dir_opt ? 1 : 0) + (heavy_active(g) ? 1 : 0);
+            g->launches += 2 + (g->P.residual_segment_len ? 1 : 0) + (g->dir_opt ? 1 : 0) + (heavy_active(g) ? 1 : 0);
         }
         CU(cudaMemcpyAsync(g->h_ctr + 6, g->ctr + 6, 4, cudaMemcpyDeviceToHost, s));
         CU(cudaMemcpyAsync(g->h_ctr + (level & 1), g->ctr + (level & 1), 4, cudaMemcpyDeviceToHost, s));
@@ -2036,6 +2307,7 @@ extern "C" gcgt_status gcgt_bfs(gcgt_graph* g, uint32_t source, int32_t* levels,
 
 extern "C" gcgt_status gcgt_cc(gcgt_graph* g, uint32_t* labels, int placement, gcgt_stats* stats) {
     if (!g || !labels) return fail(GCGT_EINVAL, "null argument");
+    if (g->is_csr) return fail(GCGT_EINVAL, "CSR baseline graph: BFS only");
     if (g->nranks > 1) return fail(GCGT_EINVAL, "partitioned graph: use the gcgt_dist_* steps (dist.py)");
     gcgt_status st;
     if (!g->parent && (st = galloc(g, &g->parent, g->n))) return st;
@@ -2065,6 +2337,7 @@ extern "C" gcgt_status gcgt_cc(gcgt_graph* g, uint32_t* labels, int placement, g
 
 extern "C" gcgt_status gcgt_bc(gcgt_graph* g, const uint32_t* sources, uint32_t k, double* bc, int placement,
                                gcgt_stats* stats) {
+    if (g && g->is_csr) return fail(GCGT_EINVAL, "CSR baseline graph: BFS only");
     if (!g || !bc || (k && !sources)) return fail(GCGT_EINVAL, "null argument");
     if (g->nranks > 1) return fail(GCGT_EINVAL, "partitioned graph: BC shards sources over full replicas (dist.py)");
     for (uint32_t i = 0; i < k; i++)
@@ -2162,6 +2435,7 @@ gcgt_status dist_sync(gcgt_graph* g) {
 extern "C" gcgt_status gcgt_dist_bfs_begin(gcgt_graph* g, uint32_t source) {
     gcgt_internal::clear_error();
     if (!g) return fail(GCGT_EINVAL, "null graph");
+    if (g->is_csr) return fail(GCGT_EINVAL, "CSR baseline graph: single-GPU BFS only");
     if (source >= g->n) return fail(GCGT_ERANGE, "source >= n");
     CU(cudaSetDevice(g->device));
     cudaStream_t s = g->stream;

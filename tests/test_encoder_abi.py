@@ -135,3 +135,20 @@ def test_encode_transpose_bit_exact(ml, sl, k):
     ob, onb, ooffs = O.encode(tro, tco, ml, sl, k)
     b, nb, offs, n, _ = G.encode_transpose(ro, co, ml, sl, k).view()
     assert nb == onb and np.array_equal(offs, ooffs) and np.array_equal(b, ob)
+
+
+def test_load_csr_validates_then_fails_loudly_without_gpu():
+    """The CSR baseline checks its input before touching the device (ERANGE for an id >= n), and has no CPU
+    fallback either (ECUDA without a device)."""
+    import torch
+    ro, co = random_graph(50, 200, seed=2)
+    bad = co.copy()
+    bad[3] = 50
+    with pytest.raises(G.GcgtError) as e:
+        G.load_csr(ro, bad)
+    assert e.value.status == G.ERANGE
+    if torch.cuda.is_available():
+        pytest.skip("GPU present")
+    with pytest.raises(G.GcgtError) as e:
+        G.load_csr(ro, co)
+    assert e.value.status == G.ECUDA

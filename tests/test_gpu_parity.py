@@ -199,7 +199,7 @@ def test_warp_decoder_random_streams(k):
 # ---------------------------------------------------------------------------------------------------------------------
 # Direction-optimizing BFS (bottom-up levels over the in-CGR, §8 a9)
 # ---------------------------------------------------------------------------------------------------------------------
-@pytest.mark.parametrize("tune", ["", "bu_alpha=100000,bu_beta=1", "bu_alpha=100000,bu_beta=100000"])
+@pytest.mark.parametrize("tune", ["", "bu_alpha=100000,bu_beta=1", "bu_alpha=100000,bu_beta=100000", "wpb_max=2"])
 @pytest.mark.parametrize("name", ["c1", "rmat_s", "web_s", "social_s"])
 def test_bfs_direction_optimizing(name, tune, monkeypatch):
     """Symmetric graphs use the out-CGR as in-CGR; directed ones the encoded transpose.  The tunes force
@@ -226,3 +226,39 @@ def test_bfs_bottom_up_random(ml, sl, k, monkeypatch):
         g = G.load(cgr, symmetric=True) if sym else G.load(cgr, in_cgr=G.encode_transpose(ro, co, ml, sl, k))
         for s in (0, 17, 5999):
             assert np.array_equal(g.bfs(s), O.bfs(ro, co, s)), (seed, s)
+
+
+# ---------------------------------------------------------------------------------------------------------------------
+# Uncompressed-CSR baseline (§8 f3): same levels as the oracle on every recipe, top-down and direction-optimizing
+# ---------------------------------------------------------------------------------------------------------------------
+@pytest.mark.parametrize("tune", ["", "bu_alpha=100000,bu_beta=1", "bu_alpha=100000,bu_beta=100000"])
+@pytest.mark.parametrize("name", ["c1", "rmat_s", "web_s", "social_s"])
+def test_csr_baseline_bfs(name, tune, monkeypatch):
+    monkeypatch.setenv("GCGT_TUNE", tune)
+    cfg = synth.CONFIGS[name]
+    ro, co = cfg.make()
+    for dopt in (False, True):
+        g = G.load_csr(ro, co, symmetric=cfg.symmetric, direction_optimizing=dopt)
+        for r in [0] + synth.pick_roots(ro, 3):
+            assert np.array_equal(g.bfs(r), O.bfs(ro, co, r)), (name, tune, dopt, r)
+        g.unload()
+
+
+def test_csr_baseline_hubs_and_errors():
+    """Hub vertices (more than kCsrHub = 4096 arcs: chunked over the grid), isolated vertices, and the BFS-only
+    contract (CC / BC refuse a CSR graph)."""
+    n = 200_000
+    rng = np.random.default_rng(5)
+    hub = np.unique(rng.integers(0, n, size=50_000))
+    src = np.concatenate([np.zeros(hub.size), rng.integers(0, n, size=100_000)]).astype(np.int64)
+    dst = np.concatenate([hub, rng.integers(0, n, size=100_000)]).astype(np.int64)
+    ro, co = csr_from_edges(n, src, dst)
+    g = G.load_csr(ro, co, direction_optimizing=True)
+    for s in (0, 1, int(hub[3]), n - 1):
+        assert np.array_equal(g.bfs(s), O.bfs(ro, co, s)), s
+    with pytest.raises(G.GcgtError) as e:
+        g.cc()
+    assert e.value.status == G.EINVAL
+    with pytest.raises(G.GcgtError) as e:
+        g.bc([0])
+    assert e.value.status == G.EINVAL
