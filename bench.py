@@ -137,6 +137,26 @@ def smi_clocks(dev):
         return {"sm_mhz": None, "sm_max_mhz": None, "reasons": ["clock sampling unavailable"], "samples": 0}
 
 
+def ncu_traffic(cfg_name, levels_per_bfs):
+    """DRAM bytes per level-expansion launch from the committed ncu launch list of one BFS of this config
+    (profiles/*_launches_<cfg>.json: `ncu --metrics gpu__time_duration.sum,dram__bytes_read.sum,dram__bytes_write.sum`
+    over tools/prof_bfs.py, one root).  ncu flushes caches before every launch, so this is a cold-cache upper bound."""
+    import glob
+    files = sorted(glob.glob(os.path.join(ROOT, "profiles", f"*_launches_{cfg_name}.json")))  # newest round last
+    if not files:
+        return None, None
+    with open(files[-1]) as f:
+        d = json.load(f)
+    tot, launches = 0.0, 0
+    for k, v in d.items():
+        if any(x in k for x in ("expand_kernel", "hub_kernel", "bu_kernel")):
+            tot += v["dram_bytes"]
+            launches = max(launches, v["launches"])
+    if not launches:
+        return None, None
+    return tot / launches, os.path.relpath(files[-1], ROOT)
+
+
 def dist_env():
     ws = int(os.environ.get("WORLD_SIZE", "1"))
     rank = int(os.environ.get("RANK", "0"))
@@ -298,6 +318,7 @@ def main():
     k_s = tot["kms"] * 1e-3
     achieved = alg_bytes / k_s / 1e9 if k_s > 0 else 0.0
     cgr_gbs = tot["bits"] / 8 / k_s / 1e9 if k_s > 0 else 0.0
+    traffic, traffic_src = ncu_traffic(args.config, tot["levels"] / args.steps)
 
     e2e = None
     if not args.no_e2e:
@@ -321,7 +342,8 @@ def main():
                            "parallelism": f"{ws} x independent BFS queries (replicas)" if ws > 1 else "1 GPU",
                            "gen_s": round(tgen, 1), "encode_s": round(tenc, 1)},
                 "roofline": {"bound": "hbm", "achieved": achieved, "peak": peak, "unit": "GB/s",
-                             "frac": achieved / peak, "traffic": None, "kernel": "level expansion (expand_kernel+hub_kernel | bu_kernel)",
+                             "frac": achieved / peak, "traffic": traffic,
+                             "traffic_source": traffic_src, "alg_bytes_per_launch": alg_bytes / max(1, tot["klaunch"]), "kernel": "level expansion (expand_kernel+hub_kernel | bu_kernel)",
                              "peak_source": peak_src, "cgr_only_gbs": cgr_gbs, "cgr_only_frac": cgr_gbs / peak,
                              "kernel_share_of_step": tot["kms"] / t_ms if t_ms else None,
                              "launches": tot["klaunch"]},

@@ -107,6 +107,10 @@ typedef struct {
                                BFS step; NULL = none (top-down only unless `symmetric`).  Same n and params.      */
     int symmetric;     /* 1: every arc u->v has v->u, so the out-CGR doubles as the in-CGR (R-MAT configs)           */
     int direction_optimizing; /* 0: top-down only; 1: switch top-down <-> bottom-up per level when an in-CGR exists */
+    int host_resident; /* 1: keep the CGR words (and the in-CGR's) in pinned, mapped HOST memory owned by the graph and
+                          decode them over the host link (zero copy; §8 f4, the out-of-core motivation PAPER.md:93-120,
+                          :474-479); bit offsets, bitmaps and outputs stay in device memory.  Results are identical;
+                          only the bandwidth differs.  0: the CGR is copied to HBM (default).                      */
 } gcgt_load_opts;
 
 /* Copies the CGR (bytes + bit_offsets) to the device and allocates the traversal work buffers.  With nranks > 1

@@ -54,7 +54,7 @@ class Stats(C.Structure):
 class LoadOpts(C.Structure):
     _fields_ = [("device", C.c_int), ("stream", C.c_void_p), ("rank", C.c_int), ("nranks", C.c_int),
                 ("nccl_comm", C.c_void_p), ("in_cgr", C.c_void_p), ("symmetric", C.c_int),
-                ("direction_optimizing", C.c_int)]
+                ("direction_optimizing", C.c_int), ("host_resident", C.c_int)]
 
 
 _lib = None
@@ -213,13 +213,14 @@ class Graph:
     """Device-resident CGR (gcgt_load)."""
 
     def __init__(self, cgr: CGR, device: int = 0, stream=None, rank: int = 0, nranks: int = 1, nccl_comm=None,
-                 in_cgr: "CGR | None" = None, symmetric: bool = False, direction_optimizing: bool = True):
+                 in_cgr: "CGR | None" = None, symmetric: bool = False, direction_optimizing: bool = True,
+                 host_resident: bool = False):
         if stream == "torch":
             import torch
             stream = torch.cuda.current_stream(device).cuda_stream
         opts = LoadOpts(device, C.c_void_p(stream) if stream else None, rank, nranks,
                         C.c_void_p(nccl_comm) if nccl_comm else None, in_cgr.handle if in_cgr is not None else None,
-                        1 if symmetric else 0, 1 if direction_optimizing else 0)
+                        1 if symmetric else 0, 1 if direction_optimizing else 0, 1 if host_resident else 0)
         self._in_cgr = in_cgr
         h = C.c_void_p()
         _check(lib().gcgt_load(cgr.handle, C.byref(opts), C.byref(h)), "gcgt_load")

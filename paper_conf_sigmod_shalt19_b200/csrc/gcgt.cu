@@ -63,6 +63,8 @@ struct HubEntry {
     uint64_t base;     // bit position of the vertex's first residual segment
     uint32_t u;        // vertex
     uint32_t seg_off;  // first flattened segment index of this entry (entries are ordered by seg_off)
+    uint32_t epoch;    // expansion launch that published the entry (fused hub consumption waits for it)
+    uint32_t pad;
 };
 
 // A long interval (more than long_len ids) deferred to the level's long-range queue and expanded grid-wide in chunks
@@ -70,6 +72,7 @@ struct HubEntry {
 // PAPER.md:667-688) at grid scale.  Entries are ordered by chunk_off (one packed atomic hands out both indices).
 struct LongRange {
     uint32_t u, start, len, chunk_off;
+    uint32_t epoch;  // as HubEntry::epoch
 };
 
 struct HeavyEntry {
@@ -94,10 +97,15 @@ struct gcgt_graph {
     uint64_t* inW = nullptr;     // in-CGR (transpose) for bottom-up; aliases W / offs when symmetric
     uint64_t* inOffs = nullptr;
     bool in_owned = false;       // inW / inOffs are separate allocations
+    // host-resident CGR (§8 f4, gcgt_load_opts.host_resident): W / inW point into pinned, mapped host memory that
+    // the kernels read over the host link (zero copy); only O(n) tables live in HBM
+    uint64_t* hostW = nullptr;
+    uint64_t* hostInW = nullptr;
     bool dir_opt = false;        // direction-optimizing BFS enabled (in-CGR available)
     // interval checkpoint table (derived at load) + per-level chunk queue
     uint32_t hv_n = 0, ck_c = 4;
     uint32_t *hv_ids = nullptr, *hv_ptr = nullptr, *hv_rem = nullptr, *ck_prev = nullptr;
+    uint32_t *hv_wptr = nullptr, *hv_bits = nullptr;  // per-word index of hv_ids (hv_index)
     uint64_t *hv_after = nullptr, *ck_pos = nullptr;
     LongRange* lrq = nullptr;              // per-level long-range queue
     unsigned long long* lr_ctr = nullptr;  // (entries << 32) | chunks
@@ -131,12 +139,17 @@ struct gcgt_graph {
     // deferring long interval areas to a separate pass costs more than the in-batch straggler it removes
     bool staged = false;
     bool persistent = false;
+    uint32_t flatb = 0;       // phase B lane-refill loop (GCGT_TUNE flatb=1; measured no faster on C2, session 3)
+    uint32_t fuse_warps = 0;  // fused hub consumption: consumer warps per expand block (GCGT_TUNE fuse=N; 0 = hub_kernel)
     bool dir_opt_knob = true;
     uint32_t engine = 0;  // 0 = phase kernel; 1 = state-machine kernel (measured slower on C2: lone long tasks)  // BFS: all levels in one cooperative launch (measured slower on C2; GCGT_TUNE knob)
     uint32_t heavy_itv = 0xFFFFFFFFu, heavy_res = 1024, hub_segs = 8, wpb_max = 8;
+    uint32_t bu_kernel = 1;  // bottom-up kernel: 1 = per-word (lane = vertex id), 2 = compacted chunks (bu_words/bu_batch)
+    uint32_t bu_words = 8, bu_batch = 4;  // bottom-up: frontier words per warp chunk, residuals per probe batch
     uint32_t bu_alpha = 4, bu_beta = 24;  // switch thresholds on vertex counts (C2/R-MAT/social sweep, r1)
     uint32_t* heavy_len = nullptr;
     unsigned long long* hub_ctr = nullptr;
+    uint32_t* fuse_ctr = nullptr;  // fused hub consumption counters [4] (Ctx::fuse_ctr)
     Stats* stats = nullptr;
     int32_t* levels = nullptr;
     uint32_t* parent = nullptr;
@@ -187,6 +200,9 @@ struct Ctx {
     uint32_t hv_n, ck_c;
     const uint32_t* __restrict__ hv_ids;
     const uint32_t* __restrict__ hv_ptr;
+    const uint32_t* __restrict__ hv_wptr;  // per-word index (hv_index), words from hv_w0
+    const uint32_t* __restrict__ hv_bits;
+    uint64_t hv_w0;
     const uint64_t* __restrict__ hv_after;  // bit after the interval area
     const uint32_t* __restrict__ hv_rem;    // unsegmented records: residual count
     const uint64_t* __restrict__ ck_pos;
@@ -194,7 +210,36 @@ struct Ctx {
     LongRange* lrq;
     unsigned long long* lr_ctr;
     uint32_t long_len, lr_chunk;
+    // fused hub consumption (expand_kernel drains the level's hub segments / long ranges itself, no hub_kernel):
+    // fuse_ctr[0] blocks done expanding, [1] long-range take cursor, [2] hub-segment take cursor, [3] epoch
+    uint32_t fuse;
+    uint32_t* fuse_ctr;
+    uint32_t flatb;  // phase B as a lane-refill loop (1) or in static rounds of 32 tasks (0)
 };
+
+// Publication of hub / long-range entries: the data, a fence, then the launch's epoch (the readiness flag).
+__device__ __forceinline__ void publish_hub(HubEntry* q, uint64_t idx, uint64_t base, uint32_t u, uint32_t off,
+                                            uint32_t epoch) {
+    HubEntry* e = q + idx;
+    e->base = base;
+    e->u = u;
+    e->seg_off = off;
+    __threadfence();
+    *(volatile uint32_t*)&e->epoch = epoch;
+}
+__device__ __forceinline__ void publish_lr(LongRange* q, uint64_t idx, uint32_t u, uint32_t start, uint32_t len,
+                                           uint32_t off, uint32_t epoch) {
+    LongRange* e = q + idx;
+    e->u = u;
+    e->start = start;
+    e->len = len;
+    e->chunk_off = off;
+    __threadfence();
+    *(volatile uint32_t*)&e->epoch = epoch;
+}
+__device__ __forceinline__ uint32_t cur_epoch(const Ctx& c) {
+    return c.fuse_ctr ? *(volatile const uint32_t*)(c.fuse_ctr + 3) : 0u;
+}
 
 __device__ __forceinline__ void add_stats(Stats* st, uint64_t v, uint64_t a, uint64_t b) {
     for (int o = 16; o; o >>= 1) {  // warp reduce (call with the full warp), one atomic per warp
@@ -277,7 +322,7 @@ __device__ __forceinline__ void range_or_defer(const Ctx& c, App& t, uint32_t u,
     }
     const uint32_t nch = (len + c.lr_chunk - 1) / c.lr_chunk;
     const unsigned long long old = atomicAdd(c.lr_ctr, (1ull << 32) | (unsigned long long)nch);
-    c.lrq[old >> 32] = LongRange{u, start, len, (uint32_t)(old & 0xffffffffu)};
+    publish_lr(c.lrq, old >> 32, u, start, len, (uint32_t)(old & 0xffffffffu), cur_epoch(c));
 }
 
 // Per-codeword global-window reader (the unstaged alternative to RegStream; same interface).
@@ -352,6 +397,7 @@ struct WarpSmem {
     uint32_t u[32], spre[33];
     uint64_t base[32];
     uint32_t ckb[32], nck[32], itv[32];  // interval-chunk tasks of long interval areas (checkpoint table)
+    uint32_t take;                       // phase-B work cursor (lane-refill loop)
 };
 
 // DEFER = true: the level's frontier pass (heavy vertices are queued); false: the heavy pass over that queue
@@ -427,11 +473,8 @@ __device__ __forceinline__ void expand_phase(const Ctx& c, const Front& fr, cons
                     bool ck = false;
                     uint64_t after = 0;
                     if (c.hv_n && itv > c.ck_c) {  // long interval area: chunks beyond the first go grid-wide
-                        uint32_t lo = 0, hi = c.hv_n - 1;
-                        while (lo < hi) {
-                            const uint32_t mid = (lo + hi) >> 1;
-                            if (c.hv_ids[mid] < u) lo = mid + 1; else hi = mid;
-                        }
+                        const uint64_t wl = (u >> 5) - c.hv_w0;
+                        const uint32_t lo = c.hv_wptr[wl] + __popc(c.hv_bits[wl] & ((1u << (u & 31)) - 1));
                         ckb = c.hv_ptr[lo];  // chunks 1.. become phase-B tasks of this batch
                         nck = c.hv_ptr[lo + 1] - ckb;
                         itv_all = (uint32_t)itv;
@@ -465,7 +508,7 @@ __device__ __forceinline__ void expand_phase(const Ctx& c, const Front& fr, cons
                         if (nseg > c.hub_segs || (!DEFER && nseg)) {  // hub: hand the segments to the whole grid
                             const unsigned long long old =
                                 atomicAdd(c.hub_ctr, (1ull << 32) | (unsigned long long)nseg);
-                            c.hubq[old >> 32] = HubEntry{segbase, u, (uint32_t)(old & 0xffffffffu)};
+                            publish_hub(c.hubq, old >> 32, segbase, u, (uint32_t)(old & 0xffffffffu), cur_epoch(c));
                             nseg = 0;
                         }
                     }
@@ -486,8 +529,72 @@ __device__ __forceinline__ void expand_phase(const Ctx& c, const Front& fr, cons
                 sm.itv[lane] = itv_all;
                 sm.spre[lane + 1] = sincl;
                 if (lane == 0) sm.spre[0] = 0;
+                if (lane == 0) sm.take = 32;
                 __syncwarp();
                 const uint32_t stotal = sm.spre[32];
+                if (c.flatb) {
+                    // lane-refill loop: a lane that finishes its task takes the next one at once (warp-local work
+                    // cursor), so a round no longer waits for its longest segment; segments are decoded four
+                    // codewords per iteration (one batched probe per four ids)
+                    uint32_t sj = lane, rem = 0, su = 0;
+                    uint64_t sp = 0;
+                    int64_t scur = 0;
+                    bool sfirst = false, open = false;
+                    App t = app;
+                    for (;;) {
+                        if (rem == 0) {
+                            if (open) {
+                                t.end();
+                                open = false;
+                            }
+                            if (sj >= stotal) break;
+                            uint32_t lo = 0, hi = 31;
+                            while (lo < hi) {
+                                const uint32_t mid = (lo + hi + 1) >> 1;
+                                if (sm.spre[mid] <= sj) lo = mid; else hi = mid - 1;
+                            }
+                            su = sm.u[lo];
+                            const uint32_t idx = sj - sm.spre[lo], snck = sm.nck[lo];
+                            t = app;
+                            t.begin(su);
+                            open = true;
+                            if (idx < snck) {  // interval chunk idx+1 of su, processed whole
+                                const uint32_t k = sm.ckb[lo] + idx;
+                                const uint32_t left = sm.itv[lo] - (idx + 1) * c.ck_c;
+                                const uint32_t cnt = left < c.ck_c ? left : c.ck_c;
+                                uint64_t p = c.ck_pos[k];
+                                uint32_t cur = c.ck_prev[k];
+                                for (uint32_t i = 0; i < cnt; i++) {
+                                    const uint32_t g = (uint32_t)decode<K>(c.W, p);
+                                    const uint32_t len = (uint32_t)(decode<K>(c.W, p) - 1) + c.min_len;
+                                    range_or_defer(c, t, su, cur + g, len);
+                                    cur += g + len - 1;
+                                    na += len;
+                                }
+                            } else {
+                                sp = sm.base[lo] + (uint64_t)(idx - snck) * c.seg_bits;
+                                rem = (uint32_t)(decode<K>(c.W, sp) - 1);
+                                na += rem;
+                                sfirst = true;
+                            }
+                            sj = atomicAdd(&sm.take, 1u);
+                            continue;
+                        }
+                        uint32_t v[4];
+                        const uint32_t nb = min(4u, rem);
+#pragma unroll
+                        for (uint32_t k = 0; k < 4; k++) {
+                            if (k < nb) {
+                                const uint64_t cw = decode<K>(c.W, sp);
+                                scur = sfirst ? unmap_first(su, cw) : scur + (int64_t)cw;
+                                sfirst = false;
+                                v[k] = (uint32_t)scur;
+                            }
+                        }
+                        t.many(v, nb);
+                        rem -= nb;
+                    }
+                } else
                 for (uint32_t k0 = 0; k0 < stotal; k0 += 32) {
                     const uint32_t sj = k0 + lane;
                     if (sj < stotal) {
@@ -526,19 +633,124 @@ __device__ __forceinline__ void expand_phase(const Ctx& c, const Front& fr, cons
     }
 }
 
+// Fused hub consumption (Ctx::fuse): a block that has finished its share of the frontier drains the level's hub
+// segments and long-range chunks while other blocks are still expanding (and publishing more), instead of a separate
+// hub_kernel launch after the whole expansion.  Warps claim 32 items at a time from a take cursor; an item whose
+// entry is not yet published is waited for; the queues are final once every block has finished expanding (the
+// grid is one co-resident wave, so waiting cannot deadlock).  Entry reads bypass L1 (volatile): they are written
+// by other SMs during this launch.
+__device__ __forceinline__ uint32_t entry_off(const volatile HubEntry* e) { return e->seg_off; }
+__device__ __forceinline__ uint32_t entry_off(const volatile LongRange* e) { return e->chunk_off; }
+template <class E>
+__device__ __forceinline__ uint32_t find_entry(const E* q, uint32_t ne, uint32_t j, uint32_t epoch) {
+    uint32_t lo = 0, hi = ne - 1;  // largest entry whose offset is <= j (entries are ordered by offset)
+    while (lo < hi) {
+        const uint32_t mid = (lo + hi + 1) >> 1;
+        const volatile E* e = q + mid;
+        while (e->epoch != epoch) __nanosleep(32);
+        if (entry_off(e) <= j) lo = mid; else hi = mid - 1;
+    }
+    const volatile E* e = q + lo;
+    while (e->epoch != epoch) __nanosleep(32);
+    __threadfence();
+    return lo;
+}
+
+__device__ __forceinline__ uint32_t ld_acquire(const uint32_t* p) {
+    uint32_t v;
+    asm volatile("ld.acquire.gpu.global.u32 %0, [%1];" : "=r"(v) : "l"(p) : "memory");
+    return v;
+}
+__device__ __forceinline__ unsigned long long ld_acquire(const unsigned long long* p) {
+    unsigned long long v;
+    asm volatile("ld.acquire.gpu.global.u64 %0, [%1];" : "=l"(v) : "l"(p) : "memory");
+    return v;
+}
+
+template <int K, bool STAGED, class App>
+__device__ __forceinline__ void hub_consume(const Ctx& c, const App& app, uint32_t epoch, uint64_t& na) {
+    const uint32_t lane = lane_id();
+    uint32_t* fc = c.fuse_ctr;
+    for (;;) {
+        const uint32_t done = ld_acquire(fc);
+        const unsigned long long lc = ld_acquire(c.lr_ctr);
+        const unsigned long long hc = ld_acquire(c.hub_ctr);
+        const bool final = done == gridDim.x;
+        const uint32_t lt = ld_acquire(fc + 1), ht = ld_acquire(fc + 2);
+        int qsel;
+        if (lt < (uint32_t)lc) qsel = 0;
+        else if (ht < (uint32_t)hc) qsel = 1;
+        else if (final) return;
+        else {
+            __nanosleep(500);
+            continue;
+        }
+        uint32_t j0 = 0;
+        if (lane == 0) j0 = atomicAdd(fc + 1 + qsel, 32u);
+        j0 = __shfl_sync(0xffffffffu, j0, 0);
+        const uint32_t j = j0 + lane;
+        bool pending = true;
+        for (;;) {
+            const uint32_t dn = ld_acquire(fc);
+            const unsigned long long cv = ld_acquire(qsel == 0 ? c.lr_ctr : c.hub_ctr);
+            const uint32_t S = (uint32_t)cv, ne = (uint32_t)(cv >> 32);
+            if (pending && j < S) {
+                pending = false;
+                App t = app;
+                if (qsel == 0) {
+                    const uint32_t k = find_entry(c.lrq, ne, j, epoch);
+                    const volatile LongRange* e = c.lrq + k;
+                    const uint32_t eu = e->u, es = e->start, el = e->len, eo = e->chunk_off;
+                    const uint32_t off = (j - eo) * c.lr_chunk;
+                    t.begin(eu);
+                    t.range(es + off, min(c.lr_chunk, el - off));
+                    t.end();
+                } else {
+                    const uint32_t k = find_entry(c.hubq, ne, j, epoch);
+                    const volatile HubEntry* e = c.hubq + k;
+                    const uint64_t eb = e->base;
+                    const uint32_t eu = e->u, eo = e->seg_off;
+                    t.begin(eu);
+                    na += decode_segment<K, STAGED>(c.W, eb + (uint64_t)(j - eo) * c.seg_bits, eu, t);
+                    t.end();
+                }
+            }
+            const bool fin = dn == gridDim.x;
+            if (__all_sync(0xffffffffu, !pending || (fin && j >= S))) break;
+            __nanosleep(200);
+        }
+    }
+}
+
 template <int K, bool SEG, class App, class Front, bool DEFER, bool STAGED>
 __global__ void __launch_bounds__(kBlock, 4) expand_kernel(Ctx c, Front fr, App app, uint32_t wpb) {
     __shared__ WarpSmem smem[kWarps];
     if (c.dir && *c.dir) return;  // this BFS level runs bottom-up: no work, cursor untouched
     uint64_t nv = 0, na = 0, nb = 0;
+    const bool fuse = DEFER && c.fuse;
+    const uint32_t epoch = fuse ? cur_epoch(c) : 0u;
     expand_phase<K, SEG, App, Front, DEFER, STAGED>(c, fr, app, wpb, smem, nv, na, nb);
+    if (fuse) {
+        __syncthreads();
+        if (threadIdx.x == 0) {
+            __threadfence();
+            atomicAdd(c.fuse_ctr, 1u);
+        }
+        if ((threadIdx.x >> 5) < c.fuse) hub_consume<K, STAGED>(c, app, epoch, na);  // c.fuse consumer warps per block
+    }
     add_stats(c.st, nv, na, nb);
-    // the last block out resets the work cursor for the next launch
+    // the last block out resets the work cursor (and the fused-hub counters, advancing the epoch) for the next launch
     __syncthreads();
     if (threadIdx.x == 0) {
         if (atomicAdd(c.cursor + 1, 1ull) == gridDim.x - 1) {
             c.cursor[0] = 0;
             c.cursor[1] = 0;
+            if (fuse) {
+                c.fuse_ctr[0] = 0;
+                c.fuse_ctr[1] = 0;
+                c.fuse_ctr[2] = 0;
+                c.fuse_ctr[3] = epoch + 1;
+            }
         }
     }
 }
@@ -608,7 +820,7 @@ __global__ void __launch_bounds__(kBlock, 4) sm_expand_kernel(Ctx c, Front fr, A
                     }
                 } else {  // ring full: the grid-wide hub queue takes them
                     const unsigned long long old = atomicAdd(c.hub_ctr, (1ull << 32) | (unsigned long long)push_n);
-                    c.hubq[old >> 32] = HubEntry{push_base, u, (uint32_t)(old & 0xffffffffu)};
+                    publish_hub(c.hubq, old >> 32, push_base, u, (uint32_t)(old & 0xffffffffu), cur_epoch(c));
                 }
                 push_n = 0;
             }
@@ -715,7 +927,7 @@ __global__ void __launch_bounds__(kBlock, 4) sm_expand_kernel(Ctx c, Front fr, A
                     state = ST_DONE;
                     if (nseg > c.hub_segs) {
                         const unsigned long long old = atomicAdd(c.hub_ctr, (1ull << 32) | (unsigned long long)nseg);
-                        c.hubq[old >> 32] = HubEntry{bb.pos(), u, (uint32_t)(old & 0xffffffffu)};
+                        publish_hub(c.hubq, old >> 32, bb.pos(), u, (uint32_t)(old & 0xffffffffu), cur_epoch(c));
                     } else if (nseg) {
                         push_n = nseg;
                         push_base = bb.pos();
@@ -781,40 +993,67 @@ __global__ void __launch_bounds__(kBlock, 4) sm_expand_kernel(Ctx c, Front fr, A
     }
 }
 
+// Entry of flattened item j in a queue ordered by offset (HubEntry::seg_off / LongRange::chunk_off), found by the
+// whole warp at once: a 32-ary search for the warp's first item jb (ballot over 32 probes per round, ~log32(ne)
+// dependent loads instead of ~log2(ne)), then each lane walks forward to its own item (entries hold >= 5 items).
+__device__ __forceinline__ uint32_t item_off(const HubEntry* e) { return e->seg_off; }
+__device__ __forceinline__ uint32_t item_off(const LongRange* e) { return e->chunk_off; }
+template <class E>
+__device__ __forceinline__ uint32_t warp_find_item(const E* __restrict__ q, uint32_t ne, uint32_t jb, uint32_t j) {
+    const uint32_t lane = lane_id();
+    uint32_t lo = 0, hi = ne;  // invariant: off[lo] <= jb, and off[hi] > jb if hi < ne
+    while (hi - lo > 1) {
+        const uint32_t span = hi - lo;
+        const uint32_t pos = span <= 32 ? lo + lane : lo + (uint32_t)(((uint64_t)span * lane) >> 5);
+        const bool le = (span > 32 || lane < span) && item_off(q + pos) <= jb;
+        const uint32_t L = 31 - __clz(__ballot_sync(0xffffffffu, le));
+        if (span <= 32) {
+            lo += L;
+            break;
+        }
+        const uint32_t nlo = lo + (uint32_t)(((uint64_t)span * L) >> 5);
+        hi = L == 31 ? hi : lo + (uint32_t)(((uint64_t)span * (L + 1)) >> 5);
+        lo = nlo;
+    }
+    uint32_t e = lo;
+    while (e + 1 < ne && item_off(q + e + 1) <= j) e++;
+    return e;
+}
+
 // Hub segments of the level, flattened over the whole grid (one segment per thread at a time).
 template <int K, bool STAGED, class App>
 __device__ __forceinline__ void hub_phase(const Ctx& c, const App& app, uint64_t& na) {
+    const uint32_t lane = lane_id();
+    const uint64_t gw0 = ((uint64_t)blockIdx.x * blockDim.x + threadIdx.x) & ~31ull;
+    const uint64_t stride = (uint64_t)gridDim.x * blockDim.x;
     if (c.lr_ctr) {  // long intervals: one lr_chunk-id piece per thread
         const unsigned long long lc = *(volatile unsigned long long*)c.lr_ctr;
         const uint32_t ne = (uint32_t)(lc >> 32), nchunks = (uint32_t)(lc & 0xffffffffu);
-        for (uint64_t j = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; j < nchunks;
-             j += (uint64_t)gridDim.x * blockDim.x) {
-            uint32_t lo = 0, hi = ne - 1;
-            while (lo < hi) {
-                const uint32_t mid = (lo + hi + 1) >> 1;
-                if (c.lrq[mid].chunk_off <= j) lo = mid; else hi = mid - 1;
+        for (uint64_t jb = gw0; jb < nchunks; jb += stride) {
+            const uint32_t j = (uint32_t)jb + lane;
+            const uint32_t k = warp_find_item(c.lrq, ne, (uint32_t)jb, min(j, nchunks - 1));
+            if (j < nchunks) {
+                const LongRange e = c.lrq[k];
+                const uint32_t off = (j - e.chunk_off) * c.lr_chunk;
+                App t = app;
+                t.begin(e.u);
+                t.range(e.start + off, min(c.lr_chunk, e.len - off));
+                t.end();
             }
-            const LongRange e = c.lrq[lo];
-            const uint32_t off = (uint32_t)(j - e.chunk_off) * c.lr_chunk;
-            App t = app;
-            t.begin(e.u);
-            t.range(e.start + off, min(c.lr_chunk, e.len - off));
-            t.end();
         }
     }
     const unsigned long long hc = *(volatile unsigned long long*)c.hub_ctr;
     const uint32_t nh = (uint32_t)(hc >> 32), S = (uint32_t)(hc & 0xffffffffu);
-    for (uint64_t j = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; j < S; j += (uint64_t)gridDim.x * blockDim.x) {
-        uint32_t lo = 0, hi = nh - 1;  // entry: largest e with seg_off <= j
-        while (lo < hi) {
-            const uint32_t mid = (lo + hi + 1) >> 1;
-            if (c.hubq[mid].seg_off <= j) lo = mid; else hi = mid - 1;
+    for (uint64_t jb = gw0; jb < S; jb += stride) {
+        const uint32_t j = (uint32_t)jb + lane;
+        const uint32_t k = warp_find_item(c.hubq, nh, (uint32_t)jb, min(j, S - 1));
+        if (j < S) {
+            const HubEntry e = c.hubq[k];
+            App t = app;
+            t.begin(e.u);
+            na += decode_segment<K, STAGED>(c.W, e.base + (j - e.seg_off) * (uint64_t)c.seg_bits, e.u, t);
+            t.end();
         }
-        const HubEntry e = c.hubq[lo];
-        App t = app;
-        t.begin(e.u);
-        na += decode_segment<K, STAGED>(c.W, e.base + (j - e.seg_off) * (uint64_t)c.seg_bits, e.u, t);
-        t.end();
     }
 }
 
@@ -1149,8 +1388,141 @@ __device__ __forceinline__ bool frontier_range(const uint32_t* __restrict__ F, u
     return false;
 }
 
+// In-record scan of one unvisited vertex v: true at the first in-neighbour in F.  Residual ids are decoded four at
+// a time and their four frontier probes issued together (one exit test per batch), so the probe latency is paid
+// once per four arcs instead of once per arc.
 template <int K, bool SEG>
-__global__ void __launch_bounds__(kBlock) bu_kernel(const uint64_t* __restrict__ W, const uint64_t* __restrict__ offs,
+__device__ __forceinline__ bool bu_scan(const uint64_t* __restrict__ W, const uint64_t* __restrict__ offs,
+                                        uint32_t min_len, uint32_t seg_bits, const uint32_t* __restrict__ F,
+                                        uint32_t v, uint32_t batch, uint64_t& na, uint64_t& nb) {
+    const uint64_t p0 = ldg64(offs + v);
+    BitBuf bb;
+    bb.init(W, p0);
+    uint64_t deg = 0, got = 0;
+    if (!SEG) deg = bb.template next<K>(W) - 1;
+    const uint64_t itv = bb.template next<K>(W) - 1;
+    uint32_t prev_end = 0;
+    bool found = false;
+    for (uint64_t i = 0; i < itv && !found; i++) {
+        const uint64_t g = bb.template next<K>(W);
+        const uint32_t len = (uint32_t)(bb.template next<K>(W) - 1) + min_len;
+        const uint32_t start = i == 0 ? (uint32_t)unmap_first(v, g) : prev_end + (uint32_t)g;
+        found = frontier_range(F, start, len);
+        prev_end = start + len - 1;
+        got += len;
+    }
+    // residuals: cnt ids starting with one anchored at v, four per probe batch
+    auto scan_res = [&](uint32_t cnt) {
+        uint32_t cur = 0;
+        for (uint32_t i = 0; i < cnt && !found; i += batch) {
+            const uint32_t k_n = min(batch, cnt - i);
+            uint32_t id[4];
+#pragma unroll
+            for (uint32_t k = 0; k < 4; k++) {
+                if (k < k_n) {
+                    const uint64_t c = bb.template next<K>(W);
+                    cur = (i + k == 0) ? (uint32_t)unmap_first(v, c) : cur + (uint32_t)c;
+                }
+                id[k] = cur;
+            }
+            uint32_t fw[4];
+#pragma unroll
+            for (uint32_t k = 0; k < 4; k++) fw[k] = k < k_n ? __ldg(F + (id[k] >> 5)) : 0u;
+#pragma unroll
+            for (uint32_t k = 0; k < 4; k++) found |= ((fw[k] >> (id[k] & 31)) & 1u) != 0;
+            got += k_n;
+        }
+    };
+    uint64_t pend;
+    if (found) {
+        pend = bb.pos();
+    } else if (!SEG) {
+        scan_res((uint32_t)(deg - got));
+        pend = bb.pos();
+    } else {
+        const uint64_t nseg = bb.template next<K>(W) - 1;
+        const uint64_t base = bb.pos();
+        pend = base;
+        for (uint64_t sg = 0; sg < nseg && !found; sg++) {
+            bb.init(W, base + sg * seg_bits);
+            scan_res((uint32_t)(bb.template next<K>(W) - 1));
+            pend = bb.pos();
+        }
+    }
+    na += got;
+    nb += pend - p0;
+    return found;
+}
+
+// A warp owns a chunk of 8 frontier words (256 vertices): the chunk's unvisited vertices are compacted and dealt to
+// the lanes round-robin (a lane per unvisited vertex, not per vertex id, so late levels with few unvisited
+// vertices still fill the warp); found vertices are collected in shared memory and the warp writes its 8 words of N
+// without atomics.
+constexpr uint32_t kBuWords = 8;
+template <int K, bool SEG>
+__global__ void __launch_bounds__(kBlock, 6) bu_kernel(const uint64_t* __restrict__ W, const uint64_t* __restrict__ offs,
+                                                    uint32_t min_len, uint32_t seg_bits, const uint32_t* __restrict__ V,
+                                                    const uint32_t* __restrict__ F, uint32_t* __restrict__ N,
+                                                    uint64_t n, uint64_t nw, const uint32_t* __restrict__ dir,
+                                                    Stats* st, uint32_t bw, uint32_t batch) {
+    if (*dir != 1) return;
+    __shared__ uint32_t found_s[kWarps][kBuWords], inc_s[kWarps][kBuWords], unv_s[kWarps][kBuWords];
+    const uint32_t lane = lane_id(), wid = threadIdx.x >> 5;
+    uint64_t nv = 0, na = 0, nb = 0;
+    const uint64_t nch = (nw + bw - 1) / bw;
+    for (uint64_t ch = ((uint64_t)blockIdx.x * blockDim.x + threadIdx.x) >> 5; ch < nch;
+         ch += ((uint64_t)gridDim.x * blockDim.x) >> 5) {
+        const uint64_t w0 = ch * bw;
+        uint32_t unv = 0;
+        if (lane < kBuWords) {
+            found_s[wid][lane] = 0;
+        }
+        if (lane < bw) {
+            const uint64_t w = w0 + lane, v0 = w * 32;
+            if (v0 < n) {
+                unv = ~__ldg(V + w);
+                if (n - v0 < 32) unv &= (1u << (n - v0)) - 1;
+            }
+        }
+        uint32_t cnt = lane < kBuWords ? __popc(unv) : 0, incl = cnt;
+        for (int o = 1; o < (int)kBuWords; o <<= 1) {
+            const uint32_t t = __shfl_up_sync(0xffffffffu, incl, o);
+            if (lane >= (uint32_t)o) incl += t;
+        }
+        const uint32_t total = __shfl_sync(0xffffffffu, incl, kBuWords - 1);
+        if (!total) continue;
+        if (lane < kBuWords) {
+            inc_s[wid][lane] = incl;
+            unv_s[wid][lane] = unv;
+        }
+        __syncwarp();
+        for (uint32_t r = lane; r < total; r += 32) {
+            // candidate r: word k with excl(k) <= r < incl(k)
+            uint32_t k = 0, ex = 0, bits = 0;
+#pragma unroll
+            for (uint32_t q = 0; q < kBuWords; q++) {
+                const uint32_t iq = inc_s[wid][q], bq = unv_s[wid][q];
+                const uint32_t eq = iq - __popc(bq);
+                if (r >= eq && r < iq) { k = q; ex = eq; bits = bq; }
+            }
+            const uint32_t bit = __fns(bits, 0, (int)(r - ex) + 1);
+            const uint32_t v = (uint32_t)((w0 + k) * 32 + bit);
+            nv++;
+            if (bu_scan<K, SEG>(W, offs, min_len, seg_bits, F, v, batch, na, nb)) atomicOr(&found_s[wid][k], 1u << bit);
+        }
+        __syncwarp();
+        if (lane < kBuWords) {
+            const uint32_t m = found_s[wid][lane];
+            if (m) N[w0 + lane] = m;
+        }
+        __syncwarp();
+    }
+    add_stats(st, nv, na, nb);
+}
+
+// Per-word variant (round 1): lane = vertex of the warp's 32-vertex word, one frontier probe per residual.
+template <int K, bool SEG>
+__global__ void __launch_bounds__(kBlock) bu_kernel1(const uint64_t* __restrict__ W, const uint64_t* __restrict__ offs,
                                                     uint32_t min_len, uint32_t seg_bits, const uint32_t* __restrict__ V,
                                                     const uint32_t* __restrict__ F, uint32_t* __restrict__ N,
                                                     uint64_t n, uint64_t nw, const uint32_t* __restrict__ dir,
@@ -1358,6 +1730,25 @@ __global__ void ck_count(const uint64_t* __restrict__ W, const uint64_t* __restr
     }
 }
 
+// Per-word index of the checkpoint table: wptr[w - w0] = number of table vertices below 32w, bits[w - w0] = which
+// of the word's 32 vertices are in the table.  A frontier vertex finds its table row with two independent loads
+// instead of a ~17-step dependent binary search over the sorted ids (the tail levels' critical path).
+__global__ void hv_index(const uint32_t* __restrict__ ids, uint32_t H, uint64_t w0, uint64_t nwl,
+                         uint32_t* __restrict__ wptr, uint32_t* __restrict__ bits) {
+    for (uint64_t i = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; i <= nwl; i += (uint64_t)gridDim.x * blockDim.x) {
+        const uint64_t v0 = (w0 + i) * 32;
+        uint32_t lo = 0, hi = H;
+        while (lo < hi) {
+            const uint32_t mid = (lo + hi) >> 1;
+            if (ids[mid] < v0) lo = mid + 1; else hi = mid;
+        }
+        wptr[i] = lo;
+        uint32_t b = 0;
+        for (uint32_t j = lo; j < H && ids[j] < v0 + 32; j++) b |= 1u << (ids[j] - v0);
+        if (i < nwl) bits[i] = b;
+    }
+}
+
 __global__ void ck_gather(uint32_t* __restrict__ ids, const uint32_t* __restrict__ cnt, uint32_t H, uint64_t lo,
                           uint32_t* __restrict__ out) {
     for (uint64_t h = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; h <= H; h += (uint64_t)gridDim.x * blockDim.x) {
@@ -1518,15 +1909,27 @@ inline cudaError_t launch_bfs_persistent(const gcgt_graph* g, cudaStream_t s, Ct
 
 template <int K, bool SEG>
 inline void launch_bu_k(const gcgt_graph* g, cudaStream_t s) {
-    static int per_sm = 0;
+    static int per_sm = 0, per_sm1 = 0;
     if (!per_sm) {
         cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per_sm, bu_kernel<K, SEG>, kBlock, 0);
+        cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per_sm1, bu_kernel1<K, SEG>, kBlock, 0);
         if (per_sm < 1) per_sm = 1;
+        if (per_sm1 < 1) per_sm1 = 1;
     }
-    const int grid = (int)std::max<uint64_t>(1, std::min<uint64_t>((g->nw + kWarps - 1) / kWarps,
+    if (g->bu_kernel == 1) {  // round-1 per-word kernel
+        const int grid = (int)std::max<uint64_t>(1, std::min<uint64_t>((g->nw + kWarps - 1) / kWarps,
+                                                                        (uint64_t)per_sm1 * g->num_sms));
+        bu_kernel1<K, SEG><<<grid, kBlock, 0, s>>>(g->inW, g->inOffs, g->P.min_interval_len,
+                                                   8 * g->P.residual_segment_len, g->V, g->F, g->N, g->n, g->nw,
+                                                   g->bstate, g->stats);
+        return;
+    }
+    const uint64_t chunks = (g->nw + g->bu_words - 1) / g->bu_words;
+    const int grid = (int)std::max<uint64_t>(1, std::min<uint64_t>((chunks + kWarps - 1) / kWarps,
                                                                     (uint64_t)per_sm * g->num_sms));
     bu_kernel<K, SEG><<<grid, kBlock, 0, s>>>(g->inW, g->inOffs, g->P.min_interval_len, 8 * g->P.residual_segment_len,
-                                              g->V, g->F, g->N, g->n, g->nw, g->bstate, g->stats);
+                                              g->V, g->F, g->N, g->n, g->nw, g->bstate, g->stats,
+                                              g->bu_words, g->bu_batch);
 }
 
 inline void launch_bu(const gcgt_graph* g, cudaStream_t s) {
@@ -1542,6 +1945,7 @@ inline void launch_bu(const gcgt_graph* g, cudaStream_t s) {
 
 template <class App>
 inline void launch_hub(const gcgt_params& P, bool staged, int grid, cudaStream_t s, const Ctx& c, const App& app) {
+    if (c.fuse) return;  // drained inside expand_kernel
     if (!P.residual_segment_len && !c.hv_n && !c.lr_ctr) return;
 #define GCGT_HUB(KK)                                                            \
     (staged ? hub_kernel<KK, true, App><<<grid, kBlock, 0, s>>>(c, app)         \
@@ -1577,8 +1981,9 @@ inline Ctx make_ctx(const gcgt_graph* g) {
     return Ctx{g->W,     g->offs,     g->P.min_interval_len, 8 * g->P.residual_segment_len,
                g->hubq, g->hub_ctr, g->stats,              g->cursor,
                g->heavyq, g->heavy_len, g->heavy_itv, g->heavy_res, g->hub_segs, g->engine, nullptr,
-               g->hv_n,  g->ck_c,      g->hv_ids,    g->hv_ptr,    g->hv_after, g->hv_rem, g->ck_pos, g->ck_prev,
-               g->lrq,   g->lr_ctr,    g->long_len,  g->lr_chunk};
+               g->hv_n,  g->ck_c,      g->hv_ids,    g->hv_ptr,    g->hv_wptr, g->hv_bits, g->lo >> 5, g->hv_after, g->hv_rem, g->ck_pos, g->ck_prev,
+               g->lrq,   g->lr_ctr,    g->long_len,  g->lr_chunk,
+               (!heavy_active(g) && g->engine == 0 && g->fuse_ctr) ? g->fuse_warps : 0u, g->fuse_ctr, g->flatb};
 }
 
 gcgt_status copy_out(gcgt_graph* g, void* dst, const void* src, size_t bytes, int placement) {
@@ -1659,6 +2064,23 @@ gcgt_status galloc(const gcgt_graph* g, T** p, uint64_t count) {
 
 }  // namespace
 
+// Host-resident CGR words (§8 f4): a pinned, mapped host buffer holding words [w0, w0 + nwords) of the canonical
+// stream, byte-swapped on the host into the device's stream-word order; *dev is its device alias.  The kernels then
+// decode straight from host memory over the host link (the paper's out-of-core motivation, PAPER.md:93-120,
+// :474-479: graphs whose CGR exceeds device memory), while every O(n) table stays in HBM.
+gcgt_status host_words(gcgt_graph* g, uint64_t** host, uint64_t** dev, const std::vector<uint64_t>& words,
+                       uint64_t w0, uint64_t nwords) {
+    (void)g;
+    CU(cudaHostAlloc((void**)host, nwords * sizeof(uint64_t), cudaHostAllocMapped | cudaHostAllocPortable));
+    uint64_t* h = *host;
+    const uint64_t avail = words.size() > w0 ? words.size() - w0 : 0;
+#pragma omp parallel for schedule(static)
+    for (int64_t i = 0; i < (int64_t)nwords; i++)
+        h[i] = (uint64_t)i < avail ? __builtin_bswap64(words[w0 + i]) : 0;
+    CU(cudaHostGetDevicePointer((void**)dev, h, 0));
+    return GCGT_OK;
+}
+
 // Builds the interval checkpoint table (see ck_count / ck_fill) and the per-level chunk queue.
 gcgt_status build_checkpoints(gcgt_graph* g) {
     gcgt_status st;
@@ -1726,6 +2148,9 @@ gcgt_status build_checkpoints(gcgt_graph* g) {
         }
 #undef GCGT_CF
         g->hv_n = H;
+        const uint64_t w0 = g->lo >> 5, nwl = ((g->hi + 31) >> 5) - w0;
+        if ((st = galloc(g, &g->hv_wptr, nwl + 1)) || (st = galloc(g, &g->hv_bits, nwl + 1))) return st;
+        hv_index<<<flat_grid(g, nwl + 1), kBlock, 0, s>>>(g->hv_ids, H, w0, nwl, g->hv_wptr, g->hv_bits);
     }
     cudaFreeAsync(flag, s);
     cudaFreeAsync(cnt, s);
@@ -1743,11 +2168,11 @@ gcgt_status build_checkpoints(gcgt_graph* g) {
 extern "C" void gcgt_unload(gcgt_graph* g) {
     if (!g) return;
     cudaSetDevice(g->device);
-    void* bufs[] = {g->W,      g->offs_alloc, g->V,      g->F,         g->N,        g->q,      g->qbits,
-                    g->ctr,    g->hubq,    g->hub_ctr, g->cursor,   g->heavyq,   g->heavy_len, g->stats,
+    void* bufs[] = {g->hostW ? nullptr : g->W, g->offs_alloc, g->V,      g->F,         g->N,        g->q,      g->qbits,
+                    g->ctr,    g->hubq,    g->hub_ctr, g->cursor, g->fuse_ctr,   g->heavyq,   g->heavy_len, g->stats,
                     g->levels, g->parent,  g->sigma,  g->delta,     g->bc,      g->bstate,
-                    g->hv_ids, g->hv_ptr,  g->hv_rem, g->ck_prev,   g->lr_ctr, g->hv_after, g->ck_pos, g->lrq,
-                    g->in_owned ? g->inW : nullptr, g->in_owned ? g->inOffs : nullptr,
+                    g->hv_ids, g->hv_ptr,  g->hv_rem, g->hv_wptr, g->hv_bits, g->ck_prev,   g->lr_ctr, g->hv_after, g->ck_pos, g->lrq,
+                    g->in_owned && !g->hostInW ? g->inW : nullptr, g->in_owned ? g->inOffs : nullptr,
                     g->crow,   g->ccol,    g->csr_hubq, g->mf,
                     g->csr_in_owned ? g->crow_in : nullptr, g->csr_in_owned ? g->ccol_in : nullptr};
     if (g->stream) {
@@ -1755,6 +2180,8 @@ extern "C" void gcgt_unload(gcgt_graph* g) {
             if (b) cudaFreeAsync(b, g->stream);
         cudaStreamSynchronize(g->stream);
     }
+    if (g->hostW) cudaFreeHost(g->hostW);
+    if (g->hostInW) cudaFreeHost(g->hostInW);
     if (g->h_ctr) cudaFreeHost(g->h_ctr);
     if (g->h_stats) cudaFreeHost(g->h_stats);
     if (g->ev0) cudaEventDestroy(g->ev0);
@@ -1809,6 +2236,11 @@ extern "C" gcgt_status gcgt_load(const gcgt_cgr* c, const gcgt_load_opts* opts, 
                 const unsigned long v = strtoul(kv.c_str() + e + 1, nullptr, 10);
                 if (k == "staged") g->staged = v != 0;
                 else if (k == "persistent") g->persistent = v != 0;
+                else if (k == "bu") g->bu_kernel = (uint32_t)(v == 2 ? 2 : 1);
+                else if (k == "bu_words") g->bu_words = (uint32_t)std::max(1ul, std::min(8ul, v));
+                else if (k == "bu_batch") g->bu_batch = (uint32_t)std::max(1ul, std::min(4ul, v));
+                else if (k == "flatb") g->flatb = (uint32_t)(v != 0);
+                else if (k == "fuse") g->fuse_warps = (uint32_t)std::min(8ul, v);
                 else if (k == "engine") g->engine = (uint32_t)v;
                 else if (k == "bu_alpha") g->bu_alpha = (uint32_t)v;
                 else if (k == "bu_beta") g->bu_beta = (uint32_t)v;
@@ -1844,12 +2276,14 @@ extern "C" gcgt_status gcgt_load(const gcgt_cgr* c, const gcgt_load_opts* opts, 
         g->hi = std::max(g->lo, bound(g->rank + 1));
         g->dir_opt_knob = false;  // bottom-up needs the whole in-CGR: top-down only when partitioned
     }
-    g->nw = (c->n + 31) / 32 + 1;
+    g->nw = ((c->n + 31) / 32 + 1 + 3) & ~3ull;  // padded to whole 16-byte groups (commit_phase)
     const uint64_t w0 = c->bit_offsets[g->lo] / 64;
     const uint64_t nwords = (c->bit_offsets[g->hi] + 63) / 64 - w0 + 2;
     const uint64_t nloc = g->hi - g->lo;
     gcgt_status st;
-    if ((st = galloc(g.get(), &g->W, nwords)) || (st = galloc(g.get(), &g->offs_alloc, nloc + 1)) || (st = galloc(g.get(), &g->V, g->nw)) ||
+    if ((o.host_resident ? (st = host_words(g.get(), &g->hostW, &g->W, c->words, w0, nwords))
+                         : (st = galloc(g.get(), &g->W, nwords))) ||
+        (st = galloc(g.get(), &g->offs_alloc, nloc + 1)) || (st = galloc(g.get(), &g->V, g->nw)) ||
         (st = galloc(g.get(), &g->F, g->nw)) || (st = galloc(g.get(), &g->N, g->nw)) || (st = galloc(g.get(), &g->ctr, 8)) ||
         (st = galloc(g.get(), &g->stats, 1)) || (st = galloc(g.get(), &g->levels, g->n)))
         return st;
@@ -1862,7 +2296,7 @@ extern "C" gcgt_status gcgt_load(const gcgt_cgr* c, const gcgt_load_opts* opts, 
     CU(cudaEventCreate(&g->kev0));
     CU(cudaEventCreate(&g->kev1));
     for (auto& e : g->sev) CU(cudaEventCreate(&e));
-    {
+    if (!o.host_resident) {
         const uint64_t avail = c->words.size() - w0;  // the host array holds >= 2 padding words
         CU(cudaMemsetAsync(g->W, 0, nwords * sizeof(uint64_t), g->stream));
         CU(cudaMemcpyAsync(g->W, c->words.data() + w0, std::min(nwords, avail) * sizeof(uint64_t),
@@ -1878,7 +2312,7 @@ extern "C" gcgt_status gcgt_load(const gcgt_cgr* c, const gcgt_load_opts* opts, 
         CU(cudaStreamSynchronize(g->stream));  // ro is a stack vector
     }
     g->offs = g->offs_alloc - g->lo;  // kernels index offs[u] with global vertex ids
-    bswap_words<<<flat_grid(g.get(), nwords), kBlock, 0, g->stream>>>(g->W, nwords);
+    if (!o.host_resident) bswap_words<<<flat_grid(g.get(), nwords), kBlock, 0, g->stream>>>(g->W, nwords);
     CU(cudaMemsetAsync(g->N, 0, g->nw * 4, g->stream));
     if ((st = galloc(g.get(), &g->bstate, 8)) || (st = galloc(g.get(), &g->mf, 1))) return st;
     CU(cudaMemsetAsync(g->mf, 0, 8, g->stream));
@@ -1890,11 +2324,16 @@ extern "C" gcgt_status gcgt_load(const gcgt_cgr* c, const gcgt_load_opts* opts, 
             ic->params.residual_segment_len != c->params.residual_segment_len)
             return fail(GCGT_EINVAL, "in_cgr must have the same n and parameters as the CGR");
         const uint64_t inwords = (ic->nbits + 63) / 64 + 2;
-        if ((st = galloc(g.get(), &g->inW, inwords)) || (st = galloc(g.get(), &g->inOffs, ic->n + 1))) return st;
+        if ((o.host_resident ? (st = host_words(g.get(), &g->hostInW, &g->inW, ic->words, 0, inwords))
+                             : (st = galloc(g.get(), &g->inW, inwords))) ||
+            (st = galloc(g.get(), &g->inOffs, ic->n + 1)))
+            return st;
         g->in_owned = true;
-        CU(cudaMemcpyAsync(g->inW, ic->words.data(), inwords * 8, cudaMemcpyHostToDevice, g->stream));
+        if (!o.host_resident) {
+            CU(cudaMemcpyAsync(g->inW, ic->words.data(), inwords * 8, cudaMemcpyHostToDevice, g->stream));
+            bswap_words<<<flat_grid(g.get(), inwords), kBlock, 0, g->stream>>>(g->inW, inwords);
+        }
         CU(cudaMemcpyAsync(g->inOffs, ic->bit_offsets.data(), (ic->n + 1) * 8, cudaMemcpyHostToDevice, g->stream));
-        bswap_words<<<flat_grid(g.get(), inwords), kBlock, 0, g->stream>>>(g->inW, inwords);
         g->dir_opt = o.direction_optimizing != 0;
     } else if (o.symmetric) {
         g->inW = g->W;
@@ -1902,8 +2341,15 @@ extern "C" gcgt_status gcgt_load(const gcgt_cgr* c, const gcgt_load_opts* opts, 
         g->dir_opt = o.direction_optimizing != 0;
     }
     g->dir_opt = g->dir_opt && g->dir_opt_knob;
-    if ((st = galloc(g.get(), &g->hub_ctr, 1)) || (st = galloc(g.get(), &g->cursor, 2))) return st;
+    if ((st = galloc(g.get(), &g->hub_ctr, 1)) || (st = galloc(g.get(), &g->cursor, 2)) ||
+        (st = galloc(g.get(), &g->fuse_ctr, 4)))
+        return st;
     CU(cudaMemsetAsync(g->cursor, 0, 16, g->stream));
+    {  // epoch 1: queue entries start zeroed (epoch 0), so no stale entry can look published
+        const uint32_t init[4] = {0, 0, 0, 1};
+        CU(cudaMemcpyAsync(g->fuse_ctr, init, 16, cudaMemcpyHostToDevice, g->stream));
+        CU(cudaStreamSynchronize(g->stream));
+    }
     unsigned long long* dcount = nullptr;
     if ((st = galloc(g.get(), &dcount, 3))) return st;
     CU(cudaMemsetAsync(dcount, 0, 24, g->stream));
@@ -1927,8 +2373,10 @@ extern "C" gcgt_status gcgt_load(const gcgt_cgr* c, const gcgt_load_opts* opts, 
     if ((st = galloc(g.get(), &g->heavyq, nheavy + 1)) || (st = galloc(g.get(), &g->heavy_len, 1))) return st;
     CU(cudaMemsetAsync(g->heavy_len, 0, 4, g->stream));
     if ((st = galloc(g.get(), &g->hubq, nhubs + nheavy + 1))) return st;
+    CU(cudaMemsetAsync(g->hubq, 0, (nhubs + nheavy + 1) * sizeof(HubEntry), g->stream));
     if ((st = build_checkpoints(g.get()))) return st;
     if ((st = galloc(g.get(), &g->lrq, nlong + 1))) return st;
+    CU(cudaMemsetAsync(g->lrq, 0, (nlong + 1) * sizeof(LongRange), g->stream));
     CU(cudaMemsetAsync(g->hub_ctr, 0, 8, g->stream));
     CU(cudaStreamSynchronize(g->stream));
     CU(cudaGetLastError());
@@ -1982,7 +2430,7 @@ extern "C" gcgt_status gcgt_load_csr(const gcgt_csr* csr, const gcgt_load_opts* 
     g->n = n;
     g->lo = 0;
     g->hi = n;
-    g->nw = (n + 31) / 32 + 1;
+    g->nw = ((n + 31) / 32 + 1 + 3) & ~3ull;
     cudaStream_t s = g->stream;
     gcgt_status st;
     if ((st = galloc(g.get(), &g->crow, n + 1)) || (st = galloc(g.get(), &g->ccol, m)) ||

@@ -199,7 +199,10 @@ def test_warp_decoder_random_streams(k):
 # ---------------------------------------------------------------------------------------------------------------------
 # Direction-optimizing BFS (bottom-up levels over the in-CGR, §8 a9)
 # ---------------------------------------------------------------------------------------------------------------------
-@pytest.mark.parametrize("tune", ["", "bu_alpha=100000,bu_beta=1", "bu_alpha=100000,bu_beta=100000", "wpb_max=2"])
+@pytest.mark.parametrize("tune", ["", "bu_alpha=100000,bu_beta=1", "bu_alpha=100000,bu_beta=100000", "wpb_max=2",
+                                  "bu_alpha=100000,bu_beta=1,bu=2,bu_words=1,bu_batch=1", "bu=2",
+                                  "bu_alpha=100000,bu_beta=1,bu=2,bu_words=3,bu_batch=2", "fuse=1", "fuse=4,wpb_max=1",
+                                  "flatb=1"])
 @pytest.mark.parametrize("name", ["c1", "rmat_s", "web_s", "social_s"])
 def test_bfs_direction_optimizing(name, tune, monkeypatch):
     """Symmetric graphs use the out-CGR as in-CGR; directed ones the encoded transpose.  The tunes force
@@ -262,3 +265,22 @@ def test_csr_baseline_hubs_and_errors():
     with pytest.raises(G.GcgtError) as e:
         g.bc([0])
     assert e.value.status == G.EINVAL
+
+
+# ---------------------------------------------------------------------------------------------------------------------
+# Host-resident CGR (§8 f4): the kernels decode from pinned, mapped host memory; results identical to the oracle
+# ---------------------------------------------------------------------------------------------------------------------
+@pytest.mark.parametrize("name", ["c1", "web_s", "social_s", "rmat_s"])
+def test_host_resident_cgr(name):
+    cfg = synth.CONFIGS[name]
+    ro, co = cfg.make()
+    p = (cfg.min_interval_len, cfg.residual_segment_len, cfg.zeta_k)
+    cgr = G.encode(ro, co, *p)
+    inc = None if cfg.symmetric else G.encode_transpose(ro, co, *p)
+    g = G.load(cgr, in_cgr=inc, symmetric=cfg.symmetric, host_resident=True)
+    for r in [0] + synth.pick_roots(ro, 3):
+        assert np.array_equal(g.bfs(r), O.bfs(ro, co, r)), (name, r)
+    assert np.array_equal(g.cc(), O.cc(ro, co)), name
+    src = synth.pick_roots(ro, 2)
+    check_bc(g.bc(src), O.bc(ro, co, src))
+    g.unload()

@@ -10,9 +10,9 @@ i=0
 while [ $# -ge 2 ]; do
   KRE=$1; SKIP=$2; shift 2; i=$((i+1))
   timeout 900 ncu --set full --clock-control none --import-source on --kernel-name-base demangled -k regex:"$KRE" -s $SKIP -c 1 \
-    -o gpurun_out/prof_${TAG}_$i python tools/prof_bfs.py --config $CFG --reps 1 > gpurun_out/prof_${TAG}_$i.log 2>&1
+    -o /tmp/prof_${TAG}_$i python tools/prof_bfs.py --config $CFG --reps 1 > gpurun_out/prof_${TAG}_$i.log 2>&1
   tail -2 gpurun_out/prof_${TAG}_$i.log
-  python tools/ncu_brief.py gpurun_out/prof_${TAG}_$i.ncu-rep > gpurun_out/ncu_${TAG}_$i.txt 2>&1
-  python tools/srcprof.py gpurun_out/prof_${TAG}_$i.ncu-rep 50 > gpurun_out/src_${TAG}_$i.txt 2>&1
+  python tools/ncu_brief.py /tmp/prof_${TAG}_$i.ncu-rep > gpurun_out/ncu_${TAG}_$i.txt 2>&1
+  python tools/srcprof.py /tmp/prof_${TAG}_$i.ncu-rep 50 > gpurun_out/src_${TAG}_$i.txt 2>&1
   head -45 gpurun_out/ncu_${TAG}_$i.txt
 done
