@@ -19,6 +19,7 @@
 #include <string.h>
 
 #include <algorithm>
+#include <chrono>
 #include <memory>
 #include <string>
 #include <type_traits>
@@ -1943,13 +1944,28 @@ inline void launch_bu(const gcgt_graph* g, cudaStream_t s) {
     }
 }
 
+// The hub pass is latency-bound (one segment's dependent codeword chain per thread): launch a full wave at the
+// kernel's occupancy rather than a fixed 4 blocks per SM (`grid` = 4 blocks per SM is the floor).
+template <int K, bool STAGED, class App>
+inline int hub_wave(int grid) {
+    static int wave = 0;
+    if (!wave) {
+        int dev = 0, sms = 0, per_sm = 0;
+        cudaGetDevice(&dev);
+        cudaDeviceGetAttribute(&sms, cudaDevAttrMultiProcessorCount, dev);
+        cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per_sm, hub_kernel<K, STAGED, App>, kBlock, 0);
+        wave = std::max(1, per_sm) * std::max(1, sms);
+    }
+    return std::max(grid, wave);
+}
+
 template <class App>
 inline void launch_hub(const gcgt_params& P, bool staged, int grid, cudaStream_t s, const Ctx& c, const App& app) {
     if (c.fuse) return;  // drained inside expand_kernel
     if (!P.residual_segment_len && !c.hv_n && !c.lr_ctr) return;
-#define GCGT_HUB(KK)                                                            \
-    (staged ? hub_kernel<KK, true, App><<<grid, kBlock, 0, s>>>(c, app)         \
-            : hub_kernel<KK, false, App><<<grid, kBlock, 0, s>>>(c, app))
+#define GCGT_HUB(KK)                                                                                   \
+    (staged ? hub_kernel<KK, true, App><<<hub_wave<KK, true, App>(grid), kBlock, 0, s>>>(c, app)         \
+            : hub_kernel<KK, false, App><<<hub_wave<KK, false, App>(grid), kBlock, 0, s>>>(c, app))
     switch (P.zeta_k) {
         case 1: GCGT_HUB(1); break;
         case 2: GCGT_HUB(2); break;
@@ -2044,6 +2060,23 @@ gcgt_status end_call(gcgt_graph* g, gcgt_stats* out, uint32_t iterations) {
     }
     return GCGT_OK;
 }
+
+// Wall-clock marks of load / unload phases on stderr when GCGT_TIMING is set (diagnostics for the bench's e2e leg).
+struct PhaseClock {
+    bool on = getenv("GCGT_TIMING") != nullptr;
+    const char* what;
+    std::chrono::steady_clock::time_point t0 = std::chrono::steady_clock::now(), t = t0;
+    explicit PhaseClock(const char* w) : what(w) {}
+    void mark(const char* phase, cudaStream_t s = nullptr) {
+        if (!on) return;
+        if (s) cudaStreamSynchronize(s);
+        const auto now = std::chrono::steady_clock::now();
+        fprintf(stderr, "[%s] %-18s %8.2f ms (total %8.2f)\n", what, phase,
+                std::chrono::duration<double, std::milli>(now - t).count(),
+                std::chrono::duration<double, std::milli>(now - t0).count());
+        t = now;
+    }
+};
 
 template <class T>
 gcgt_status dalloc(T** p, uint64_t count) {
@@ -2175,11 +2208,13 @@ extern "C" void gcgt_unload(gcgt_graph* g) {
                     g->in_owned && !g->hostInW ? g->inW : nullptr, g->in_owned ? g->inOffs : nullptr,
                     g->crow,   g->ccol,    g->csr_hubq, g->mf,
                     g->csr_in_owned ? g->crow_in : nullptr, g->csr_in_owned ? g->ccol_in : nullptr};
+    PhaseClock pc("unload");
     if (g->stream) {
         for (void* b : bufs)
             if (b) cudaFreeAsync(b, g->stream);
         cudaStreamSynchronize(g->stream);
     }
+    pc.mark("free+sync");
     if (g->hostW) cudaFreeHost(g->hostW);
     if (g->hostInW) cudaFreeHost(g->hostInW);
     if (g->h_ctr) cudaFreeHost(g->h_ctr);
@@ -2191,7 +2226,9 @@ extern "C" void gcgt_unload(gcgt_graph* g) {
     for (auto& e : g->sev)
         if (e) cudaEventDestroy(e);
     if (g->own_stream && g->stream) cudaStreamDestroy(g->stream);
+    pc.mark("host frees+events");
     delete g;
+    pc.mark("delete");
 }
 
 extern "C" gcgt_status gcgt_load(const gcgt_cgr* c, const gcgt_load_opts* opts, gcgt_graph** out) {
@@ -2276,6 +2313,7 @@ extern "C" gcgt_status gcgt_load(const gcgt_cgr* c, const gcgt_load_opts* opts, 
         g->hi = std::max(g->lo, bound(g->rank + 1));
         g->dir_opt_knob = false;  // bottom-up needs the whole in-CGR: top-down only when partitioned
     }
+    PhaseClock pc("load");
     g->nw = ((c->n + 31) / 32 + 1 + 3) & ~3ull;  // padded to whole 16-byte groups (commit_phase)
     const uint64_t w0 = c->bit_offsets[g->lo] / 64;
     const uint64_t nwords = (c->bit_offsets[g->hi] + 63) / 64 - w0 + 2;
@@ -2311,6 +2349,7 @@ extern "C" gcgt_status gcgt_load(const gcgt_cgr* c, const gcgt_load_opts* opts, 
         CU(cudaMemcpyAsync(g->offs_alloc, ro.data(), (nloc + 1) * sizeof(uint64_t), cudaMemcpyHostToDevice, g->stream));
         CU(cudaStreamSynchronize(g->stream));  // ro is a stack vector
     }
+    pc.mark("alloc+H2D cgr", g->stream);
     g->offs = g->offs_alloc - g->lo;  // kernels index offs[u] with global vertex ids
     if (!o.host_resident) bswap_words<<<flat_grid(g.get(), nwords), kBlock, 0, g->stream>>>(g->W, nwords);
     CU(cudaMemsetAsync(g->N, 0, g->nw * 4, g->stream));
@@ -2341,6 +2380,7 @@ extern "C" gcgt_status gcgt_load(const gcgt_cgr* c, const gcgt_load_opts* opts, 
         g->dir_opt = o.direction_optimizing != 0;
     }
     g->dir_opt = g->dir_opt && g->dir_opt_knob;
+    pc.mark("in-cgr", g->stream);
     if ((st = galloc(g.get(), &g->hub_ctr, 1)) || (st = galloc(g.get(), &g->cursor, 2)) ||
         (st = galloc(g.get(), &g->fuse_ctr, 4)))
         return st;
@@ -2369,17 +2409,20 @@ extern "C" gcgt_status gcgt_load(const gcgt_cgr* c, const gcgt_load_opts* opts, 
     CU(cudaMemcpyAsync(counts, dcount, 24, cudaMemcpyDeviceToHost, g->stream));
     CU(cudaStreamSynchronize(g->stream));
     cudaFreeAsync(dcount, g->stream);
+    pc.mark("count_special");
     const uint64_t nhubs = counts[0], nheavy = counts[1], nlong = counts[2];
     if ((st = galloc(g.get(), &g->heavyq, nheavy + 1)) || (st = galloc(g.get(), &g->heavy_len, 1))) return st;
     CU(cudaMemsetAsync(g->heavy_len, 0, 4, g->stream));
     if ((st = galloc(g.get(), &g->hubq, nhubs + nheavy + 1))) return st;
     CU(cudaMemsetAsync(g->hubq, 0, (nhubs + nheavy + 1) * sizeof(HubEntry), g->stream));
     if ((st = build_checkpoints(g.get()))) return st;
+    pc.mark("checkpoints", g->stream);
     if ((st = galloc(g.get(), &g->lrq, nlong + 1))) return st;
     CU(cudaMemsetAsync(g->lrq, 0, (nlong + 1) * sizeof(LongRange), g->stream));
     CU(cudaMemsetAsync(g->hub_ctr, 0, 8, g->stream));
     CU(cudaStreamSynchronize(g->stream));
     CU(cudaGetLastError());
+    pc.mark("end");
     *out = g.release();
     return GCGT_OK;
 }
