@@ -13,7 +13,7 @@ import os
 import numpy as np
 
 _HERE = os.path.dirname(os.path.abspath(__file__))
-LIB_PATH = os.path.join(_HERE, "libgcgt.so")
+LIB_PATH = os.environ.get("GCGT_LIB") or os.path.join(_HERE, "libgcgt.so")  # GCGT_LIB: A/B builds (tools/)
 
 OK, EINVAL, EUNSORTED, ERANGE, ESEGLEN, ENOMEM, ECUDA, ENCCL, EFORMAT = 0, -1, -2, -3, -4, -5, -6, -7, -8
 STATUS_NAMES = {0: "OK", -1: "EINVAL", -2: "EUNSORTED", -3: "ERANGE", -4: "ESEGLEN", -5: "ENOMEM", -6: "ECUDA",

@@ -172,6 +172,9 @@ struct gcgt_graph {
 namespace {
 
 constexpr int kBlock = 256;
+#ifndef GCGT_EXPAND_MINB
+#define GCGT_EXPAND_MINB 4  // resident expand blocks per SM the register budget is sized for (64 regs)
+#endif
 constexpr int kWarps = kBlock / 32;
 // A vertex with more residual segments than this is not expanded by its own warp: its segments go to the
 // level's hub queue and are spread over the whole grid (segment-level work stealing, the B200 analogue of the
@@ -724,7 +727,7 @@ __device__ __forceinline__ void hub_consume(const Ctx& c, const App& app, uint32
 }
 
 template <int K, bool SEG, class App, class Front, bool DEFER, bool STAGED>
-__global__ void __launch_bounds__(kBlock, 4) expand_kernel(Ctx c, Front fr, App app, uint32_t wpb) {
+__global__ void __launch_bounds__(kBlock, GCGT_EXPAND_MINB) expand_kernel(Ctx c, Front fr, App app, uint32_t wpb) {
     __shared__ WarpSmem smem[kWarps];
     if (c.dir && *c.dir) return;  // this BFS level runs bottom-up: no work, cursor untouched
     uint64_t nv = 0, na = 0, nb = 0;
