@@ -72,13 +72,15 @@ else:
     roots = synth.pick_roots(ro, arg or 8)
     deg = np.diff(ro.astype(np.int64))
     ms, edges = [], 0
-    lv = g.bfs(roots[0])
+    dlv = torch.empty(int(n), dtype=torch.int32, device="cuda")  # device output: device_ms excludes the D2H
+    g.bfs(roots[0], out=dlv)
     for r in roots:
-        lv = g.bfs(r)
+        g.bfs(r, out=dlv)
         ms.append(g.last_stats["device_ms"])
+        lv = dlv.cpu().numpy()
         e = int(deg[lv >= 0].sum())
         edges += e / 2 if cfg.symmetric else e
-    out.update({"roots": len(roots), "ms_per_bfs": float(np.mean(ms)),
-                "gteps": edges / (sum(ms) * 1e-3) / 1e9})
+    out.update({"roots": len(roots), "ms_per_bfs": float(np.mean(ms)), "ms_each": [round(x, 3) for x in ms],
+                "gteps": edges / (sum(ms) * 1e-3) / 1e9, "levels_on": "device"})
     out["parity_1_root"] = bool(np.array_equal(lv, O.bfs(ro, co, roots[-1])))
 print(json.dumps(out), flush=True)
