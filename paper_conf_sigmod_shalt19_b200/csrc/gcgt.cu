@@ -140,6 +140,7 @@ struct gcgt_graph {
     // deferring long interval areas to a separate pass costs more than the in-batch straggler it removes
     bool staged = false;
     bool persistent = false;
+    uint32_t nfilter = 0;     // BfsApp: filter claims on an L1 read of N before the atomic (GCGT_TUNE nfilter=1)
     uint32_t flatb = 0;       // phase B lane-refill loop (GCGT_TUNE flatb=1; measured no faster on C2, session 3)
     uint32_t fuse_warps = 0;  // fused hub consumption: consumer warps per expand block (GCGT_TUNE fuse=N; 0 = hub_kernel)
     bool dir_opt_knob = true;
@@ -1079,11 +1080,20 @@ struct BfsApp {
     uint32_t* __restrict__ N;
     int32_t* __restrict__ levels;
     int32_t level;
+    uint32_t nfilter = 0;  // 1: skip the atomic when a (possibly stale) L1 read of N already shows the bits set
     __device__ __forceinline__ void begin(uint32_t) {}
     __device__ __forceinline__ void end() {}
     __device__ __forceinline__ void vertex(uint32_t) {}  // levels are written when a vertex is discovered
+    // N is written concurrently: a plain (L1-cached, possibly stale) read can only under-report set bits, so
+    // filtering on it never drops a claim; it only saves L2 atomics on vertices already claimed this level
+    __device__ __forceinline__ static uint32_t ld_n(const uint32_t* p) {
+        uint32_t v;
+        asm volatile("ld.global.ca.u32 %0, [%1];" : "=r"(v) : "l"(p));
+        return v;
+    }
     __device__ __forceinline__ void claim(uint32_t w, uint32_t mask) {
-        const uint32_t cand = mask & ~__ldg(V + w);
+        uint32_t cand = mask & ~__ldg(V + w);
+        if (cand && nfilter) cand &= ~ld_n(N + w);
         if (cand) atomicOr(N + w, cand);
     }
     __device__ __forceinline__ void one(uint32_t v) { claim(v >> 5, 1u << (v & 31)); }
@@ -1092,6 +1102,11 @@ struct BfsApp {
         uint32_t m[4];
 #pragma unroll
         for (uint32_t k = 0; k < 4; k++) m[k] = k < n ? __ldg(V + (v[k] >> 5)) : 0xffffffffu;
+        if (nfilter) {
+#pragma unroll
+            for (uint32_t k = 0; k < 4; k++)
+                if (k < n && !(m[k] & (1u << (v[k] & 31)))) m[k] |= ld_n(N + (v[k] >> 5));
+        }
 #pragma unroll
         for (uint32_t k = 0; k < 4; k++) {
             const uint32_t bit = 1u << (v[k] & 31);
@@ -1966,9 +1981,8 @@ template <class App>
 inline void launch_hub(const gcgt_params& P, bool staged, int grid, cudaStream_t s, const Ctx& c, const App& app) {
     if (c.fuse) return;  // drained inside expand_kernel
     if (!P.residual_segment_len && !c.hv_n && !c.lr_ctr) return;
-#define GCGT_HUB(KK)                                                                                   \
-    (staged ? hub_kernel<KK, true, App><<<hub_wave<KK, true, App>(grid), kBlock, 0, s>>>(c, app)         \
-            : hub_kernel<KK, false, App><<<hub_wave<KK, false, App>(grid), kBlock, 0, s>>>(c, app))
+    (void)staged;  // hub segments always use the BitBuf reader (C3: hub pass 1.40 vs 2.05 ms; C2 unchanged)
+#define GCGT_HUB(KK) hub_kernel<KK, true, App><<<hub_wave<KK, true, App>(grid), kBlock, 0, s>>>(c, app)
     switch (P.zeta_k) {
         case 1: GCGT_HUB(1); break;
         case 2: GCGT_HUB(2); break;
@@ -2279,6 +2293,7 @@ extern "C" gcgt_status gcgt_load(const gcgt_cgr* c, const gcgt_load_opts* opts, 
                 else if (k == "bu") g->bu_kernel = (uint32_t)(v == 2 ? 2 : 1);
                 else if (k == "bu_words") g->bu_words = (uint32_t)std::max(1ul, std::min(8ul, v));
                 else if (k == "bu_batch") g->bu_batch = (uint32_t)std::max(1ul, std::min(4ul, v));
+                else if (k == "nfilter") g->nfilter = (uint32_t)(v != 0);
                 else if (k == "flatb") g->flatb = (uint32_t)(v != 0);
                 else if (k == "fuse") g->fuse_warps = (uint32_t)std::min(8ul, v);
                 else if (k == "engine") g->engine = (uint32_t)v;
@@ -2653,7 +2668,7 @@ gcgt_status csr_bfs(gcgt_graph* g, uint32_t source, int32_t* levels, int placeme
         for (uint32_t i = 0; i < nlev; i++, level++) {
             const int cur = level & 1, nxt = cur ^ 1;
             const QueueFront fr{q[cur], g->ctr + cur, g->F, nullptr};
-            const BfsApp app{g->V, g->N, g->levels, (int32_t)level};
+            const BfsApp app{g->V, g->N, g->levels, (int32_t)level, g->nfilter};
             if ((st = kprof_begin(g))) return st;
             if (g->profile) CU(cudaEventRecord(g->sev[0], s));
             csr_expand_kernel<QueueFront><<<egrid, kBlock, 0, s>>>(g->crow, g->ccol, fr, app, g->cursor, hubq,
@@ -2750,7 +2765,7 @@ extern "C" gcgt_status gcgt_bfs(gcgt_graph* g, uint32_t source, int32_t* levels,
             if (level == 0) wpb = 1;
             else wpb = 0;  // device-side sizing
             const QueueFront fr{q[cur], g->ctr + cur, g->F, nullptr};
-            const BfsApp app{g->V, g->N, g->levels, (int32_t)level};
+            const BfsApp app{g->V, g->N, g->levels, (int32_t)level, g->nfilter};
             // profiled span = the level's expansion: top-down kernel (+ heavy pass + hub segments) or bottom-up
             if ((st = kprof_begin(g))) return st;
             if (g->profile) CU(cudaEventRecord(g->sev[0], s));
