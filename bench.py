@@ -456,26 +456,35 @@ def measure_e2e(G, cgr, incgr, roots, edges_of_root, cfg, n, nbits, dev, local, 
         inwords = ((inb.value + 63) // 64 + 2) * 8
         reg += [(ib.value, inwords), (io.value, (n + 1) * 8)]
         h2d += inwords + (n + 1) * 8
+    codes = []
     for ptr, size in reg:
-        cudart.cudaHostRegister(ptr, size, 0)
+        codes.append(int(cudart.cudaHostRegister(ptr, size, 0)))
     levels = torch.empty(n, dtype=torch.int32).pin_memory()
     tot_e, tot_t = 0.0, 0.0
+    split = {"load_ms": [], "bfs_ms": [], "unload_ms": []}
     try:
         for i in range(steps):
             torch.cuda.synchronize()
             t0 = time.perf_counter()
             g = G.load(cgr, device=local, stream="torch", in_cgr=incgr, symmetric=cfg.symmetric)
+            t1 = time.perf_counter()
             r = roots[i % len(roots)]
             g.bfs(r, out=levels)
+            t2 = time.perf_counter()
             g.unload()
             torch.cuda.synchronize()
-            tot_t += time.perf_counter() - t0
+            t3 = time.perf_counter()
+            tot_t += t3 - t0
             tot_e += edges_of_root[r]
+            split["load_ms"].append(round((t1 - t0) * 1e3, 1))
+            split["bfs_ms"].append(round((t2 - t1) * 1e3, 1))
+            split["unload_ms"].append(round((t3 - t2) * 1e3, 1))
     finally:
-        for ptr, _ in reg:
-            cudart.cudaHostUnregister(ptr)
+        for (ptr, _), c in zip(reg, codes):
+            if c == 0:
+                cudart.cudaHostUnregister(ptr)
     return {"value": tot_e / tot_t / 1e9, "unit": "GTEPS", "h2d_bytes_per_step": int(h2d),
-            "d2h_bytes_per_step": int(4 * n),
+            "d2h_bytes_per_step": int(4 * n), "host_register_status": codes, "per_step": split,
             "note": "per step: gcgt_load (CGR + in-CGR + bit offsets H2D from pinned host memory, pool allocation) + "
                     "gcgt_bfs with a pinned host levels array + gcgt_unload; host wall clock"}
 

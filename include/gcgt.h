@@ -129,11 +129,13 @@ gcgt_status gcgt_load_csr(const gcgt_csr* csr, const gcgt_load_opts* opts, gcgt_
 void gcgt_unload(gcgt_graph* g);
 
 /* Enables (1) / disables (0) per-launch CUDA-event timing of the dominant kernel (fills gcgt_stats.kernel_ms).
- * Adds one event pair per launch; results are unchanged. */
+ * Adds one event pair per launch, read at the call's existing host syncs (the BFS level loop stays asynchronous);
+ * results are unchanged.  2 = also per-level spans (gcgt_profile_spans): the BFS level loop then waits per level. */
 gcgt_status gcgt_profile(gcgt_graph* g, int enable);
 
-/* With profiling on, the last gcgt_bfs call's device time split into spans (ms): [0] top-down expansion kernel(s),
- * [1] hub segments / interval chunks, [2] bottom-up kernel, [3] contraction + direction choice.  count <= 4. */
+/* With span profiling on (gcgt_profile(g, 2)), the last gcgt_bfs call's device time split into spans (ms): [0]
+ * top-down expansion kernel(s), [1] hub segments / interval chunks, [2] bottom-up kernel, [3] contraction +
+ * direction choice.  count <= 4. */
 gcgt_status gcgt_profile_spans(const gcgt_graph* g, double* ms, int count);
 
 /* Owned vertex range [*lo, *hi) of this rank (whole [0, n) on a single GPU). */

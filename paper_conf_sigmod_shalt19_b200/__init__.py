@@ -228,8 +228,10 @@ class Graph:
         self.n = cgr_n(cgr)
         self.last_stats: dict = {}
 
-    def profile(self, enable: bool = True):
-        _check(lib().gcgt_profile(self._h, 1 if enable else 0), "gcgt_profile")
+    def profile(self, enable: bool = True, spans: bool = False):
+        """Kernel timing (gcgt_stats.kernel_ms); spans=True also per-level spans (the level loop then waits per
+        level)."""
+        _check(lib().gcgt_profile(self._h, (2 if spans else 1) if enable else 0), "gcgt_profile")
 
     def profile_spans(self):
         """Last profiled gcgt_bfs split into spans (ms): expand, hub, bottom-up, contraction."""

@@ -140,6 +140,7 @@ struct gcgt_graph {
     // deferring long interval areas to a separate pass costs more than the in-batch straggler it removes
     bool staged = false;
     bool persistent = false;
+    uint32_t chunk = 4;       // BFS levels enqueued per host check of the queue length (GCGT_TUNE chunk=N)
     uint32_t nfilter = 0;     // BfsApp: filter claims on an L1 read of N before the atomic (GCGT_TUNE nfilter=1)
     uint32_t flatb = 0;       // phase B lane-refill loop (GCGT_TUNE flatb=1; measured no faster on C2, session 3)
     uint32_t fuse_warps = 0;  // fused hub consumption: consumer warps per expand block (GCGT_TUNE fuse=N; 0 = hub_kernel)
@@ -163,6 +164,10 @@ struct gcgt_graph {
     // profiling of the dominant kernel
     bool profile = false;
     cudaEvent_t kev0 = nullptr, kev1 = nullptr;
+    static constexpr int kKev = 64;           // event pairs: one per profiled launch between host syncs
+    cudaEvent_t kevp[2 * kKev] = {};
+    int kev_n = 0;
+    bool spans = false;  // per-level span events (profile mode 2): the level loop then waits per level
     cudaEvent_t sev[5] = {nullptr, nullptr, nullptr, nullptr, nullptr};  // span marks within a BFS level
     double span_ms[4] = {0, 0, 0, 0};  // expand(+heavy), hub, bottom-up, contraction (+decide)
     double kernel_ms = 0;
@@ -2028,20 +2033,33 @@ gcgt_status copy_out(gcgt_graph* g, void* dst, const void* src, size_t bytes, in
 #include "csr_bfs.cuh"
 
 // Brackets one launch of the dominant kernel when profiling (the caller syncs before reading).
+// Profiled launches record into a pool of event pairs (created on first use) and are read at the next host sync,
+// so timing does not force a per-level wait (the chunked BFS level loop keeps its asynchronous enqueue).
 inline gcgt_status kprof_begin(gcgt_graph* g) {
-    if (g->profile) CU(cudaEventRecord(g->kev0, g->stream));
+    if (!g->profile) return GCGT_OK;
+    if (g->kev_n >= gcgt_graph::kKev) return fail(GCGT_EINVAL, "too many profiled launches between syncs");
+    cudaEvent_t& e = g->kevp[2 * g->kev_n];
+    if (!e) CU(cudaEventCreate(&e));
+    CU(cudaEventRecord(e, g->stream));
     return GCGT_OK;
 }
 inline gcgt_status kprof_end(gcgt_graph* g) {
-    if (g->profile) CU(cudaEventRecord(g->kev1, g->stream));
+    if (!g->profile) return GCGT_OK;
+    cudaEvent_t& e = g->kevp[2 * g->kev_n + 1];
+    if (!e) CU(cudaEventCreate(&e));
+    CU(cudaEventRecord(e, g->stream));
+    g->kev_n++;
     return GCGT_OK;
 }
 inline gcgt_status kprof_collect(gcgt_graph* g) {  // after a stream sync
     if (!g->profile) return GCGT_OK;
-    float ms = 0;
-    CU(cudaEventElapsedTime(&ms, g->kev0, g->kev1));
-    g->kernel_ms += ms;
-    g->kernel_launches++;
+    for (int i = 0; i < g->kev_n; i++) {
+        float ms = 0;
+        CU(cudaEventElapsedTime(&ms, g->kevp[2 * i], g->kevp[2 * i + 1]));
+        g->kernel_ms += ms;
+        g->kernel_launches++;
+    }
+    g->kev_n = 0;
     return GCGT_OK;
 }
 
@@ -2238,6 +2256,8 @@ extern "C" void gcgt_unload(gcgt_graph* g) {
     if (g->h_stats) cudaFreeHost(g->h_stats);
     if (g->ev0) cudaEventDestroy(g->ev0);
     if (g->ev1) cudaEventDestroy(g->ev1);
+    for (auto& e : g->kevp)
+        if (e) cudaEventDestroy(e);
     if (g->kev0) cudaEventDestroy(g->kev0);
     if (g->kev1) cudaEventDestroy(g->kev1);
     for (auto& e : g->sev)
@@ -2293,6 +2313,7 @@ extern "C" gcgt_status gcgt_load(const gcgt_cgr* c, const gcgt_load_opts* opts, 
                 else if (k == "bu") g->bu_kernel = (uint32_t)(v == 2 ? 2 : 1);
                 else if (k == "bu_words") g->bu_words = (uint32_t)std::max(1ul, std::min(8ul, v));
                 else if (k == "bu_batch") g->bu_batch = (uint32_t)std::max(1ul, std::min(4ul, v));
+                else if (k == "chunk") g->chunk = (uint32_t)std::max(1ul, std::min(64ul, v));
                 else if (k == "nfilter") g->nfilter = (uint32_t)(v != 0);
                 else if (k == "flatb") g->flatb = (uint32_t)(v != 0);
                 else if (k == "fuse") g->fuse_warps = (uint32_t)std::min(8ul, v);
@@ -2617,6 +2638,8 @@ extern "C" gcgt_status gcgt_debug_warp_decode(const uint8_t* bytes, uint64_t nbi
 extern "C" gcgt_status gcgt_profile(gcgt_graph* g, int enable) {
     if (!g) return fail(GCGT_EINVAL, "null graph");
     g->profile = enable != 0;
+    g->spans = enable >= 2;
+    g->kev_n = 0;
     return GCGT_OK;
 }
 
@@ -2662,25 +2685,24 @@ gcgt_status csr_bfs(gcgt_graph* g, uint32_t source, int32_t* levels, int placeme
     uint64_t qlen = 1;
     uint32_t level = 0;
     gcgt_status st;
-    constexpr uint32_t kChunk = 4;
     while (qlen) {
-        const uint32_t nlev = g->profile ? 1 : kChunk;
+        const uint32_t nlev = g->spans ? 1 : std::min<uint32_t>(g->chunk, gcgt_graph::kKev);
         for (uint32_t i = 0; i < nlev; i++, level++) {
             const int cur = level & 1, nxt = cur ^ 1;
             const QueueFront fr{q[cur], g->ctr + cur, g->F, nullptr};
             const BfsApp app{g->V, g->N, g->levels, (int32_t)level, g->nfilter};
             if ((st = kprof_begin(g))) return st;
-            if (g->profile) CU(cudaEventRecord(g->sev[0], s));
+            if (g->spans) CU(cudaEventRecord(g->sev[0], s));
             csr_expand_kernel<QueueFront><<<egrid, kBlock, 0, s>>>(g->crow, g->ccol, fr, app, g->cursor, hubq,
                                                                     g->hub_ctr, g->dir_opt ? g->bstate : nullptr,
                                                                     g->stats);
-            if (g->profile) CU(cudaEventRecord(g->sev[1], s));
+            if (g->spans) CU(cudaEventRecord(g->sev[1], s));
             csr_hub_kernel<<<hub_grid(g), kBlock, 0, s>>>(g->ccol, hubq, g->hub_ctr, app, g->stats);
-            if (g->profile) CU(cudaEventRecord(g->sev[2], s));
+            if (g->spans) CU(cudaEventRecord(g->sev[2], s));
             if (g->dir_opt)
                 csr_bu_kernel<<<bgrid, kBlock, 0, s>>>(g->crow_in, g->ccol_in, g->V, g->F, g->N, g->n, g->bstate,
                                                         g->stats);
-            if (g->profile) CU(cudaEventRecord(g->sev[3], s));
+            if (g->spans) CU(cudaEventRecord(g->sev[3], s));
             if ((st = kprof_end(g))) return st;
             commit_dense<<<flat_grid(g, g->nw), kBlock, 0, s>>>(g->V, g->F, g->N, 0, g->nw, q[nxt], g->ctr + nxt,
                                                                  nullptr, g->ctr + cur, g->hub_ctr, nullptr,
@@ -2691,7 +2713,7 @@ gcgt_status csr_bfs(gcgt_graph* g, uint32_t source, int32_t* levels, int placeme
                            g->dir_bits && g->dir_opt ? g->mf : nullptr,
                            (double)g->nbits / (double)std::max<uint64_t>(1, g->n), g->alpha_bits, g->ctr + 7});
             g->launches += 3 + (g->dir_opt ? 1 : 0);
-            if (g->profile) {
+            if (g->spans) {
                 CU(cudaEventRecord(g->sev[4], s));
                 CU(cudaEventSynchronize(g->sev[4]));
                 for (int k = 0; k < 4; k++) {
@@ -2754,9 +2776,8 @@ extern "C" gcgt_status gcgt_bfs(gcgt_graph* g, uint32_t source, int32_t* levels,
     // length, so the host enqueues kChunk levels at a time and checks for an empty queue once per chunk (levels
     // enqueued past the end find an empty queue and exit at once).  With profiling on, the loop waits per level to
     // time the expansion kernel.
-    constexpr uint32_t kChunk = 4;
     while (qlen) {
-        const uint32_t nlev = g->profile ? 1 : kChunk;
+        const uint32_t nlev = g->spans ? 1 : std::min<uint32_t>(g->chunk, gcgt_graph::kKev);
         for (uint32_t i = 0; i < nlev; i++, level++) {
             const int cur = level & 1, nxt = cur ^ 1;
             int grid;
@@ -2768,14 +2789,14 @@ extern "C" gcgt_status gcgt_bfs(gcgt_graph* g, uint32_t source, int32_t* levels,
             const BfsApp app{g->V, g->N, g->levels, (int32_t)level, g->nfilter};
             // profiled span = the level's expansion: top-down kernel (+ heavy pass + hub segments) or bottom-up
             if ((st = kprof_begin(g))) return st;
-            if (g->profile) CU(cudaEventRecord(g->sev[0], s));
+            if (g->spans) CU(cudaEventRecord(g->sev[0], s));
             launch_expand(g->P, g->staged, grid, s, c, fr, app, wpb);
             launch_heavy(g, s, c, app);
-            if (g->profile) CU(cudaEventRecord(g->sev[1], s));
+            if (g->spans) CU(cudaEventRecord(g->sev[1], s));
             launch_hub(g->P, g->staged, hub_grid(g), s, c, app);
-            if (g->profile) CU(cudaEventRecord(g->sev[2], s));
+            if (g->spans) CU(cudaEventRecord(g->sev[2], s));
             if (g->dir_opt) launch_bu(g, s);
-            if (g->profile) CU(cudaEventRecord(g->sev[3], s));
+            if (g->spans) CU(cudaEventRecord(g->sev[3], s));
             if ((st = kprof_end(g))) return st;
             commit_dense<<<flat_grid(g, g->nw), kBlock, 0, s>>>(g->V, g->F, g->N, 0, g->nw, q[nxt], g->ctr + nxt,
                                                                  nullptr, g->ctr + cur, g->hub_ctr, g->heavy_len,
@@ -2785,7 +2806,7 @@ extern "C" gcgt_status gcgt_bfs(gcgt_graph* g, uint32_t source, int32_t* levels,
                 DecideArgs{g->bstate, g->n, g->bu_alpha, g->bu_beta, g->dir_opt ? 1 : 0, g->ctr + nxt, g->ctr + 6,
                            g->dir_bits && g->dir_opt ? g->mf : nullptr,
                            (double)g->nbits / (double)std::max<uint64_t>(1, g->n), g->alpha_bits, g->ctr + 7});
-            if (g->profile) {  // profiling waits per level anyway (nlev = 1)
+            if (g->spans) {  // span profiling waits per level (nlev = 1)
                 CU(cudaEventRecord(g->sev[4], s));
                 CU(cudaEventSynchronize(g->sev[4]));
                 float lms[4];

@@ -22,7 +22,7 @@ for tune in tunes:
     g = G.load(cgr, stream="torch", in_cgr=incgr, symmetric=cfg.symmetric)
     for r in roots[:2]:
         g.bfs(r, out=out)
-    g.profile(True)
+    g.profile(True, spans=True)
     t = 0.0
     k = 0.0
     spans = {}

@@ -20,7 +20,7 @@ g = G.load(G.encode(ro, co, *P), stream="torch", in_cgr=incgr, symmetric=cfg.sym
 roots = synth.pick_roots(ro, 16)
 out = torch.empty(ro.size - 1, dtype=torch.int32, device="cuda")
 g.bfs(roots[0], out=out)  # warm
-g.profile(True)
+g.profile(True, spans=True)
 for i in range(nroots):
     print(f"# root {roots[i]}", file=sys.stderr, flush=True)
     g.bfs(roots[i], out=out)
