@@ -463,6 +463,10 @@ def measure_e2e(G, cgr, incgr, roots, edges_of_root, cfg, n, nbits, dev, local, 
     tot_e, tot_t = 0.0, 0.0
     split = {"load_ms": [], "bfs_ms": [], "unload_ms": []}
     try:
+        # one untimed warm-up cycle: the first load grows the device memory pool (kept afterwards, as in a service)
+        g = G.load(cgr, device=local, stream="torch", in_cgr=incgr, symmetric=cfg.symmetric)
+        g.bfs(roots[0], out=levels)
+        g.unload()
         for i in range(steps):
             torch.cuda.synchronize()
             t0 = time.perf_counter()
@@ -485,7 +489,8 @@ def measure_e2e(G, cgr, incgr, roots, edges_of_root, cfg, n, nbits, dev, local, 
                 cudart.cudaHostUnregister(ptr)
     return {"value": tot_e / tot_t / 1e9, "unit": "GTEPS", "h2d_bytes_per_step": int(h2d),
             "d2h_bytes_per_step": int(4 * n), "host_register_status": codes, "per_step": split,
-            "note": "per step: gcgt_load (CGR + in-CGR + bit offsets H2D from pinned host memory, pool allocation) + "
+            "note": "per step (after 1 untimed warm-up cycle): gcgt_load (CGR + in-CGR + bit offsets H2D from pinned "
+                    "host memory, pool allocation) + "
                     "gcgt_bfs with a pinned host levels array + gcgt_unload; host wall clock"}
 
 
