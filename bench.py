@@ -274,6 +274,7 @@ def main():
     evs = [(torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)) for _ in range(args.steps)]
     clocks = ClockSampler(local, dev)
     tot = {"arcs": 0, "bits": 0, "vertices": 0, "levels": 0, "kms": 0.0, "klaunch": 0, "launches": 0, "edges": 0.0}
+    step_edges = []
     if ws > 1:
         dist.barrier()
     torch.cuda.synchronize()
@@ -285,6 +286,7 @@ def main():
         g.bfs(r, out=levels)
         evs[i][1].record(stream)
         tot["edges"] += edges_of_root[r]
+        step_edges.append(edges_of_root[r])
         st = g.last_stats
         tot["launches"] += st["launches"]
         tot["arcs"] += st["arcs_decoded"]
@@ -298,8 +300,10 @@ def main():
         dist.barrier()
     ck = clocks.stop()
     g.profile(False)
-    t_ms = sum(a.elapsed_time(b) for a, b in evs)
+    step_ms = [a.elapsed_time(b) for a, b in evs]
+    t_ms = sum(step_ms)
     edges = tot["edges"]
+    per_root = [e / (t * 1e-3) / 1e9 for e, t in zip(step_edges, step_ms)]  # GTEPS of each timed BFS
     if ws > 1:
         tt = torch.tensor([t_ms], dtype=torch.float64, device=dev)
         dist.all_reduce(tt, op=dist.ReduceOp.MAX)
@@ -338,6 +342,8 @@ def main():
                            "zeta_k": cfg.zeta_k, "roots_per_rank": len(roots), "levels_per_bfs": tot["levels"] / args.steps,
                            "direction_optimizing": True, "in_cgr": "transpose" if incgr is not None else "symmetric",
                            "edges_per_bfs": edges / args.steps,
+                           "gteps_per_root_hmean": len(per_root) / sum(1.0 / x for x in per_root),
+                           "gteps_per_root_median": float(np.median(per_root)),
                            "l2": "flushed between steps (256 MiB fill, outside the per-step CUDA events)",
                            "parallelism": f"{ws} x independent BFS queries (replicas)" if ws > 1 else "1 GPU",
                            "gen_s": round(tgen, 1), "encode_s": round(tenc, 1)},
