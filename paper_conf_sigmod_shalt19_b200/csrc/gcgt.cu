@@ -149,7 +149,7 @@ struct gcgt_graph {
     uint32_t heavy_itv = 0xFFFFFFFFu, heavy_res = 1024, hub_segs = 8, wpb_max = 8;
     uint32_t bu_kernel = 1;  // bottom-up kernel: 1 = per-word (lane = vertex id), 2 = compacted chunks (bu_words/bu_batch)
     uint32_t bu_words = 8, bu_batch = 4;  // bottom-up: frontier words per warp chunk, residuals per probe batch
-    uint32_t bu_alpha = 4, bu_beta = 24;  // switch thresholds on vertex counts (C2/R-MAT/social sweep, r1)
+    uint32_t bu_alpha = 4, bu_beta = 128;  // switch thresholds on vertex counts (beta: r1 session-4 sweep, C2+C3)
     uint32_t* heavy_len = nullptr;
     unsigned long long* hub_ctr = nullptr;
     uint32_t* fuse_ctr = nullptr;  // fused hub consumption counters [4] (Ctx::fuse_ctr)
