@@ -21,6 +21,7 @@
 #include <algorithm>
 #include <chrono>
 #include <memory>
+#include <mutex>
 #include <string>
 #include <type_traits>
 #include <vector>
@@ -2108,6 +2109,29 @@ gcgt_status end_call(gcgt_graph* g, gcgt_stats* out, uint32_t iterations) {
     return GCGT_OK;
 }
 
+// Small pinned host blocks (per-graph counters and stats) are recycled process-wide: cudaFreeHost on every unload
+// measured 0.6 ms typical with stalls of 12-314 ms (tools/e2e_breakdown.py, session 4), inside the e2e step.
+static constexpr size_t kSmallPinned = 256;
+static std::mutex g_small_mu;
+static std::vector<void*> g_small_free;
+static cudaError_t small_pinned_get(void** p) {
+    {
+        std::lock_guard<std::mutex> lk(g_small_mu);
+        if (!g_small_free.empty()) {
+            *p = g_small_free.back();
+            g_small_free.pop_back();
+            return cudaSuccess;
+        }
+    }
+    return cudaMallocHost(p, kSmallPinned);
+}
+static void small_pinned_put(void* p) {
+    if (!p) return;
+    std::lock_guard<std::mutex> lk(g_small_mu);
+    g_small_free.push_back(p);
+}
+static_assert(sizeof(Stats) <= kSmallPinned && 8 * sizeof(uint32_t) <= kSmallPinned, "small pinned block size");
+
 // Wall-clock marks of load / unload phases on stderr when GCGT_TIMING is set (diagnostics for the bench's e2e leg).
 struct PhaseClock {
     bool on = getenv("GCGT_TIMING") != nullptr;
@@ -2264,8 +2288,8 @@ extern "C" void gcgt_unload(gcgt_graph* g) {
     pc.mark("free+sync");
     if (g->hostW) cudaFreeHost(g->hostW);
     if (g->hostInW) cudaFreeHost(g->hostInW);
-    if (g->h_ctr) cudaFreeHost(g->h_ctr);
-    if (g->h_stats) cudaFreeHost(g->h_stats);
+    small_pinned_put(g->h_ctr);
+    small_pinned_put(g->h_stats);
     if (g->ev0) cudaEventDestroy(g->ev0);
     if (g->ev1) cudaEventDestroy(g->ev1);
     for (auto& e : g->kevp)
@@ -2378,8 +2402,8 @@ extern "C" gcgt_status gcgt_load(const gcgt_cgr* c, const gcgt_load_opts* opts, 
         return st;
     g->qcap = 2 * g->nw;
     if ((st = galloc(g.get(), &g->q, g->qcap))) return st;
-    CU(cudaMallocHost((void**)&g->h_ctr, 8 * sizeof(uint32_t)));
-    CU(cudaMallocHost((void**)&g->h_stats, sizeof(Stats)));
+    CU(small_pinned_get((void**)&g->h_ctr));
+    CU(small_pinned_get((void**)&g->h_stats));
     CU(cudaEventCreate(&g->ev0));
     CU(cudaEventCreate(&g->ev1));
     CU(cudaEventCreate(&g->kev0));
@@ -2538,8 +2562,8 @@ extern "C" gcgt_status gcgt_load_csr(const gcgt_csr* csr, const gcgt_load_opts* 
         return st;
     g->qcap = 2 * g->nw;
     if ((st = galloc(g.get(), &g->q, g->qcap))) return st;
-    CU(cudaMallocHost((void**)&g->h_ctr, 8 * sizeof(uint32_t)));
-    CU(cudaMallocHost((void**)&g->h_stats, sizeof(Stats)));
+    CU(small_pinned_get((void**)&g->h_ctr));
+    CU(small_pinned_get((void**)&g->h_stats));
     CU(cudaEventCreate(&g->ev0));
     CU(cudaEventCreate(&g->ev1));
     CU(cudaEventCreate(&g->kev0));

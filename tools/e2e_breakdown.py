@@ -11,13 +11,16 @@ import synth  # noqa: E402
 
 cfg = synth.CONFIGS[sys.argv[1] if len(sys.argv) > 1 else "c2"]
 ro, co = cfg.make()
-cgr = G.encode(ro, co, cfg.min_interval_len, cfg.residual_segment_len, cfg.zeta_k)
+P = (cfg.min_interval_len, cfg.residual_segment_len, cfg.zeta_k)
+cgr = G.encode(ro, co, *P)
+incgr = None if cfg.symmetric else G.encode_transpose(ro, co, *P)  # as bench.py e2e
+iters = int(sys.argv[2]) if len(sys.argv) > 2 else 3
 root = synth.pick_roots(ro, 1)[0]
 levels = torch.empty(ro.size - 1, dtype=torch.int32).pin_memory()
-for i in range(3):
+for i in range(iters):
     torch.cuda.synchronize()
     t0 = time.perf_counter()
-    g = G.load(cgr, stream="torch")
+    g = G.load(cgr, stream="torch", in_cgr=incgr, symmetric=cfg.symmetric)
     torch.cuda.synchronize()
     t1 = time.perf_counter()
     g.bfs(root, out=levels)
