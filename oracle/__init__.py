@@ -13,6 +13,7 @@ import numpy as np
 
 _HERE = os.path.dirname(os.path.abspath(__file__))
 _SRC = os.path.join(_HERE, "gcgt_oracle.c")
+_SRC_PAR = os.path.join(_HERE, "gcgt_oracle_par.c")
 _LIB = os.path.join(_HERE, "liboracle.so")
 
 ERRORS = {0: "OK", -1: "EINVAL", -2: "EUNSORTED", -3: "ERANGE", -4: "ESEGLEN", -5: "ENOMEM", -8: "EFORMAT"}
@@ -25,9 +26,11 @@ class OracleError(RuntimeError):
 
 
 def build(force: bool = False) -> str:
-    """Compile the oracle (plain C, -O2, no OpenMP).  Building the checker is not using it."""
-    if force or not os.path.exists(_LIB) or os.path.getmtime(_LIB) < os.path.getmtime(_SRC):
-        subprocess.check_call(["gcc", "-O2", "-std=c11", "-fPIC", "-shared", "-Wall", "-o", _LIB, _SRC])
+    """Compile the oracle (plain C, -O2; OpenMP only in gcgt_oracle_par.c).  Building the checker is not using it."""
+    if (force or not os.path.exists(_LIB) or os.path.getmtime(_LIB) < os.path.getmtime(_SRC)
+            or os.path.getmtime(_LIB) < os.path.getmtime(_SRC_PAR)):
+        subprocess.check_call(["gcc", "-O2", "-std=c11", "-fPIC", "-shared", "-Wall", "-fopenmp", "-o", _LIB, _SRC,
+                               _SRC_PAR])
     return _LIB
 
 
@@ -55,6 +58,11 @@ def lib():
         L.orc_bfs_cgr.argtypes = [u64, p, p, u32, u32, u32, u64, p, C.POINTER(u64)]
         L.orc_cc.argtypes = [u64, p, p, p]
         L.orc_bc.argtypes = [u64, p, p, p, u64, p]
+        L.orc_bfs_cgr_par.argtypes = [u64, p, p, u32, u32, u32, u64, p, C.POINTER(u64), i32]
+        L.orc_bfs_par.argtypes = [u64, p, p, u64, p, i32]
+        L.orc_max_threads.restype = i32
+        L.orc_encode_par.argtypes = [u64, p, p, u32, u32, u32, C.POINTER(p), C.POINTER(u64), p, i32]
+        L.orc_bc_par.argtypes = [u64, p, p, p, u64, p, i32]
         _lib = L
     return _lib
 
@@ -147,6 +155,24 @@ def encode(rowoff, cols, min_interval_len=4, residual_segment_len=32, zeta_k=3):
     return out, int(nb.value), offs
 
 
+def encode_par(rowoff, cols, min_interval_len=4, residual_segment_len=32, zeta_k=3, threads: int = 0):
+    """Same output as encode(), records encoded per vertex in parallel and concatenated (gcgt_oracle_par.c)."""
+    rowoff, cols = _csr(rowoff, cols)
+    n = rowoff.size - 1
+    offs = np.zeros(n + 1, dtype=np.uint64)
+    bp = C.c_void_p()
+    nb = C.c_uint64(0)
+    st = lib().orc_encode_par(n, _ptr(rowoff), _ptr(cols), min_interval_len, residual_segment_len, zeta_k,
+                              C.byref(bp), C.byref(nb), _ptr(offs), threads)
+    if st != 0:
+        raise OracleError(st, "encode_par")
+    nbytes = (nb.value + 7) // 8
+    out = np.empty(max(nbytes, 1), dtype=np.uint8)
+    C.memmove(out.ctypes.data, bp.value, max(nbytes, 1))
+    lib().orc_free(bp)
+    return out[:nbytes], int(nb.value), offs
+
+
 def _padded(bytes_):
     b = np.zeros(np.asarray(bytes_).size + 16, dtype=np.uint8)
     b[: np.asarray(bytes_).size] = bytes_
@@ -218,6 +244,47 @@ def bfs_cgr(bytes_, bit_offsets, min_interval_len, residual_segment_len, zeta_k,
     if st != 0:
         raise OracleError(st, "bfs_cgr")
     return lv, int(e.value)
+
+
+def bfs_par(rowoff, cols, source: int, threads: int = 0) -> np.ndarray:
+    """Level-synchronous OpenMP BFS over the CSR (gcgt_oracle_par.c); threads = 0: all cores."""
+    rowoff, cols = _csr(rowoff, cols)
+    n = rowoff.size - 1
+    lv = np.zeros(n, dtype=np.int32)
+    st = lib().orc_bfs_par(n, _ptr(rowoff), _ptr(cols), source, _ptr(lv), threads)
+    if st != 0:
+        raise OracleError(st, "bfs_par")
+    return lv
+
+
+def bfs_cgr_par(bytes_, bit_offsets, min_interval_len, residual_segment_len, zeta_k, source: int, threads: int = 0):
+    """Level-synchronous OpenMP BFS decoding the oracle's own CGR; returns (levels, edges)."""
+    b = _padded(bytes_)
+    offs = np.ascontiguousarray(bit_offsets, dtype=np.uint64)
+    n = offs.size - 1
+    lv = np.zeros(n, dtype=np.int32)
+    e = C.c_uint64(0)
+    st = lib().orc_bfs_cgr_par(n, _ptr(b), _ptr(offs), min_interval_len, residual_segment_len, zeta_k, source,
+                               _ptr(lv), C.byref(e), threads)
+    if st != 0:
+        raise OracleError(st, "bfs_cgr_par")
+    return lv, int(e.value)
+
+
+def bc_par(rowoff, cols, sources, threads: int = 0) -> np.ndarray:
+    """Brandes BC parallel over sources, summed in source order (bit-identical to bc())."""
+    rowoff, cols = _csr(rowoff, cols)
+    n = rowoff.size - 1
+    src = np.ascontiguousarray(sources, dtype=np.uint32)
+    out = np.zeros(n, dtype=np.float64)
+    st = lib().orc_bc_par(n, _ptr(rowoff), _ptr(cols), _ptr(src) if src.size else None, src.size, _ptr(out), threads)
+    if st != 0:
+        raise OracleError(st, "bc_par")
+    return out
+
+
+def max_threads() -> int:
+    return int(lib().orc_max_threads())
 
 
 def cc(rowoff, cols) -> np.ndarray:

@@ -250,6 +250,30 @@ int orc_encode(uint64_t n, const uint64_t *rowoff, const uint32_t *cols, uint32_
     return ORC_OK;
 }
 
+/* The records of vertices [u0, u1) as a standalone bit stream (R2 concatenation), for the per-vertex-parallel
+ * encoder of gcgt_oracle_par.c ("per-vertex parallel with a prefix sum").  rel_offsets[i] = start
+ * of u0+i relative to the chunk (u1-u0 entries).  Rows are assumed validated (orc_encode_par validates first). */
+int orc_encode_range(const uint64_t *rowoff, const uint32_t *cols, uint32_t minLen, uint32_t segLen, uint32_t k,
+                     uint64_t u0, uint64_t u1, uint8_t **bytes_out, uint64_t *nbits_out, uint64_t *rel_offsets) {
+    uint64_t maxdeg = 0;
+    for (uint64_t u = u0; u < u1; u++) if (rowoff[u + 1] - rowoff[u] > maxdeg) maxdeg = rowoff[u + 1] - rowoff[u];
+    uint32_t *a = (uint32_t *)malloc(sizeof(uint32_t) * (maxdeg + 1));
+    uint32_t *b = (uint32_t *)malloc(sizeof(uint32_t) * (maxdeg + 1));
+    uint32_t *c = (uint32_t *)malloc(sizeof(uint32_t) * (maxdeg + 1));
+    bitbuf bb = {0};
+    int st = (a && b && c) ? ORC_OK : ORC_ENOMEM;
+    for (uint64_t u = u0; u < u1 && st == ORC_OK; u++) {
+        rel_offsets[u - u0] = bb.nbits;
+        st = encode_vertex(&bb, u, cols + rowoff[u], rowoff[u + 1] - rowoff[u], minLen, segLen, (int)k, 0, a, b, c);
+        if (bb.oom) st = ORC_ENOMEM;
+    }
+    free(a); free(b); free(c);
+    if (st != ORC_OK) { free(bb.buf); return st; }
+    *bytes_out = bb.buf;
+    *nbits_out = bb.nbits;
+    return ORC_OK;
+}
+
 /* Encodes one vertex record standalone (u, sorted list adj[0..deg-1]) for the hand-worked pins.  Returns the bit
  * length (>= 0) and writes the bits as a '0'/'1' string into out (cap chars), or a negative status.  This is the only
  * entry that accepts illustrative != 0 (Fig. 2's pre-App. C mode, gamma, unsegmented). */

@@ -64,6 +64,48 @@ def test_bfs_on_cgr_equals_bfs(ml, sl, k):
         assert edges == int(deg[ref >= 0].sum())
 
 
+@pytest.mark.parametrize("threads", [1, 2, 3, 8])
+def test_bfs_par_equals_bfs(threads):
+    """The OpenMP level-synchronous BFS (gcgt_oracle_par.c) gives the FIFO BFS's unique levels,
+    over the CSR and over the oracle's own CGR, with the edge count of the reached vertices."""
+    for seed, (n, m, sym) in enumerate([(1, 0, False), (64, 200, True), (3000, 30000, False), (20000, 250000, True)]):
+        if m:
+            ro, co = random_graph(n, m, seed=seed + 31 * threads, symmetric=sym)
+        else:
+            ro, co = np.zeros(n + 1, np.uint64), np.zeros(0, np.uint32)
+        deg = np.diff(ro.astype(np.int64))
+        for ml, sl, k in [(4, 32, 3), (0, 0, 1), (2, 8, 5)]:
+            b, nb, offs = O.encode(ro, co, ml, sl, k)
+            for s in sorted({0, n // 2, n - 1}):
+                ref = O.bfs(ro, co, s)
+                assert np.array_equal(O.bfs_par(ro, co, s, threads), ref), (seed, s)
+                lv, edges = O.bfs_cgr_par(b, offs, ml, sl, k, s, threads)
+                assert np.array_equal(lv, ref), (seed, ml, sl, k, s)
+                assert edges == int(deg[ref >= 0].sum())
+
+
+@pytest.mark.parametrize("name", ["c1", "web_s", "social_s", "rmat_s"])
+def test_bfs_par_on_recipes(name):
+    import synth
+    cfg = synth.CONFIGS[name]
+    ro, co = cfg.make()
+    b, nb, offs = O.encode(ro, co, cfg.min_interval_len, cfg.residual_segment_len, cfg.zeta_k)
+    for r in [0] + synth.pick_roots(ro, 2):
+        ref = O.bfs(ro, co, r)
+        assert np.array_equal(O.bfs_par(ro, co, r), ref)
+        lv, _ = O.bfs_cgr_par(b, offs, cfg.min_interval_len, cfg.residual_segment_len, cfg.zeta_k, r)
+        assert np.array_equal(lv, ref)
+
+
+@pytest.mark.parametrize("threads", [1, 3, 8])
+def test_bc_par_bit_identical(threads):
+    """orc_bc_par sums the per-source dependency vectors in source order: bit-identical to orc_bc."""
+    for seed, (n, m, sym) in enumerate([(12, 30, False), (700, 5000, True), (3000, 20000, False)]):
+        ro, co = random_graph(n, m, seed=seed + threads, symmetric=sym)
+        src = [0, 5, 5, n - 1, 3, 1, 7, 2, 9, 11][: 4 + seed * 3]
+        assert np.array_equal(O.bc_par(ro, co, src, threads), O.bc(ro, co, src))
+
+
 def brute_cc(n, adj):
     und = [set() for _ in range(n)]
     for u in range(n):

@@ -302,3 +302,22 @@ def test_input_validation():
     with pytest.raises(O.OracleError) as e:
         O.encode(ro, co, 4, 1, 1)
     assert e.value.code == -4
+
+
+@pytest.mark.parametrize("threads", [1, 4, 8])
+def test_encode_par_byte_identical(threads):
+    """The per-vertex-parallel oracle encoder (chunks concatenated at the prefix sum of their bit lengths, R2) is
+    byte-identical to the serial orc_encode, across chunk boundaries (n > 65536) and every parameter family."""
+    import synth
+    from graphs import random_graph
+    cases = [random_graph(1, 0, seed=1), random_graph(70_000, 400_000, seed=threads),
+             synth.CONFIGS["web_s"].make(), synth.CONFIGS["social_s"].make()]
+    for ro, co in cases:
+        for ml, sl, k in [(4, 32, 3), (0, 0, 1), (2, 8, 5), (4, 0, 2)]:
+            b, nb, offs = O.encode(ro, co, ml, sl, k)
+            pb, pnb, poffs = O.encode_par(ro, co, ml, sl, k, threads)
+            assert nb == pnb and np.array_equal(offs, poffs) and np.array_equal(b, pb), (ml, sl, k)
+    for ro, co, code in [([0, 2, 2], [1, 1], -2), ([0, 1, 1], [5], -3)]:  # duplicate id (R6), id >= n
+        with pytest.raises(O.OracleError) as e:
+            O.encode_par(np.array(ro, np.uint64), np.array(co, np.uint32), 4, 32, 3)
+        assert e.value.code == code
