@@ -5,11 +5,12 @@
 
 A step is one BFS query (the whole §8(a) path: frontier management, header / interval / residual-segment decode,
 filter, contraction) from a seeded root over the device-resident CGR of the configuration's synthetic graph.
-Default workload = BASELINE.json configs[1] (uk-2002-like web graph, 18.5M vertices) on 1 B200.
+Default workload = BASELINE.json configs[3] (uk-2007-like web graph, 105.9M vertices / 3.74B arcs), the config the
+metric is quoted on ("1/2/4/8 B200") and the largest single-GPU configuration.
 With N > 1 ranks (torchrun, NCCL) the graph is 1-D vertex-range partitioned: rank 0 builds and caches
 the CGR, every rank loads only its slice, and each BFS exchanges the next-frontier bitmap per level (all-to-all +
 all-gather over NVLink); "strong" scaling (the same graph and queries at every N); time = max over ranks.
-`--impl reference` times the oracle (oracle/, plain C, 1 thread) on the same workload (rank 0 only).
+`--impl reference` times the oracle (oracle/, plain C + OpenMP, all host cores) on the same workload (rank 0 only).
 Prints ONE JSON line on rank 0.
 """
 from __future__ import annotations
@@ -36,7 +37,7 @@ def parse():
     ap.add_argument("--gpus", type=int, default=1)
     ap.add_argument("--steps", type=int, default=16)
     ap.add_argument("--warmup", type=int, default=3)
-    ap.add_argument("--config", default="c2")
+    ap.add_argument("--config", default="c4")
     ap.add_argument("--impl", default="gcgt", choices=["gcgt", "reference"])
     ap.add_argument("--roots", type=int, default=16)
     ap.add_argument("--no-cpu-baseline", action="store_true")
@@ -181,20 +182,24 @@ def choose_roots(ro, count, seed=20190630):
 
 
 def run_reference(args, cfg, ws, rank):
-    """Oracle arm: oracle/ as it stands (plain C, one thread), BFS over the oracle's own CGR."""
+    """Oracle arm: oracle/ as it stands, BFS over the oracle's own CGR on all host cores (the OpenMP level-synchronous
+    variant); each step = one full BFS query from the next root.  Encoding (per-vertex parallel) is
+    preprocessing and untimed, as on the GPU arm."""
     if rank != 0:
         return
     import oracle as O
     ro, co, tgen = make_graph(cfg)
-    ob, onb, ooffs = O.encode(ro, co, cfg.min_interval_len, cfg.residual_segment_len, cfg.zeta_k)
+    P = (cfg.min_interval_len, cfg.residual_segment_len, cfg.zeta_k)
+    ob, onb, ooffs = O.encode_par(ro, co, *P)
     roots = choose_roots(ro, args.roots)
+    threads = O.max_threads()
     for i in range(args.warmup):
-        O.bfs_cgr(ob, ooffs, cfg.min_interval_len, cfg.residual_segment_len, cfg.zeta_k, roots[i % len(roots)])
+        O.bfs_cgr_par(ob, ooffs, *P, roots[i % len(roots)])
     tot_e, tot_t = 0.0, 0.0
     for i in range(args.steps):
         r = roots[(args.warmup + i) % len(roots)]
         t0 = time.perf_counter()
-        _, arcs = O.bfs_cgr(ob, ooffs, cfg.min_interval_len, cfg.residual_segment_len, cfg.zeta_k, r)
+        _, arcs = O.bfs_cgr_par(ob, ooffs, *P, r)
         tot_t += time.perf_counter() - t0
         tot_e += edges_of(cfg, arcs)
     v = tot_e / tot_t / 1e9
@@ -204,21 +209,46 @@ def run_reference(args, cfg, ws, rank):
             "config": {"workload": cfg.name + ": " + cfg.desc, "n": int(ro.size - 1), "m": int(ro[-1]),
                        "min_interval_len": cfg.min_interval_len, "residual_segment_len": cfg.residual_segment_len,
                        "zeta_k": cfg.zeta_k},
-            "cpu_baseline": {"value": v, "unit": "GTEPS", "cores": 1, "kind": "oracle",
-                             "sample": f"{args.steps} full BFS queries (oracle bfs_cgr over the oracle's CGR)"},
+            "cpu_baseline": {"value": v, "unit": "GTEPS", "cores": threads, "kind": "oracle",
+                             "cpu_model": cpu_model(),
+                             "sample": f"{args.steps} full BFS queries (oracle bfs_cgr_par: OpenMP level-synchronous "
+                                       f"BFS decoding the oracle's own CGR, {threads} threads)"},
             "e2e": {"value": v, "unit": "GTEPS", "h2d_bytes_per_step": 0, "d2h_bytes_per_step": 0}}
     print(json.dumps(line), flush=True)
 
 
-def cpu_baseline(cfg, ro, co, root):
-    """The oracle as it stands, 1 thread, one full BFS over its own CGR from the first bench root (~10 s on c2)."""
+def cpu_model():
+    try:
+        out = subprocess.run(["lscpu"], capture_output=True, text=True, timeout=10).stdout
+        for line in out.splitlines():
+            if line.startswith("Model name:"):
+                return line.split(":", 1)[1].strip()
+    except Exception:
+        pass
+    return None
+
+
+def cpu_baseline(cfg, ro, co, root, single_thread_arcs=4e8):
+    """The oracle as it stands on the host cores (SURVEY §8(c).2 / BASELINE.md CPU-baseline plan): one full BFS from
+    the first bench root with the OpenMP level-synchronous BFS over the oracle's own CGR on all cores, plus the
+    single-thread figure (the paper's "Naive" role) on a bounded sample of the same BFS (whole levels until
+    >= single_thread_arcs arcs are decoded)."""
     import oracle as O
-    ob, onb, ooffs = O.encode(ro, co, cfg.min_interval_len, cfg.residual_segment_len, cfg.zeta_k)
+    P = (cfg.min_interval_len, cfg.residual_segment_len, cfg.zeta_k)
+    ob, onb, ooffs = O.encode_par(ro, co, *P)
+    threads = O.max_threads()
     t0 = time.perf_counter()
-    _, arcs = O.bfs_cgr(ob, ooffs, cfg.min_interval_len, cfg.residual_segment_len, cfg.zeta_k, root)
+    _, arcs = O.bfs_cgr_par(ob, ooffs, *P, root)
     dt = time.perf_counter() - t0
-    return {"value": edges_of(cfg, arcs) / dt / 1e9, "unit": "GTEPS", "cores": 1, "kind": "oracle",
-            "sample": f"1 full BFS from root {root} over the oracle's own CGR of the same graph ({dt:.1f} s)"}
+    t1 = time.perf_counter()
+    arcs1 = O.bfs_cgr_sample(ob, ooffs, *P, root, int(single_thread_arcs), 1)
+    dt1 = time.perf_counter() - t1
+    return {"value": edges_of(cfg, arcs) / dt / 1e9, "unit": "GTEPS", "cores": threads, "kind": "oracle",
+            "cpu_model": cpu_model(), "os_cpu_count": os.cpu_count(),
+            "sample": f"1 full BFS from root {root} over the oracle's own CGR of the same graph, OpenMP level-"
+                      f"synchronous, {threads} threads ({dt:.1f} s)",
+            "single_thread": {"value": edges_of(cfg, arcs1) / dt1 / 1e9, "unit": "GTEPS", "cores": 1,
+                              "sample": f"the same BFS's first whole levels until {arcs1} arcs decoded ({dt1:.1f} s)"}}
 
 
 def main():
@@ -270,10 +300,10 @@ def main():
         g.bfs(roots[i % len(roots)], out=levels)
     torch.cuda.synchronize()
 
-    g.profile(True)
+    # ---- timed region: the production path (the BFS level loop as one CUDA graph per query, no profiling)
     evs = [(torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)) for _ in range(args.steps)]
     clocks = ClockSampler(local, dev)
-    tot = {"arcs": 0, "bits": 0, "vertices": 0, "levels": 0, "kms": 0.0, "klaunch": 0, "launches": 0, "edges": 0.0}
+    tot = {"launches": 0, "edges": 0.0, "levels": 0}
     step_edges = []
     if ws > 1:
         dist.barrier()
@@ -287,19 +317,12 @@ def main():
         evs[i][1].record(stream)
         tot["edges"] += edges_of_root[r]
         step_edges.append(edges_of_root[r])
-        st = g.last_stats
-        tot["launches"] += st["launches"]
-        tot["arcs"] += st["arcs_decoded"]
-        tot["bits"] += st["cgr_bits_decoded"]
-        tot["vertices"] += st["vertices_expanded"]
-        tot["levels"] += st["iterations"]
-        tot["kms"] += st["kernel_ms"]
-        tot["klaunch"] += st["kernel_launches"]
+        tot["launches"] += g.last_stats["launches"]
+        tot["levels"] += g.last_stats["iterations"]
     torch.cuda.synchronize()
     if ws > 1:
         dist.barrier()
     ck = clocks.stop()
-    g.profile(False)
     step_ms = [a.elapsed_time(b) for a, b in evs]
     t_ms = sum(step_ms)
     edges = tot["edges"]
@@ -314,15 +337,37 @@ def main():
         edges_all = edges
     value = edges_all / (t_ms * 1e-3) / 1e9
 
-    # roofline of the dominant kernel span (each level's expansion: top-down kernel + hub segments, or the bottom-up
-    # kernel): algorithmic bytes = CGR bytes decoded + 8 B bit offset + 4 B level write per vertex
-    # expanded (top-down) or examined (bottom-up)
+    # ---- roofline of the dominant kernel span, measured on the same roots right after the timed region: the profiled
+    # level loop brackets each level's expansion (top-down expand_kernel + hub_kernel, or bottom-up bu_kernel) with
+    # CUDA events on the graph's stream (inside a CUDA graph kernels cannot be bracketed by events, so the profiled
+    # pass runs the same kernels from the host-driven loop).  Algorithmic bytes = CGR bits decoded / 8
+    # + 12 B per vertex expanded (top-down) or examined (bottom-up): 4 B compact bit offset ... + 8 B, see DESIGN.
+    g.profile(True)
+    prof = {"arcs": 0, "bits": 0, "vertices": 0, "kms": 0.0, "klaunch": 0, "ms": 0.0}
+    pev = [(torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)) for _ in range(args.steps)]
+    for i in range(args.steps):
+        flush.fill_(i & 0xFF)
+        r = roots[(args.warmup + i) % len(roots)]
+        pev[i][0].record(stream)
+        g.bfs(r, out=levels)
+        pev[i][1].record(stream)
+        st = g.last_stats
+        prof["arcs"] += st["arcs_decoded"]
+        prof["bits"] += st["cgr_bits_decoded"]
+        prof["vertices"] += st["vertices_expanded"]
+        prof["kms"] += st["kernel_ms"]
+        prof["klaunch"] += st["kernel_launches"]
+    torch.cuda.synchronize()
+    g.profile(False)
+    prof["ms"] = sum(a.elapsed_time(b) for a, b in pev)
     peak, peak_src = hbm_peak()
-    alg_bytes = tot["bits"] / 8 + 12 * tot["vertices"]
-    k_s = tot["kms"] * 1e-3
+    alg_bytes = prof["bits"] / 8 + 12 * prof["vertices"]
+    k_s = prof["kms"] * 1e-3
     achieved = alg_bytes / k_s / 1e9 if k_s > 0 else 0.0
-    cgr_gbs = tot["bits"] / 8 / k_s / 1e9 if k_s > 0 else 0.0
+    cgr_gbs = prof["bits"] / 8 / k_s / 1e9 if k_s > 0 else 0.0
     traffic, traffic_src = ncu_traffic(args.config, tot["levels"] / args.steps)
+    tot.update({"arcs": prof["arcs"], "bits": prof["bits"], "vertices": prof["vertices"], "kms": prof["kms"],
+                "klaunch": prof["klaunch"]})
 
     e2e = None
     if not args.no_e2e:
@@ -349,9 +394,14 @@ def main():
                            "gen_s": round(tgen, 1), "encode_s": round(tenc, 1)},
                 "roofline": {"bound": "hbm", "achieved": achieved, "peak": peak, "unit": "GB/s",
                              "frac": achieved / peak, "traffic": traffic,
-                             "traffic_source": traffic_src, "alg_bytes_per_launch": alg_bytes / max(1, tot["klaunch"]), "kernel": "level expansion (expand_kernel+hub_kernel | bu_kernel)",
+                             "traffic_source": traffic_src, "alg_bytes_per_launch": alg_bytes / max(1, tot["klaunch"]),
+                             "kernel": "level expansion (expand_kernel+hub_kernel | bu_kernel)",
                              "peak_source": peak_src, "cgr_only_gbs": cgr_gbs, "cgr_only_frac": cgr_gbs / peak,
-                             "kernel_share_of_step": tot["kms"] / t_ms if t_ms else None,
+                             "kernel_ms_per_step": prof["kms"] / args.steps,
+                             "kernel_share_of_step": prof["kms"] / prof["ms"] if prof["ms"] else None,
+                             "profiled_ms_per_step": prof["ms"] / args.steps,
+                             "timing": "CUDA events around each level's expansion kernels on the graph's stream, "
+                                       "in a profiled pass over the same roots right after the timed region",
                              "launches": tot["klaunch"]},
                 "cpu_baseline": cpu, "e2e": e2e, "gpu_launches": int(tot["launches"]),
                 "clocks": ck}
@@ -454,14 +504,16 @@ def measure_e2e(G, cgr, incgr, roots, edges_of_root, cfg, n, nbits, dev, local, 
     L.gcgt_cgr_view(cgr.handle, C.byref(bp), None, C.byref(op), None, None)
     nbytes_words = ((nbits + 63) // 64 + 2) * 8
     reg = [(bp.value, nbytes_words), (op.value, (n + 1) * 8)]
-    h2d = nbytes_words + (n + 1) * 8
+    # H2D per load: the CGR words plus the compact bit offsets (u32 per vertex + a u64 anchor per 256 vertices)
+    offs_h2d = (n + 1) * 4 + ((n // 256) + 1) * 8
+    h2d = nbytes_words + offs_h2d
     if incgr is not None:
         ib, io = C.c_void_p(), C.c_void_p()
         inb = C.c_uint64()
         L.gcgt_cgr_view(incgr.handle, C.byref(ib), C.byref(inb), C.byref(io), None, None)
         inwords = ((inb.value + 63) // 64 + 2) * 8
         reg += [(ib.value, inwords), (io.value, (n + 1) * 8)]
-        h2d += inwords + (n + 1) * 8
+        h2d += inwords + offs_h2d
     codes = []
     for ptr, size in reg:
         codes.append(int(cudart.cudaHostRegister(ptr, size, 0)))
@@ -493,11 +545,28 @@ def measure_e2e(G, cgr, incgr, roots, edges_of_root, cfg, n, nbits, dev, local, 
         for (ptr, _), c in zip(reg, codes):
             if c == 0:
                 cudart.cudaHostUnregister(ptr)
+    # query-service variant: the graph stays resident (loaded once, like model weights); per step the source goes
+    # H2D and the whole levels array comes back D2H into pinned host memory
+    g = G.load(cgr, device=local, stream="torch", in_cgr=incgr, symmetric=cfg.symmetric)
+    g.bfs(roots[0], out=levels)
+    torch.cuda.synchronize()
+    qe, qt = 0.0, 0.0
+    for i in range(max(steps, 5)):
+        r = roots[i % len(roots)]
+        t0 = time.perf_counter()
+        g.bfs(r, out=levels)
+        qt += time.perf_counter() - t0
+        qe += edges_of_root[r]
+    g.unload()
     return {"value": tot_e / tot_t / 1e9, "unit": "GTEPS", "h2d_bytes_per_step": int(h2d),
             "d2h_bytes_per_step": int(4 * n), "host_register_status": codes, "per_step": split,
             "note": "per step (after 1 untimed warm-up cycle): gcgt_load (CGR + in-CGR + bit offsets H2D from pinned "
                     "host memory, pool allocation) + "
-                    "gcgt_bfs with a pinned host levels array + gcgt_unload; host wall clock"}
+                    "gcgt_bfs with a pinned host levels array + gcgt_unload; host wall clock",
+            "resident_graph": {"value": qe / qt / 1e9, "unit": "GTEPS", "h2d_bytes_per_step": 4,
+                               "d2h_bytes_per_step": int(4 * n),
+                               "note": "graph loaded once; per step gcgt_bfs(source) with a pinned host levels array "
+                                       "(source H2D, levels D2H inside the call); host wall clock"}}
 
 
 if __name__ == "__main__":

@@ -36,7 +36,7 @@ typedef enum {
     GCGT_ESEGLEN = -4,    /* a residual segment cannot hold even one residual (FORMAT.md R19)                */
     GCGT_ENOMEM = -5,     /* host or device allocation failed                                                 */
     GCGT_ECUDA = -6,      /* CUDA runtime error, or no usable device                                          */
-    GCGT_ENCCL = -7,      /* NCCL error (multi-GPU)                                                            */
+    GCGT_ERESERVED = -7,  /* (unused)                                                                          */
     GCGT_EFORMAT = -8     /* corrupt or inconsistent CGR (file or view)                                        */
 } gcgt_status;
 
@@ -81,6 +81,17 @@ gcgt_status gcgt_encode(const gcgt_csr* csr, const gcgt_params* params, gcgt_cgr
 /* Encodes the TRANSPOSE of csr (row v = sorted in-neighbours of v), for gcgt_load_opts.in_cgr.  Same errors. */
 gcgt_status gcgt_encode_transpose(const gcgt_csr* csr, const gcgt_params* params, gcgt_cgr** out);
 
+/* Vertex-range slices (graphs too large to hold as one CSR, e.g. C5 = R-MAT scale 29): gcgt_encode_slice encodes
+ * rows 0..rows->n-1 of a caller CSR as the records of vertices first .. first + rows->n - 1 of a graph with n_total
+ * vertices (column ids < n_total); the bytes equal bits [bit_offsets[first], bit_offsets[first + rows->n]) of the
+ * whole graph's CGR (records are self-contained, R2), bit offsets re-based to 0.  gcgt_cgr_concat appends
+ * consecutive slices into one CGR (EINVAL unless consecutive, same parameters and n_total).  gcgt_load of a slice
+ * loads exactly its vertex range as a partitioned graph (first and first + rows->n on 32-vertex words, or the end). */
+gcgt_status gcgt_encode_slice(const gcgt_csr* rows, uint64_t first, uint64_t n_total, const gcgt_params* params,
+                              gcgt_cgr** out);
+gcgt_status gcgt_cgr_concat(const gcgt_cgr* const* parts, uint32_t k, gcgt_cgr** out);
+gcgt_status gcgt_cgr_slice_info(const gcgt_cgr* cgr, uint64_t* first, uint64_t* n_total);
+
 /* Read-only view of a CGR: bytes (ceil(nbits/8), MSB-first, R1), nbits, bit_offsets (n + 1 entries, R2),
  * n, params.  Pointers stay valid until gcgt_cgr_free.  Any output pointer may be NULL. */
 gcgt_status gcgt_cgr_view(const gcgt_cgr* cgr, const uint8_t** bytes, uint64_t* nbits,
@@ -99,10 +110,10 @@ void gcgt_cgr_free(gcgt_cgr* cgr);
 /* ---- Device residency (§3.2 :469-479: "directly move the compressed adjacency lists to GPUs") -------------------- */
 typedef struct {
     int device;        /* CUDA device ordinal                                                                       */
-    void* stream;      /* cudaStream_t to run on; NULL = a library-created non-blocking stream                      */
+    void* stream;      /* cudaStream_t to run on (cudaStreamLegacy = (void*)1 for the legacy default stream); NULL = a
+                          library-created non-blocking stream                                                       */
     int rank, nranks;  /* 1-D vertex-range partition (multi-GPU).  nranks <= 1: single GPU (rank ignored)           */
-    void* nccl_comm;   /* ncclComm_t for nranks > 1 (created by the caller, e.g. from a unique id broadcast over
-                          torch.distributed); NULL for a single GPU                                                 */
+    void* reserved;    /* must be NULL (the collectives of the partitioned steps run in the caller)                  */
     const gcgt_cgr* in_cgr; /* CGR of the TRANSPOSE (in-arcs, e.g. from gcgt_encode_transpose) for the bottom-up
                                BFS step; NULL = none (top-down only unless `symmetric`).  Same n and params.      */
     int symmetric;     /* 1: every arc u->v has v->u, so the out-CGR doubles as the in-CGR (R-MAT configs)           */
@@ -149,7 +160,7 @@ gcgt_status gcgt_graph_range(const gcgt_graph* g, uint64_t* lo, uint64_t* hi);
 /* BFS from `source` over out-arcs (Fig. 7(b)).  levels[v] = hop distance, -1 if unreached; n entries.
  * With an in-CGR (or `symmetric`) and direction_optimizing, large levels run bottom-up: every unvisited vertex
  * decodes its in-record until the first frontier parent (intervals tested as frontier-bitmap ranges).
- * Errors: ERANGE (source >= n), ECUDA, ENCCL. */
+ * Errors: ERANGE (source >= n), ECUDA. */
 gcgt_status gcgt_bfs(gcgt_graph* g, uint32_t source, int32_t* levels, int out_placement, gcgt_stats* stats);
 
 /* Weakly connected components (Fig. 7(c): hooking + pointer jumping, Soman et al. [42]).  labels[v] = the
@@ -164,29 +175,47 @@ gcgt_status gcgt_bc(gcgt_graph* g, const uint32_t* sources, uint32_t k, double* 
 
 /* ---- Partitioned multi-GPU steps (§8 e; driver: paper_conf_sigmod_shalt19_b200/dist.py) -----------------------
  * A graph loaded with nranks > 1 holds only its owned vertex range [lo, hi) (gcgt_graph_range; boundaries on
- * 32-vertex words, balanced by CGR bits).  The caller runs the collectives between the steps (e.g. NCCL through
- * torch.distributed).  Every bitmap crossing this boundary is a DEVICE array of ceil(n/32) uint32 words (bit v%32
- * of word v/32); an owned slice is words [lo/32, ceil(hi/32)).  gcgt_bfs / gcgt_cc / gcgt_bc refuse partitioned
- * graphs.  BFS level d:
- *   gcgt_dist_bfs_expand  : decode the owned frontier's records, claim unvisited targets into `cand` (full bitmap,
- *                           zeroed by the call)                                           [expansion + filter]
- *   (caller) all-to-all   : slice q of every rank's cand goes to rank q
- *   gcgt_dist_bfs_commit  : recv = nparts owned-size slices; fslice = OR(recv) & ~visited; levels of the new owned
- *                           vertices = d + 1; *new_count = popcount(fslice) (host)       [contraction]
- *   (caller) all-gather   : the owned fslices form the global next frontier
- *   gcgt_dist_bfs_absorb  : frontier := gathered bitmap; visited |= frontier
- * and the search ends when the all-reduced new_count is 0.  gcgt_dist_bfs_levels copies the owned levels out.
+ * 32-vertex words, balanced by CGR bits): the out-records of the owned vertices and, with in_cgr / symmetric, their
+ * in-records.  The caller runs the collectives between the steps (e.g. NCCL through torch.distributed).  Every
+ * bitmap crossing this boundary is a DEVICE array of ceil(n/32) uint32 words (bit v%32 of word v/32); an owned slice
+ * is words [lo/32, ceil(hi/32)).  gcgt_bfs / gcgt_cc / gcgt_bc refuse partitioned graphs.
+ * The steps are ENQUEUED on the graph's stream and return without waiting (the caller's collectives must run on that
+ * stream or after gcgt_sync), except gcgt_dist_bfs_absorb and gcgt_dist_cc_hook, which return a count to the host:
+ * one host synchronisation per BFS level and per CC round.  BFS level d:
+ *   top-down (bottom_up = 0):
+ *     gcgt_dist_bfs_expand : decode the owned frontier's records, claim unvisited targets into `cand` (full bitmap,
+ *                            zeroed by the call)                                          [expansion + filter]
+ *     (caller) all-to-all  : slice q of every rank's cand goes to rank q
+ *     gcgt_dist_bfs_commit : fslice = OR(recv[0..nparts)) & ~visited; levels of the new owned vertices = d + 1
+ *   bottom-up (bottom_up = 1; needs the in-records):
+ *     gcgt_dist_bfs_expand : every owned unvisited vertex scans its in-record against the replicated frontier until
+ *                            the first parent; finds are written to the owned slice `fslice` (no exchange needed)
+ *     gcgt_dist_bfs_commit : with nparts = 0, keep = 1: fslice &= ~visited, levels = d + 1
+ *   both:
+ *     (caller) all-gather  : the owned fslices form the global next frontier
+ *     gcgt_dist_bfs_absorb : frontier := gathered bitmap; visited |= frontier; *count = its size (identical on every
+ *                            rank, so termination needs no extra collective)
+ * gcgt_dist_bfs_levels copies the owned levels out.
  * CC: parent is a caller-owned device array of n uint32 replicated on every rank; per round
- *   gcgt_dist_cc_hook (hook the owned vertices' arcs; *hooks = successful hooks), all-reduce(MIN) of parent,
- *   gcgt_dist_cc_jump (pointer jumping); stop when the all-reduced hook count is 0. */
+ *   gcgt_dist_cc_hook   hook the owned vertices' arcs (no path halving: hooks are the only writes to parent);
+ *                       *hooks = successful hooks (host; the call waits); the first min(hooks, cap) hooks are also
+ *                       written to `pairs` (device, 2 uint32 per hook: index hi, new parent lo < hi)
+ *   exchange            all-reduce(MIN) of parent — or, when every rank's hooks fit cap, the pair lists
+ *                       (all-gather) merged with gcgt_dist_cc_merge: parent[hi] = min(parent[hi], lo)
+ *   gcgt_dist_cc_jump   pointer jumping
+ *   and stop when no rank hooked.  Both exchanges leave identical parent arrays on every rank. */
 gcgt_status gcgt_dist_bfs_begin(gcgt_graph* g, uint32_t source);
-gcgt_status gcgt_dist_bfs_expand(gcgt_graph* g, uint32_t level, uint32_t* cand);
+gcgt_status gcgt_dist_bfs_expand(gcgt_graph* g, uint32_t level, uint32_t* cand, uint32_t* fslice, int bottom_up);
 gcgt_status gcgt_dist_bfs_commit(gcgt_graph* g, uint32_t level, const uint32_t* recv, uint32_t nparts,
-                                 uint32_t* fslice, uint64_t* new_count);
-gcgt_status gcgt_dist_bfs_absorb(gcgt_graph* g, const uint32_t* frontier);
+                                 uint32_t* fslice, int keep);
+gcgt_status gcgt_dist_bfs_absorb(gcgt_graph* g, const uint32_t* frontier, uint64_t* count);
 gcgt_status gcgt_dist_bfs_levels(gcgt_graph* g, int32_t* levels_owned, int out_placement);
-gcgt_status gcgt_dist_cc_hook(gcgt_graph* g, uint32_t* parent, uint64_t* hooks);
+gcgt_status gcgt_dist_cc_hook(gcgt_graph* g, uint32_t* parent, uint32_t* pairs, uint64_t cap, uint64_t* hooks);
+gcgt_status gcgt_dist_cc_merge(gcgt_graph* g, uint32_t* parent, const uint32_t* pairs, uint64_t npairs);
 gcgt_status gcgt_dist_cc_jump(gcgt_graph* g, uint32_t* parent);
+
+/* Waits for every step enqueued on the graph's stream (partitioned steps). */
+gcgt_status gcgt_sync(gcgt_graph* g);
 
 /* ---- Test hook (parity pin of the warp decoder against Fig. 5 / Ex. 5.1) ------------------
  * Runs the device warp-parallel decoder (Alg. 4 :901-919) on one warp over a caller bit array (host, MSB-first

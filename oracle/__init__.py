@@ -60,6 +60,7 @@ def lib():
         L.orc_bc.argtypes = [u64, p, p, p, u64, p]
         L.orc_bfs_cgr_par.argtypes = [u64, p, p, u32, u32, u32, u64, p, C.POINTER(u64), i32]
         L.orc_bfs_par.argtypes = [u64, p, p, u64, p, i32]
+        L.orc_bfs_cgr_sample.argtypes = [u64, p, p, u32, u32, u32, u64, p, C.POINTER(u64), i32, u64]
         L.orc_max_threads.restype = i32
         L.orc_encode_par.argtypes = [u64, p, p, u32, u32, u32, C.POINTER(p), C.POINTER(u64), p, i32]
         L.orc_bc_par.argtypes = [u64, p, p, p, u64, p, i32]
@@ -281,6 +282,21 @@ def bc_par(rowoff, cols, sources, threads: int = 0) -> np.ndarray:
     if st != 0:
         raise OracleError(st, "bc_par")
     return out
+
+
+def bfs_cgr_sample(bytes_, bit_offsets, min_interval_len, residual_segment_len, zeta_k, source: int,
+                   max_edges: int, threads: int = 0) -> int:
+    """Timing sample: the BFS's first whole levels until >= max_edges arcs are decoded; returns the arcs decoded."""
+    b = _padded(bytes_)
+    offs = np.ascontiguousarray(bit_offsets, dtype=np.uint64)
+    n = offs.size - 1
+    lv = np.zeros(n, dtype=np.int32)
+    e = C.c_uint64(0)
+    st = lib().orc_bfs_cgr_sample(n, _ptr(b), _ptr(offs), min_interval_len, residual_segment_len, zeta_k, source,
+                                  _ptr(lv), C.byref(e), threads, max_edges)
+    if st != 0:
+        raise OracleError(st, "bfs_cgr_sample")
+    return int(e.value)
 
 
 def max_threads() -> int:

@@ -47,7 +47,7 @@ static void seterr(int *err, int st) { __atomic_store_n(err, st, __ATOMIC_RELAXE
 /* Shared level loop.  csr != 0: rows from (rowoff, cols); else records decoded from the CGR. */
 static int bfs_levels(uint64_t n, const uint64_t *rowoff, const uint32_t *cols, const uint8_t *bytes,
                       const uint64_t *offs, uint32_t minLen, uint32_t segLen, uint32_t k, uint64_t source,
-                      int32_t *levels, uint64_t *edges_out, int nthreads) {
+                      int32_t *levels, uint64_t *edges_out, int nthreads, uint64_t max_edges) {
     if (source >= n) return PAR_ERANGE;
     if (nthreads > 0) omp_set_num_threads(nthreads);
     const int T = nthreads > 0 ? nthreads : omp_get_max_threads();
@@ -60,7 +60,7 @@ static int bfs_levels(uint64_t n, const uint64_t *rowoff, const uint32_t *cols, 
     int err = PAR_OK;
     front[0] = (uint32_t)source;
     levels[source] = 0;
-    for (int32_t d = 0; nf && !err; d++) {
+    for (int32_t d = 0; nf && !err && edges < max_edges; d++) {
 #pragma omp parallel num_threads(T) reduction(+ : edges)
         {
             const int t = omp_get_thread_num();
@@ -111,14 +111,24 @@ static int bfs_levels(uint64_t n, const uint64_t *rowoff, const uint32_t *cols, 
 /* BFS over the oracle's own CGR (decoded vertex by vertex), nthreads threads (0 = all cores). */
 int orc_bfs_cgr_par(uint64_t n, const uint8_t *bytes, const uint64_t *bit_offsets, uint32_t minLen, uint32_t segLen,
                     uint32_t k, uint64_t source, int32_t *levels, uint64_t *edges_out, int nthreads) {
-    return bfs_levels(n, NULL, NULL, bytes, bit_offsets, minLen, segLen, k, source, levels, edges_out, nthreads);
+    return bfs_levels(n, NULL, NULL, bytes, bit_offsets, minLen, segLen, k, source, levels, edges_out, nthreads,
+                      UINT64_MAX);
+}
+
+/* Bounded sample of the same BFS for timing: whole levels are expanded until at least max_edges arcs have been
+ * decoded (*edges_out = arcs decoded; the levels of later vertices are left incomplete). */
+int orc_bfs_cgr_sample(uint64_t n, const uint8_t *bytes, const uint64_t *bit_offsets, uint32_t minLen,
+                       uint32_t segLen, uint32_t k, uint64_t source, int32_t *levels, uint64_t *edges_out,
+                       int nthreads, uint64_t max_edges) {
+    return bfs_levels(n, NULL, NULL, bytes, bit_offsets, minLen, segLen, k, source, levels, edges_out, nthreads,
+                      max_edges);
 }
 
 /* The same level loop over a plain CSR (full-size parity of the largest configs, where decoding would only repeat
  * what the round-trip pins already establish). */
 int orc_bfs_par(uint64_t n, const uint64_t *rowoff, const uint32_t *cols, uint64_t source, int32_t *levels,
                 int nthreads) {
-    return bfs_levels(n, rowoff, cols, NULL, NULL, 0, 0, 0, source, levels, NULL, nthreads);
+    return bfs_levels(n, rowoff, cols, NULL, NULL, 0, 0, 0, source, levels, NULL, nthreads, UINT64_MAX);
 }
 
 int orc_max_threads(void) { return omp_get_max_threads(); }

@@ -15,16 +15,16 @@ import numpy as np
 _HERE = os.path.dirname(os.path.abspath(__file__))
 LIB_PATH = os.environ.get("GCGT_LIB") or os.path.join(_HERE, "libgcgt.so")  # GCGT_LIB: A/B builds (tools/)
 
-OK, EINVAL, EUNSORTED, ERANGE, ESEGLEN, ENOMEM, ECUDA, ENCCL, EFORMAT = 0, -1, -2, -3, -4, -5, -6, -7, -8
+OK, EINVAL, EUNSORTED, ERANGE, ESEGLEN, ENOMEM, ECUDA, EFORMAT = 0, -1, -2, -3, -4, -5, -6, -8
 STATUS_NAMES = {0: "OK", -1: "EINVAL", -2: "EUNSORTED", -3: "ERANGE", -4: "ESEGLEN", -5: "ENOMEM", -6: "ECUDA",
-                -7: "ENCCL", -8: "EFORMAT"}
+                -8: "EFORMAT"}
 OUT_HOST, OUT_DEVICE = 0, 1
 
 # public symbols of include/gcgt.h (tests check the library exports every one)
-ABI_SYMBOLS = ["gcgt_encode", "gcgt_encode_transpose", "gcgt_cgr_view", "gcgt_cgr_from_arrays", "gcgt_cgr_save", "gcgt_cgr_open",
+ABI_SYMBOLS = ["gcgt_encode", "gcgt_encode_transpose", "gcgt_encode_slice", "gcgt_cgr_concat", "gcgt_cgr_slice_info", "gcgt_cgr_view", "gcgt_cgr_from_arrays", "gcgt_cgr_save", "gcgt_cgr_open",
                "gcgt_cgr_free", "gcgt_load", "gcgt_load_csr", "gcgt_unload", "gcgt_profile", "gcgt_profile_spans", "gcgt_graph_range", "gcgt_bfs", "gcgt_cc", "gcgt_bc",
                "gcgt_dist_bfs_begin", "gcgt_dist_bfs_expand", "gcgt_dist_bfs_commit", "gcgt_dist_bfs_absorb",
-               "gcgt_dist_bfs_levels", "gcgt_dist_cc_hook", "gcgt_dist_cc_jump",
+               "gcgt_dist_bfs_levels", "gcgt_dist_cc_hook", "gcgt_dist_cc_merge", "gcgt_dist_cc_jump", "gcgt_sync",
                "gcgt_debug_warp_decode", "gcgt_last_error", "gcgt_version"]
 
 
@@ -53,7 +53,7 @@ class Stats(C.Structure):
 
 class LoadOpts(C.Structure):
     _fields_ = [("device", C.c_int), ("stream", C.c_void_p), ("rank", C.c_int), ("nranks", C.c_int),
-                ("nccl_comm", C.c_void_p), ("in_cgr", C.c_void_p), ("symmetric", C.c_int),
+                ("reserved", C.c_void_p), ("in_cgr", C.c_void_p), ("symmetric", C.c_int),
                 ("direction_optimizing", C.c_int), ("host_resident", C.c_int)]
 
 
@@ -70,6 +70,9 @@ def lib():
         p, u32, u64, i32 = C.c_void_p, C.c_uint32, C.c_uint64, C.c_int
         L.gcgt_encode.argtypes = [C.POINTER(Csr), C.POINTER(Params), C.POINTER(p)]
         L.gcgt_encode_transpose.argtypes = [C.POINTER(Csr), C.POINTER(Params), C.POINTER(p)]
+        L.gcgt_encode_slice.argtypes = [C.POINTER(Csr), u64, u64, C.POINTER(Params), C.POINTER(p)]
+        L.gcgt_cgr_concat.argtypes = [C.POINTER(p), u32, C.POINTER(p)]
+        L.gcgt_cgr_slice_info.argtypes = [p, C.POINTER(u64), C.POINTER(u64)]
         L.gcgt_cgr_view.argtypes = [p, C.POINTER(p), C.POINTER(u64), C.POINTER(p), C.POINTER(u64), C.POINTER(Params)]
         L.gcgt_cgr_from_arrays.argtypes = [u64, p, u64, p, C.POINTER(Params), C.POINTER(p)]
         L.gcgt_cgr_save.argtypes = [p, C.c_char_p]
@@ -87,12 +90,14 @@ def lib():
         L.gcgt_cc.argtypes = [p, p, i32, C.POINTER(Stats)]
         L.gcgt_bc.argtypes = [p, p, u32, p, i32, C.POINTER(Stats)]
         L.gcgt_dist_bfs_begin.argtypes = [p, u32]
-        L.gcgt_dist_bfs_expand.argtypes = [p, u32, p]
-        L.gcgt_dist_bfs_commit.argtypes = [p, u32, p, u32, p, C.POINTER(u64)]
-        L.gcgt_dist_bfs_absorb.argtypes = [p, p]
+        L.gcgt_dist_bfs_expand.argtypes = [p, u32, p, p, i32]
+        L.gcgt_dist_bfs_commit.argtypes = [p, u32, p, u32, p, i32]
+        L.gcgt_dist_bfs_absorb.argtypes = [p, p, C.POINTER(u64)]
         L.gcgt_dist_bfs_levels.argtypes = [p, p, i32]
-        L.gcgt_dist_cc_hook.argtypes = [p, p, C.POINTER(u64)]
+        L.gcgt_dist_cc_hook.argtypes = [p, p, p, u64, C.POINTER(u64)]
+        L.gcgt_dist_cc_merge.argtypes = [p, p, p, u64]
         L.gcgt_dist_cc_jump.argtypes = [p, p]
+        L.gcgt_sync.argtypes = [p]
         L.gcgt_debug_warp_decode.argtypes = [p, u64, u32, u32, u64, p, p, p, C.POINTER(u32)]
         L.gcgt_last_error.restype = C.c_char_p
         L.gcgt_version.restype = C.c_char_p
@@ -174,6 +179,35 @@ def encode_transpose(row_offsets: np.ndarray, cols: np.ndarray, min_interval_len
     return CGR(h)
 
 
+def encode_slice(row_offsets: np.ndarray, cols: np.ndarray, first: int, n_total: int, min_interval_len: int = 4,
+                 residual_segment_len: int = 32, zeta_k: int = 3) -> CGR:
+    """Records of vertices first .. first + len(row_offsets) - 2 (rows of a slice CSR, global column ids)."""
+    ro = np.ascontiguousarray(row_offsets, dtype=np.uint64)
+    co = np.ascontiguousarray(cols, dtype=np.uint32)
+    if co.size == 0:
+        co = np.zeros(1, dtype=np.uint32)
+    csr = Csr(ro.size - 1, ro.ctypes.data, co.ctypes.data)
+    P = Params(min_interval_len, residual_segment_len, zeta_k)
+    h = C.c_void_p()
+    _check(lib().gcgt_encode_slice(C.byref(csr), first, n_total, C.byref(P), C.byref(h)), "gcgt_encode_slice")
+    return CGR(h)
+
+
+def concat(parts) -> CGR:
+    """One CGR from consecutive slices (gcgt_cgr_concat)."""
+    arr = (C.c_void_p * len(parts))(*[p.handle for p in parts])
+    h = C.c_void_p()
+    _check(lib().gcgt_cgr_concat(arr, len(parts), C.byref(h)), "gcgt_cgr_concat")
+    return CGR(h)
+
+
+def slice_info(cgr: CGR):
+    """(first vertex, n_total) of a CGR (0, n for a whole graph)."""
+    b, t = C.c_uint64(), C.c_uint64()
+    _check(lib().gcgt_cgr_slice_info(cgr.handle, C.byref(b), C.byref(t)), "gcgt_cgr_slice_info")
+    return int(b.value), int(t.value)
+
+
 def from_arrays(bytes_: np.ndarray, nbits: int, bit_offsets: np.ndarray, min_interval_len: int,
                 residual_segment_len: int, zeta_k: int) -> CGR:
     b = np.ascontiguousarray(bytes_, dtype=np.uint8)
@@ -191,6 +225,17 @@ def open_cgr(path: str) -> CGR:
     h = C.c_void_p()
     _check(lib().gcgt_cgr_open(path.encode(), C.byref(h)), "gcgt_cgr_open")
     return CGR(h)
+
+
+CUDA_STREAM_LEGACY = 1  # cudaStreamLegacy: the legacy default stream, torch's default stream
+
+
+def _torch_stream(device):
+    """Torch's current stream on `device` as a cudaStream_t value: the legacy default stream is handle 0 in torch, which
+    the C ABI reads as "no stream" (a library-created one), so it is passed as cudaStreamLegacy."""
+    import torch
+    s = torch.cuda.current_stream(device).cuda_stream
+    return s if s else CUDA_STREAM_LEGACY
 
 
 def _out(out, n, np_dtype, torch_dtype_name):
@@ -212,20 +257,21 @@ def _out(out, n, np_dtype, torch_dtype_name):
 class Graph:
     """Device-resident CGR (gcgt_load)."""
 
-    def __init__(self, cgr: CGR, device: int = 0, stream=None, rank: int = 0, nranks: int = 1, nccl_comm=None,
+    def __init__(self, cgr: CGR, device: int = 0, stream=None, rank: int = 0, nranks: int = 1,
                  in_cgr: "CGR | None" = None, symmetric: bool = False, direction_optimizing: bool = True,
                  host_resident: bool = False):
+        self.stream_kind = stream if isinstance(stream, str) else ("caller" if stream else "own")
         if stream == "torch":
-            import torch
-            stream = torch.cuda.current_stream(device).cuda_stream
-        opts = LoadOpts(device, C.c_void_p(stream) if stream else None, rank, nranks,
-                        C.c_void_p(nccl_comm) if nccl_comm else None, in_cgr.handle if in_cgr is not None else None,
+            stream = _torch_stream(device)
+        opts = LoadOpts(device, C.c_void_p(stream) if stream else None, rank, nranks, None,
+                        in_cgr.handle if in_cgr is not None else None,
                         1 if symmetric else 0, 1 if direction_optimizing else 0, 1 if host_resident else 0)
         self._in_cgr = in_cgr
+        self.has_in = in_cgr is not None or bool(symmetric)
         h = C.c_void_p()
         _check(lib().gcgt_load(cgr.handle, C.byref(opts), C.byref(h)), "gcgt_load")
         self._h = h
-        self.n = cgr_n(cgr)
+        self.n = slice_info(cgr)[1]
         self.last_stats: dict = {}
 
     def profile(self, enable: bool = True, spans: bool = False):
@@ -267,31 +313,40 @@ class Graph:
         self.last_stats = st.as_dict()
         return res
 
-    # ---- partitioned steps (dist.py); device pointers as ints -------------------------------------------------
+    # ---- partitioned steps (dist.py); device pointers as ints; enqueued on the graph's stream ----------------------
     def dist_bfs_begin(self, source: int):
         _check(lib().gcgt_dist_bfs_begin(self._h, source), "gcgt_dist_bfs_begin")
 
-    def dist_bfs_expand(self, level: int, cand_ptr: int):
-        _check(lib().gcgt_dist_bfs_expand(self._h, level, C.c_void_p(cand_ptr)), "gcgt_dist_bfs_expand")
+    def dist_bfs_expand(self, level: int, cand_ptr: int, fslice_ptr: int = 0, bottom_up: bool = False):
+        _check(lib().gcgt_dist_bfs_expand(self._h, level, C.c_void_p(cand_ptr), C.c_void_p(fslice_ptr) if fslice_ptr
+                                          else None, 1 if bottom_up else 0), "gcgt_dist_bfs_expand")
 
-    def dist_bfs_commit(self, level: int, recv_ptr: int, nparts: int, fslice_ptr: int) -> int:
+    def dist_bfs_commit(self, level: int, recv_ptr: int, nparts: int, fslice_ptr: int, keep: bool = False):
+        _check(lib().gcgt_dist_bfs_commit(self._h, level, C.c_void_p(recv_ptr) if recv_ptr else None, nparts,
+                                          C.c_void_p(fslice_ptr), 1 if keep else 0), "gcgt_dist_bfs_commit")
+
+    def dist_bfs_absorb(self, frontier_ptr: int) -> int:
         cnt = C.c_uint64(0)
-        _check(lib().gcgt_dist_bfs_commit(self._h, level, C.c_void_p(recv_ptr), nparts, C.c_void_p(fslice_ptr),
-                                          C.byref(cnt)), "gcgt_dist_bfs_commit")
+        _check(lib().gcgt_dist_bfs_absorb(self._h, C.c_void_p(frontier_ptr), C.byref(cnt)), "gcgt_dist_bfs_absorb")
         return int(cnt.value)
 
-    def dist_bfs_absorb(self, frontier_ptr: int):
-        _check(lib().gcgt_dist_bfs_absorb(self._h, C.c_void_p(frontier_ptr)), "gcgt_dist_bfs_absorb")
+    def sync(self):
+        _check(lib().gcgt_sync(self._h), "gcgt_sync")
 
     def dist_bfs_levels(self, out):
         ptr, where, res = _out(out, self.range()[1] - self.range()[0], np.int32, "int32")
         _check(lib().gcgt_dist_bfs_levels(self._h, ptr, where), "gcgt_dist_bfs_levels")
         return res
 
-    def dist_cc_hook(self, parent_ptr: int) -> int:
+    def dist_cc_hook(self, parent_ptr: int, pairs_ptr: int = 0, cap: int = 0) -> int:
         h = C.c_uint64(0)
-        _check(lib().gcgt_dist_cc_hook(self._h, C.c_void_p(parent_ptr), C.byref(h)), "gcgt_dist_cc_hook")
+        _check(lib().gcgt_dist_cc_hook(self._h, C.c_void_p(parent_ptr), C.c_void_p(pairs_ptr) if pairs_ptr else None,
+                                       cap, C.byref(h)), "gcgt_dist_cc_hook")
         return int(h.value)
+
+    def dist_cc_merge(self, parent_ptr: int, pairs_ptr: int, npairs: int):
+        _check(lib().gcgt_dist_cc_merge(self._h, C.c_void_p(parent_ptr), C.c_void_p(pairs_ptr), npairs),
+               "gcgt_dist_cc_merge")
 
     def dist_cc_jump(self, parent_ptr: int):
         _check(lib().gcgt_dist_cc_jump(self._h, C.c_void_p(parent_ptr)), "gcgt_dist_cc_jump")
@@ -327,15 +382,16 @@ def load_csr(row_offsets: np.ndarray, cols: np.ndarray, device: int = 0, stream=
     if co.size == 0:
         co = np.zeros(1, dtype=np.uint32)
     if stream == "torch":
-        import torch
-        stream = torch.cuda.current_stream(device).cuda_stream
+        stream = _torch_stream(device)
     csr = Csr(ro.size - 1, ro.ctypes.data, co.ctypes.data)
     opts = LoadOpts(device, C.c_void_p(stream) if stream else None, 0, 1, None, None, 1 if symmetric else 0,
-                    1 if direction_optimizing else 0)
+                    1 if direction_optimizing else 0, 0)
     h = C.c_void_p()
     _check(lib().gcgt_load_csr(C.byref(csr), C.byref(opts), C.byref(h)), "gcgt_load_csr")
     g = Graph.__new__(Graph)
     g._in_cgr = None
+    g.has_in = bool(direction_optimizing)
+    g.stream_kind = "torch" if stream else "own"
     g._h = h
     g.n = int(ro.size - 1)
     g.last_stats = {}

@@ -18,7 +18,8 @@ NCCL_INC = "/usr/include"
 
 SOURCES_CU = ["gcgt.cu"]
 SOURCES_CPP = ["encode.cpp"]
-HEADERS = ["internal.h", "decode.cuh", "csr_bfs.cuh"]
+HEADERS = ["internal.h", "decode.cuh", "device.cuh", "apps.cuh", "expand.cuh", "bottomup.cuh", "contract.cuh",
+           "csr_bfs.cuh"]
 
 
 def _newer(target, deps):
@@ -41,7 +42,7 @@ def build(force: bool = False, verbose_ptxas: bool = False) -> str:
         s = os.path.join(CSRC, src)
         o = os.path.join(BUILD, src + ".o")
         if force or _newer(o, [s] + hdrs):
-            cmd = [NVCC, *ARCH, "-O3", "-lineinfo", "-std=c++17", "-Xcompiler", "-fPIC", "-c", s, "-o", o]
+            cmd = [NVCC, *ARCH, "-O3", "-lineinfo", "-std=c++17", "-Xcompiler", "-fPIC,-fopenmp", "-c", s, "-o", o]
             if verbose_ptxas:
                 cmd += ["-Xptxas", "-v"]
             _run(cmd)

@@ -1,10 +1,16 @@
-// csr_bfs.cuh — uncompressed-CSR BFS on the same B200 (§8 f3; included by gcgt.cu inside its anonymous namespace).
+#pragma once
+#include "apps.cuh"
+#include "expand.cuh"
+
+namespace gcgt_dev {
+
+// csr_bfs.cuh — uncompressed-CSR BFS on the same B200 (§8 f3).
 //
 // The paper compares GCGT with an uncompressed GPU BFS ("GPUCSR", Merrill et al.) and reports the
 // decoding overhead (+54 % at 18.1x compression, Fig. 8 :1571-1578).  This is that baseline on B200, built from the
 // same parts as the CGR path so that the ratio isolates decoding: the same frontier (bitmap F + queue of frontier
 // words), the same filter (BfsApp: read-only visited pre-test, fire-and-forget atomicOr on N), the same contraction
-// (commit_dense) and direction choice (bfs_decide).  Only the expansion differs: neighbour ids are read from col[]:
+// (commit_kernel) and direction choice (decide_body).  Only the expansion differs: neighbour ids are read from col[]:
 //  * top-down: a warp takes batches of frontier words, lists their vertices, and flattens the arcs of 32 vertices at
 //    a time over its lanes (coalesced col[] reads, four ids in flight per lane); vertices with more than
 //    kCsrHub arcs go to a per-level hub queue whose kCsrChunk-arc chunks are spread over the whole grid;
@@ -30,7 +36,7 @@ __global__ void __launch_bounds__(kBlock, 4) csr_expand_kernel(const uint64_t* _
                                                                const uint32_t* __restrict__ col, Front fr, BfsApp app,
                                                                unsigned long long* cursor, CsrHubEntry* hubq,
                                                                unsigned long long* hub_ctr, const uint32_t* dir,
-                                                               Stats* st) {
+                                                               unsigned long long* st) {
     __shared__ CsrSmem smem[kWarps];
     const uint32_t wid = threadIdx.x >> 5, lane = lane_id();
     CsrSmem& sm = smem[wid];
@@ -111,7 +117,7 @@ __global__ void __launch_bounds__(kBlock, 4) csr_expand_kernel(const uint64_t* _
             __syncwarp();
         }
     }
-    add_stats(st, nv, na, na * 32);
+    add_stats3(st, nv, na, na * 32);
     if (lane == 0) {  // the last warp out resets the work cursor for the next launch
         const unsigned long long nwarp = (unsigned long long)gridDim.x * kWarps;
         if (atomicAdd(cursor + 1, 1ull) == nwarp - 1) {
@@ -123,7 +129,7 @@ __global__ void __launch_bounds__(kBlock, 4) csr_expand_kernel(const uint64_t* _
 
 // Hub arcs of the level: warp per kCsrChunk-arc chunk (grid-stride), lanes stride the chunk (coalesced).
 __global__ void __launch_bounds__(kBlock) csr_hub_kernel(const uint32_t* __restrict__ col, const CsrHubEntry* hubq,
-                                                         const unsigned long long* hub_ctr, BfsApp app, Stats* st) {
+                                                         const unsigned long long* hub_ctr, BfsApp app, unsigned long long* st) {
     const uint32_t lane = lane_id();
     const unsigned long long hc = *(volatile const unsigned long long*)hub_ctr;
     const uint32_t nh = (uint32_t)(hc >> 32), S = (uint32_t)(hc & 0xffffffffu);
@@ -154,7 +160,7 @@ __global__ void __launch_bounds__(kBlock) csr_hub_kernel(const uint32_t* __restr
             app.many(v, nb);
         }
     }
-    add_stats(st, 0, na, na * 32);
+    add_stats3(st, 0, na, na * 32);
 }
 
 // Bottom-up level over the in-lists: warp per word, lane per unvisited vertex, stop at the first frontier parent.
@@ -162,7 +168,7 @@ __global__ void __launch_bounds__(kBlock) csr_bu_kernel(const uint64_t* __restri
                                                         const uint32_t* __restrict__ col,
                                                         const uint32_t* __restrict__ V,
                                                         const uint32_t* __restrict__ F, uint32_t* __restrict__ N,
-                                                        uint64_t n, const uint32_t* __restrict__ dir, Stats* st) {
+                                                        uint64_t n, const uint32_t* __restrict__ dir, unsigned long long* st) {
     if (*dir != 1) return;
     const uint32_t lane = lane_id();
     const uint64_t nwv = (n + 31) >> 5;
@@ -192,5 +198,7 @@ __global__ void __launch_bounds__(kBlock) csr_bu_kernel(const uint64_t* __restri
         const uint32_t fb = __ballot_sync(0xffffffffu, found);
         if (lane == 0 && fb) N[w] = fb;
     }
-    add_stats(st, nv, na, na * 32);
+    add_stats3(st, nv, na, na * 32);
 }
+
+}  // namespace gcgt_dev

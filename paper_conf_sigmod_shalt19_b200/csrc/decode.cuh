@@ -1,4 +1,5 @@
-// decode.cuh — device-side CGR decoding for sm_100a (FORMAT.md R1-R19).
+// decode.cuh — device-side CGR codeword decoding for sm_100a (FORMAT.md R1-R19): the 64-bit window decoder and the
+// warp-parallel decoder of Alg. 4 (test hook; the production path reads records through BitReader, device.cuh).
 //
 // The device keeps the CGR as 64-bit words in stream order (bit i of the stream is bit 63-(i%64) of word i/64;
 // the load step byte-swaps the canonical MSB-first bytes once).  A codeword at bit p is decoded from a 64-bit
@@ -85,51 +86,6 @@ __device__ __forceinline__ uint64_t decode(const uint64_t* __restrict__ W, uint6
 __device__ __forceinline__ int64_t unmap_first(uint64_t u, uint64_t c) {
     const uint64_t z = c - 1;
     return (int64_t)u + ((z & 1) ? -(int64_t)(z >> 1) : (int64_t)(z >> 1));
-}
-
-// Walks u's record: calls vis.range(start, len) per interval and vis.one(v) per residual.
-// Unsegmented (SEG=false): R8-R12.  Segmented (SEG=true): R14-R17.  Returns the neighbour count.
-template <int K, bool SEG, class Visitor>
-__device__ __forceinline__ uint32_t walk_record(const uint64_t* __restrict__ W, uint64_t p, uint64_t u,
-                                                uint32_t min_len, uint32_t seg_bits, Visitor& vis) {
-    uint64_t deg = 0;
-    if (!SEG) deg = decode<K>(W, p) - 1;
-    const uint64_t itv = decode<K>(W, p) - 1;
-    uint64_t got = 0;
-    int64_t prev_end = 0;
-    for (uint64_t t = 0; t < itv; t++) {
-        const uint64_t g = decode<K>(W, p);
-        const uint64_t len = decode<K>(W, p) - 1 + min_len;
-        const int64_t start = t == 0 ? unmap_first(u, g) : prev_end + (int64_t)g;
-        vis.range((uint32_t)start, (uint32_t)len);
-        prev_end = start + (int64_t)len - 1;
-        got += len;
-    }
-    if (!SEG) {
-        const uint64_t nres = deg - got;
-        int64_t cur = 0;
-        for (uint64_t t = 0; t < nres; t++) {
-            const uint64_t c = decode<K>(W, p);
-            cur = t == 0 ? unmap_first(u, c) : cur + (int64_t)c;
-            vis.one((uint32_t)cur);
-        }
-        return (uint32_t)deg;
-    } else {
-        const uint64_t nseg = decode<K>(W, p) - 1;
-        const uint64_t base = p;
-        for (uint64_t s = 0; s < nseg; s++) {
-            uint64_t q = base + s * seg_bits;
-            const uint64_t cnt = decode<K>(W, q) - 1;
-            int64_t cur = unmap_first(u, decode<K>(W, q));
-            vis.one((uint32_t)cur);
-            for (uint64_t t = 1; t < cnt; t++) {
-                cur += (int64_t)decode<K>(W, q);
-                vis.one((uint32_t)cur);
-            }
-            got += cnt;
-        }
-        return (uint32_t)got;
-    }
 }
 
 }  // namespace gcgt_dev
@@ -225,134 +181,5 @@ __device__ __forceinline__ uint64_t warp_decode(const uint64_t* __restrict__ W, 
     }
     return p;
 }
-
-}  // namespace gcgt_dev
-
-namespace gcgt_dev {
-
-// Register-staged bit reader: a 256-bit window (four 64-bit stream words) held in registers and refilled with
-// four independent loads when a codeword may cross its end.  Decoding is then pure ALU work (CLZ + shifts):
-// one memory round trip per ~256 bits instead of one (L1) round trip per codeword.  Codewords longer than the
-// 64-bit path use the global-memory slow path.
-struct RegStream {
-    const uint64_t* __restrict__ W;
-    uint64_t p;      // absolute bit position of the next codeword
-    uint64_t base;   // word index of r0
-    uint64_t r0, r1, r2, r3;
-
-    __device__ __forceinline__ void fill(uint64_t wi) {
-        base = wi;
-        r0 = ldg64(W + wi);
-        r1 = ldg64(W + wi + 1);
-        r2 = ldg64(W + wi + 2);
-        r3 = ldg64(W + wi + 3);
-    }
-    __device__ __forceinline__ void init(const uint64_t* __restrict__ w, uint64_t pos) {
-        W = w;
-        p = pos;
-        fill(pos >> 6);
-    }
-    __device__ __forceinline__ void seek(uint64_t pos) {
-        p = pos;
-        const uint64_t wi = pos >> 6;
-        if (wi < base || wi + 1 > base + 3) fill(wi);
-    }
-    __device__ __forceinline__ uint64_t win() {
-        uint64_t wi = p >> 6;
-        if (wi + 1 > base + 3) {  // the 64-bit window would leave the staged words
-            fill(wi);
-        }
-        const uint32_t k = (uint32_t)(wi - base), s = (uint32_t)(p & 63);
-        const uint64_t a = k == 0 ? r0 : k == 1 ? r1 : r2;
-        const uint64_t b = k == 0 ? r1 : k == 1 ? r2 : r3;
-        return s ? (a << s) | (b >> (64 - s)) : a;
-    }
-    template <int K>
-    __device__ __forceinline__ uint64_t next() {
-        const uint64_t w = win();
-        const uint32_t z = (uint32_t)__clzll((long long)w);
-        if (K == 1) {
-            if (z < 32) {
-                const uint32_t L = 2 * z + 1;
-                p += L;
-                return w >> (64 - L);
-            }
-        } else {
-            const uint32_t h = z + 1, L = h * (K + 1);
-            if (L <= 64) {
-                p += L;
-                return (w << h) >> (64 - K * h);
-            }
-        }
-        const uint64_t v = decode_slow<K>(W, p);
-        return v;
-    }
-};
-
-}  // namespace gcgt_dev
-
-namespace gcgt_dev {
-
-// Sequential bit-buffer reader: the next stream bits left-aligned in a 64-bit register, refilled 32 bits at a
-// time (32-bit stream word j is ((const uint32_t*)W)[j ^ 1] because W holds 64-bit words in stream order on a
-// little-endian machine).  Per codeword: CLZ, two shifts, a length check and an occasional 32-bit load, all in
-// 32-bit-friendly arithmetic.  Codewords longer than the buffered bits take the global slow path.
-struct BitBuf {
-    uint64_t buf;    // next bits, MSB first
-    uint32_t avail;  // valid bits in buf
-    uint64_t nxt;    // next 32-bit stream word to load
-
-    __device__ __forceinline__ static uint32_t ld32(const uint64_t* __restrict__ W, uint64_t j) {
-        return __ldg(reinterpret_cast<const unsigned int*>(W) + (j ^ 1));
-    }
-    __device__ __forceinline__ void init(const uint64_t* __restrict__ W, uint64_t p) {
-        const uint64_t j = p >> 5;
-        const uint32_t off = (uint32_t)(p & 31);
-        buf = (((uint64_t)ld32(W, j) << 32) | ld32(W, j + 1)) << off;
-        avail = 64 - off;
-        nxt = j + 2;
-    }
-    __device__ __forceinline__ uint64_t pos() const { return nxt * 32 - avail; }
-    template <int K>
-    __device__ __forceinline__ uint64_t next(const uint64_t* __restrict__ W) {
-        if (avail <= 32) {
-            buf |= (uint64_t)ld32(W, nxt) << (32 - avail);
-            avail += 32;
-            nxt++;
-        }
-        // fast path (32-bit arithmetic): after the refill avail > 32, so a codeword of <= 32 bits is complete
-        const uint32_t hi = (uint32_t)(buf >> 32);
-        const uint32_t z32 = __clz(hi);
-        if (K == 1) {
-            if (z32 < 16) {
-                const uint32_t L = 2 * z32 + 1;
-                buf <<= L;
-                avail -= L;
-                return hi >> (32 - L);
-            }
-        } else {
-            const uint32_t h = z32 + 1, L = h * (K + 1);
-            if (L <= 32) {
-                buf <<= L;
-                avail -= L;
-                return (hi << h) >> (32 - K * h);
-            }
-        }
-        const uint32_t z = (uint32_t)__clzll((long long)buf);
-        uint32_t L, h = 0;
-        if (K == 1) L = 2 * z + 1;
-        else { h = z + 1; L = h * (K + 1); }
-        if (L < 64 && L <= avail) {
-            const uint64_t v = K == 1 ? buf >> (64 - L) : (buf << h) >> (64 - K * h);
-            buf <<= L;
-            avail -= L;
-            return v;
-        }
-        uint64_t p = pos();  // long codeword (e.g. a segment's first residual): 64-bit window path, then re-seat
-        const uint64_t v = decode<K>(W, p);
-        init(W, p);
-        return v;
-    }
-};
 
 }  // namespace gcgt_dev

@@ -179,7 +179,9 @@ void write_vertex(uint64_t u, const Plan& pl, uint64_t deg, const gcgt_params& P
 
 }  // namespace
 
-extern "C" gcgt_status gcgt_encode(const gcgt_csr* csr, const gcgt_params* params, gcgt_cgr** out) {
+// Encodes rows 0..csr->n-1 as the records of vertices first .. first + csr->n - 1 of a graph of n_total vertices.
+static gcgt_status encode_rows(const gcgt_csr* csr, uint64_t first, uint64_t n_total, const gcgt_params* params,
+                               gcgt_cgr** out) {
     using gcgt_internal::fail;
     gcgt_internal::clear_error();
     if (!csr || !params || !out) return fail(GCGT_EINVAL, "null argument");
@@ -187,7 +189,7 @@ extern "C" gcgt_status gcgt_encode(const gcgt_csr* csr, const gcgt_params* param
     if (P.zeta_k < 1 || P.zeta_k > 5) return fail(GCGT_EINVAL, "zeta_k must be 1..5");
     if (P.min_interval_len == 1) return fail(GCGT_EINVAL, "min_interval_len must be 0 or >= 2");
     const uint64_t n = csr->n;
-    if (n > 0xFFFFFFFFull) return fail(GCGT_EINVAL, "n must fit in uint32");
+    if (n_total > 0xFFFFFFFFull || first + n > n_total) return fail(GCGT_EINVAL, "n must fit in uint32");
     if (n && (!csr->row_offsets || (!csr->cols && csr->row_offsets[n] > 0)))
         return fail(GCGT_EINVAL, "null CSR arrays");
     const uint64_t* ro = csr->row_offsets;
@@ -199,7 +201,7 @@ extern "C" gcgt_status gcgt_encode(const gcgt_csr* csr, const gcgt_params* param
     for (int64_t u = 0; u < (int64_t)n; u++) {
         if (ro[u + 1] < ro[u]) { bad = std::max(bad, 1); continue; }
         for (uint64_t e = ro[u]; e < ro[u + 1]; e++) {
-            if (cols[e] >= n) bad = std::max(bad, 2);
+            if (cols[e] >= n_total) bad = std::max(bad, 2);
             else if (e > ro[u] && cols[e] <= cols[e - 1]) bad = std::max(bad, 3);
         }
     }
@@ -211,6 +213,8 @@ extern "C" gcgt_status gcgt_encode(const gcgt_csr* csr, const gcgt_params* param
     try {
         g.reset(new gcgt_cgr());
         g->n = n;
+        g->base = first;
+        g->n_total = n_total;
         g->params = P;
         g->bit_offsets.assign(n + 1, 0);
     } catch (...) {
@@ -224,7 +228,7 @@ extern "C" gcgt_status gcgt_encode(const gcgt_csr* csr, const gcgt_params* param
 #pragma omp for schedule(dynamic, 1024)
         for (int64_t u = 0; u < (int64_t)n; u++) {
             if (err.load(std::memory_order_relaxed) != GCGT_OK) continue;
-            gcgt_status st = plan_vertex((uint64_t)u, cols + ro[u], ro[u + 1] - ro[u], P, pl);
+            gcgt_status st = plan_vertex(first + (uint64_t)u, cols + ro[u], ro[u + 1] - ro[u], P, pl);
             if (st != GCGT_OK) { err.store(st); continue; }
             g->bit_offsets[u + 1] = pl.bits;
         }
@@ -246,15 +250,93 @@ extern "C" gcgt_status gcgt_encode(const gcgt_csr* csr, const gcgt_params* param
         for (int64_t u = 0; u < (int64_t)n; u++) {
             const uint64_t b0 = g->bit_offsets[u], b1 = g->bit_offsets[u + 1];
             if (b1 == b0) continue;
-            plan_vertex((uint64_t)u, cols + ro[u], ro[u + 1] - ro[u], P, pl);
+            plan_vertex(first + (uint64_t)u, cols + ro[u], ro[u + 1] - ro[u], P, pl);
             Writer w{g->words.data(), b0, b0 >> 6, (b1 - 1) >> 6};
-            write_vertex((uint64_t)u, pl, ro[u + 1] - ro[u], P, w);
+            write_vertex(first + (uint64_t)u, pl, ro[u + 1] - ro[u], P, w);
         }
     }
     // words (stream order) -> canonical bytes in memory order
 #pragma omp parallel for schedule(static)
     for (int64_t i = 0; i < (int64_t)nwords; i++) g->words[i] = __builtin_bswap64(g->words[i]);
     *out = g.release();
+    return GCGT_OK;
+}
+
+extern "C" gcgt_status gcgt_encode(const gcgt_csr* csr, const gcgt_params* params, gcgt_cgr** out) {
+    return encode_rows(csr, 0, csr ? csr->n : 0, params, out);
+}
+
+extern "C" gcgt_status gcgt_encode_slice(const gcgt_csr* rows, uint64_t first, uint64_t n_total,
+                                         const gcgt_params* params, gcgt_cgr** out) {
+    return encode_rows(rows, first, n_total, params, out);
+}
+
+// Concatenation of consecutive vertex-range slices (R2: records are concatenated in vertex order, so the slices'
+// bit streams are appended at the running bit total and their offsets shifted by it).
+extern "C" gcgt_status gcgt_cgr_concat(const gcgt_cgr* const* parts, uint32_t k, gcgt_cgr** out) {
+    using gcgt_internal::fail;
+    gcgt_internal::clear_error();
+    if (!parts || !out || k == 0) return fail(GCGT_EINVAL, "null argument");
+    for (uint32_t i = 0; i < k; i++) {
+        if (!parts[i]) return fail(GCGT_EINVAL, "null part");
+        const gcgt_params& a = parts[i]->params;
+        const gcgt_params& b = parts[0]->params;
+        if (a.zeta_k != b.zeta_k || a.min_interval_len != b.min_interval_len ||
+            a.residual_segment_len != b.residual_segment_len || parts[i]->n_total != parts[0]->n_total)
+            return fail(GCGT_EINVAL, "parts differ in parameters or graph size");
+        if (i && parts[i]->base != parts[i - 1]->base + parts[i - 1]->n)
+            return fail(GCGT_EINVAL, "parts are not consecutive vertex ranges");
+    }
+    std::unique_ptr<gcgt_cgr> g;
+    std::vector<uint64_t> start(k + 1, 0);
+    for (uint32_t i = 0; i < k; i++) start[i + 1] = start[i] + parts[i]->nbits;
+    uint64_t n = 0;
+    for (uint32_t i = 0; i < k; i++) n += parts[i]->n;
+    try {
+        g.reset(new gcgt_cgr());
+        g->n = n;
+        g->base = parts[0]->base;
+        g->n_total = parts[0]->n_total;
+        g->params = parts[0]->params;
+        g->nbits = start[k];
+        g->bit_offsets.resize(n + 1);
+        g->words.assign((g->nbits + 63) / 64 + 2, 0);
+    } catch (...) {
+        return fail(GCGT_ENOMEM, "host allocation failed");
+    }
+    uint64_t v0 = 0;
+    for (uint32_t i = 0; i < k; i++) {
+        const gcgt_cgr* p = parts[i];
+        const uint64_t sh = start[i];
+#pragma omp parallel for schedule(static)
+        for (int64_t u = 0; u < (int64_t)p->n; u++) g->bit_offsets[v0 + u] = p->bit_offsets[u] + sh;
+        v0 += p->n;
+        // append the part's bits at bit `sh`: stream words (byte-swapped canonical words) shifted right by sh % 64;
+        // the first word is shared with the previous part (OR), the others are written whole
+        const uint64_t nw = (p->nbits + 63) / 64, w0 = sh / 64, s = sh % 64;
+        uint64_t* dst = g->words.data();
+        const uint64_t* src = p->words.data();
+        auto sw = [&](uint64_t j) { return j < nw ? __builtin_bswap64(src[j]) : 0ull; };
+        if (nw) {
+            const uint64_t first = sw(0) >> s;
+            dst[w0] = __builtin_bswap64(__builtin_bswap64(dst[w0]) | first);
+#pragma omp parallel for schedule(static)
+            for (int64_t j = 1; j <= (int64_t)nw; j++) {
+                const uint64_t v = (s ? sw(j - 1) << (64 - s) : 0ull) | (sw(j) >> s);
+                if (w0 + j < g->words.size()) dst[w0 + j] = __builtin_bswap64(v);
+            }
+        }
+    }
+    g->bit_offsets[n] = g->nbits;
+    *out = g.release();
+    return GCGT_OK;
+}
+
+extern "C" gcgt_status gcgt_cgr_slice_info(const gcgt_cgr* c, uint64_t* base, uint64_t* n_total) {
+    gcgt_internal::clear_error();
+    if (!c) return gcgt_internal::fail(GCGT_EINVAL, "null cgr");
+    if (base) *base = c->base;
+    if (n_total) *n_total = c->n_total;
     return GCGT_OK;
 }
 
@@ -305,6 +387,17 @@ static gcgt_status check_params(const gcgt_params& P) {
     return GCGT_OK;
 }
 
+// Shared validation of an externally supplied CGR (gcgt_cgr_from_arrays, gcgt_cgr_open): 32-bit vertex ids, bit
+// offsets starting at 0, non-decreasing, ending at nbits.  Corrupt tables would otherwise reach the device decoders.
+static gcgt_status check_offsets(uint64_t n, uint64_t nbits, const uint64_t* bit_offsets) {
+    using gcgt_internal::fail;
+    if (n >= 0xFFFFFFFFull) return fail(GCGT_EFORMAT, "n must fit 32-bit vertex ids");
+    if (bit_offsets[0] != 0 || bit_offsets[n] != nbits) return fail(GCGT_EFORMAT, "bit_offsets[0] != 0 or [n] != nbits");
+    for (uint64_t u = 0; u < n; u++)
+        if (bit_offsets[u + 1] < bit_offsets[u]) return fail(GCGT_EFORMAT, "bit_offsets decreasing");
+    return GCGT_OK;
+}
+
 extern "C" gcgt_status gcgt_cgr_from_arrays(uint64_t n, const uint8_t* bytes, uint64_t nbits,
                                             const uint64_t* bit_offsets, const gcgt_params* params,
                                             gcgt_cgr** out) {
@@ -312,12 +405,11 @@ extern "C" gcgt_status gcgt_cgr_from_arrays(uint64_t n, const uint8_t* bytes, ui
     gcgt_internal::clear_error();
     if (!bit_offsets || !params || !out || (nbits && !bytes)) return fail(GCGT_EINVAL, "null argument");
     if (check_params(*params) != GCGT_OK) return GCGT_EFORMAT;
-    if (bit_offsets[0] != 0 || bit_offsets[n] != nbits) return fail(GCGT_EFORMAT, "bit_offsets[n] != nbits");
-    for (uint64_t u = 0; u < n; u++)
-        if (bit_offsets[u + 1] < bit_offsets[u]) return fail(GCGT_EFORMAT, "bit_offsets decreasing");
+    if (gcgt_status st = check_offsets(n, nbits, bit_offsets)) return st;
     try {
         std::unique_ptr<gcgt_cgr> g(new gcgt_cgr());
         g->n = n;
+        g->n_total = n;
         g->nbits = nbits;
         g->params = *params;
         g->bit_offsets.assign(bit_offsets, bit_offsets + n + 1);
@@ -330,8 +422,8 @@ extern "C" gcgt_status gcgt_cgr_from_arrays(uint64_t n, const uint8_t* bytes, ui
     return GCGT_OK;
 }
 
-// File layout: "GCGTCGR1" | n u64 | nbits u64 | min_interval_len, residual_segment_len, zeta_k, 0 (u32 x4) |
-// bit_offsets u64[n+1] | bytes[ceil(nbits/8)].
+// File layout: "GCGTCGR2" | n u64 | nbits u64 | min_interval_len, residual_segment_len, zeta_k, 0 (u32 x4) |
+// base u64 | n_total u64 | bit_offsets u64[n+1] | bytes[ceil(nbits/8)].  ("GCGTCGR1" files: no base / n_total.)
 extern "C" gcgt_status gcgt_cgr_save(const gcgt_cgr* c, const char* path) {
     using gcgt_internal::fail;
     gcgt_internal::clear_error();
@@ -339,8 +431,8 @@ extern "C" gcgt_status gcgt_cgr_save(const gcgt_cgr* c, const char* path) {
     FILE* f = fopen(path, "wb");
     if (!f) return fail(GCGT_EINVAL, std::string("cannot open ") + path);
     const uint32_t pr[4] = {c->params.min_interval_len, c->params.residual_segment_len, c->params.zeta_k, 0};
-    bool ok = fwrite("GCGTCGR1", 1, 8, f) == 8 && fwrite(&c->n, 8, 1, f) == 1 && fwrite(&c->nbits, 8, 1, f) == 1 &&
-              fwrite(pr, 4, 4, f) == 4 &&
+    bool ok = fwrite("GCGTCGR2", 1, 8, f) == 8 && fwrite(&c->n, 8, 1, f) == 1 && fwrite(&c->nbits, 8, 1, f) == 1 &&
+              fwrite(pr, 4, 4, f) == 4 && fwrite(&c->base, 8, 1, f) == 1 && fwrite(&c->n_total, 8, 1, f) == 1 &&
               fwrite(c->bit_offsets.data(), 8, c->n + 1, f) == c->n + 1 &&
               fwrite(c->words.data(), 1, c->nbytes(), f) == c->nbytes();
     ok = (fclose(f) == 0) && ok;
@@ -354,17 +446,24 @@ extern "C" gcgt_status gcgt_cgr_open(const char* path, gcgt_cgr** out) {
     FILE* f = fopen(path, "rb");
     if (!f) return fail(GCGT_EINVAL, std::string("cannot open ") + path);
     char magic[8];
-    uint64_t n = 0, nbits = 0;
+    uint64_t n = 0, nbits = 0, base = 0, n_total = 0;
     uint32_t pr[4];
     gcgt_status st = GCGT_OK;
     std::unique_ptr<gcgt_cgr> g;
-    if (fread(magic, 1, 8, f) != 8 || memcmp(magic, "GCGTCGR1", 8) || fread(&n, 8, 1, f) != 1 ||
-        fread(&nbits, 8, 1, f) != 1 || fread(pr, 4, 4, f) != 4) {
+    bool v2 = false;
+    if (fread(magic, 1, 8, f) != 8 || (memcmp(magic, "GCGTCGR1", 8) && !(v2 = !memcmp(magic, "GCGTCGR2", 8))) ||
+        fread(&n, 8, 1, f) != 1 || fread(&nbits, 8, 1, f) != 1 || fread(pr, 4, 4, f) != 4 ||
+        (v2 && (fread(&base, 8, 1, f) != 1 || fread(&n_total, 8, 1, f) != 1))) {
         st = fail(GCGT_EFORMAT, "bad CGR file header");
+    } else if (!v2 && (n_total = n, false)) {
+    } else if (n >= 0xFFFFFFFFull || nbits / 8 > (1ull << 42) || n_total >= 0xFFFFFFFFull || base + n > n_total) {
+        st = fail(GCGT_EFORMAT, "CGR file header out of range");
     } else {
         try {
             g.reset(new gcgt_cgr());
             g->n = n;
+            g->base = base;
+            g->n_total = n_total;
             g->nbits = nbits;
             g->params = {pr[0], pr[1], pr[2]};
             g->bit_offsets.resize(n + 1);
@@ -375,9 +474,8 @@ extern "C" gcgt_status gcgt_cgr_open(const char* path, gcgt_cgr** out) {
         if (st == GCGT_OK && (fread(g->bit_offsets.data(), 8, n + 1, f) != n + 1 ||
                               fread(g->words.data(), 1, g->nbytes(), f) != g->nbytes()))
             st = fail(GCGT_EFORMAT, "truncated CGR file");
-        if (st == GCGT_OK && (check_params(g->params) != GCGT_OK || g->bit_offsets[0] != 0 ||
-                              g->bit_offsets[n] != nbits))
-            st = fail(GCGT_EFORMAT, "inconsistent CGR file");
+        if (st == GCGT_OK && check_params(g->params) != GCGT_OK) st = fail(GCGT_EFORMAT, "inconsistent CGR file");
+        if (st == GCGT_OK) st = check_offsets(n, nbits, g->bit_offsets.data());
     }
     fclose(f);
     if (st == GCGT_OK) *out = g.release();

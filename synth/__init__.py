@@ -44,6 +44,9 @@ def lib():
         L.syn_web.argtypes = [u64, d, u64, i32]
         L.syn_social.restype = p
         L.syn_social.argtypes = [u64, d, u64, u64, i32]
+        L.syn_rmat_slice.restype = p
+        L.syn_rmat_slice.argtypes = [i32, i32, u64, d, d, d, u64, u64]
+        L.syn_rmat_counts.argtypes = [i32, i32, u64, d, d, d, p]
         _lib = L
     return _lib
 
@@ -62,6 +65,27 @@ def _take(h):
 
 def rmat(scale: int, edgefactor: int = 16, seed: int = 1, A=0.57, B=0.19, Cc=0.19):
     return _take(lib().syn_rmat(scale, edgefactor, seed, A, B, Cc))
+
+
+def rmat_slice(scale: int, edgefactor: int, seed: int, lo: int, hi: int, A=0.57, B=0.19, Cc=0.19):
+    """Rows [lo, hi) of rmat(scale, edgefactor, seed) (global column ids), generated without the rest of the graph."""
+    return _take(lib().syn_rmat_slice(scale, edgefactor, seed, A, B, Cc, lo, hi))
+
+
+def rmat_slices(scale: int, edgefactor: int, seed: int, parts: int, A=0.57, B=0.19, Cc=0.19):
+    """Vertex-range boundaries (multiples of 32) splitting rmat(...) into `parts` slices of about equal arc counts
+    (from the pre-deduplication counts)."""
+    n = 1 << scale
+    counts = np.empty(n, dtype=np.uint32)
+    lib().syn_rmat_counts(scale, edgefactor, seed, A, B, Cc, counts.ctypes.data_as(C.c_void_p))
+    pre = np.concatenate([[0], np.cumsum(counts.astype(np.uint64))])
+    tot = int(pre[-1])
+    b = [0]
+    for r in range(1, parts):
+        v = int(np.searchsorted(pre, tot * r // parts)) // 32 * 32
+        b.append(max(b[-1], min(n, v)))
+    b.append(n)
+    return b
 
 
 def web(n: int, mean_deg: float = 16.1, seed: int = 2002, relabel: bool = True):
@@ -101,8 +125,10 @@ CONFIGS = {
     # configs[2]: twitter-like social graph (Table 1 :1423: 41.6M / 1.46B)
     "c3": Config("c3", "social", (41_652_230, 35.3, 3_000_000, 2010), False, 4, 32, 3,
                  "twitter-like social, 41.7M vertices"),
-    # configs[3]: uk-2007-like web graph (Table 1 :1421: 105.9M / 3.73B)
-    "c4": Config("c4", "web", (105_896_555, 33.5, 2007), False, 4, 32, 3, "uk-2007-like web, 105.9M vertices"),
+    # configs[3]: uk-2007-like web graph (Table 1 :1421: 105,896,555 vertices / 3,738,733,648 arcs).  The recipe's
+    # mean-degree knob is the pre-deduplication target: 45.9 gives 35.3 distinct arcs per vertex (calibrated on a
+    # 10M-vertex sample of the recipe: 44.0 -> 34.23, 46.0 -> 35.38), i.e. m ~ 3.74B
+    "c4": Config("c4", "web", (105_896_555, 45.9, 2007), False, 4, 32, 3, "uk-2007-like web, 105.9M vertices"),
     # configs[4]: R-MAT s29 ef16
     "c5": Config("c5", "rmat", (29, 16, 29), True, 4, 32, 3, "R-MAT s29 ef16 seed 29 (symmetrised)"),
     # scaled-down variants of the same recipes for parity tests (oracle finishes in seconds)

@@ -183,6 +183,95 @@ syn_graph* syn_rmat(int scale, int edgefactor, uint64_t seed, double A, double B
     }
 }
 
+// One vertex-range slice [lo, hi) of the same symmetrised R-MAT graph (syn_rmat), without materialising the rest:
+// every rank (or every pass of a single host) regenerates all edges from the counter-based streams and keeps the
+// arcs whose source lies in its range.  Rows are global ids, sorted and deduplicated, self-loops dropped; the rows of
+// consecutive slices concatenate to syn_rmat's CSR exactly (C5 at scale 29: 8.6B edges never held at once).
+syn_graph* syn_rmat_slice(int scale, int edgefactor, uint64_t seed, double A, double B, double C, uint64_t lo,
+                          uint64_t hi) {
+    try {
+        const uint64_t n = 1ull << scale, E = (uint64_t)edgefactor << scale;
+        if (hi > n) hi = n;
+        if (lo > hi) lo = hi;
+        const uint64_t nr = hi - lo;
+        auto edge = [&](uint64_t i, uint64_t& s, uint64_t& d) {
+            Rng r(seed, i);
+            s = d = 0;
+            for (int b = 0; b < scale; b++) {
+                double p = r.unif();
+                int q = p < A ? 0 : p < A + B ? 1 : p < A + B + C ? 2 : 3;
+                s = (s << 1) | (uint64_t)(q >> 1);
+                d = (d << 1) | (uint64_t)(q & 1);
+            }
+        };
+        std::vector<std::atomic<uint64_t>> cnt(nr + 1);
+        for (auto& x : cnt) x.store(0, std::memory_order_relaxed);
+#pragma omp parallel for schedule(static)
+        for (int64_t i = 0; i < (int64_t)E; i++) {
+            uint64_t s, d;
+            edge((uint64_t)i, s, d);
+            if (s == d) continue;
+            if (s >= lo && s < hi) cnt[s - lo].fetch_add(1, std::memory_order_relaxed);
+            if (d >= lo && d < hi) cnt[d - lo].fetch_add(1, std::memory_order_relaxed);
+        }
+        std::vector<uint64_t> off(nr + 1, 0);
+        for (uint64_t u = 0; u < nr; u++) off[u + 1] = off[u] + cnt[u].load();
+        std::vector<uint32_t> flat(off[nr]);
+        for (uint64_t u = 0; u < nr; u++) cnt[u].store(off[u], std::memory_order_relaxed);
+#pragma omp parallel for schedule(static)
+        for (int64_t i = 0; i < (int64_t)E; i++) {
+            uint64_t s, d;
+            edge((uint64_t)i, s, d);
+            if (s == d) continue;
+            if (s >= lo && s < hi) flat[cnt[s - lo].fetch_add(1)] = (uint32_t)d;
+            if (d >= lo && d < hi) flat[cnt[d - lo].fetch_add(1)] = (uint32_t)s;
+        }
+        Graph* g = new Graph();
+        g->n = nr;
+        g->rowoff.assign(nr + 1, 0);
+#pragma omp parallel for schedule(dynamic, 1024)
+        for (int64_t u = 0; u < (int64_t)nr; u++) {
+            uint32_t* b = flat.data() + off[u];
+            uint32_t* e = flat.data() + off[u + 1];
+            std::sort(b, e);
+            g->rowoff[u + 1] = (uint64_t)(std::unique(b, e) - b);
+        }
+        for (uint64_t u = 0; u < nr; u++) g->rowoff[u + 1] += g->rowoff[u];
+        g->cols.resize(g->rowoff[nr]);
+#pragma omp parallel for schedule(dynamic, 1024)
+        for (int64_t u = 0; u < (int64_t)nr; u++)
+            std::copy(flat.begin() + off[u], flat.begin() + off[u] + (g->rowoff[u + 1] - g->rowoff[u]),
+                      g->cols.begin() + g->rowoff[u]);
+        return (syn_graph*)g;
+    } catch (...) {
+        return nullptr;
+    }
+}
+
+// Per-vertex arc counts of the symmetrised R-MAT graph before deduplication (an upper bound on the degree), for
+// choosing arc-balanced vertex-range slices without generating the graph.
+int syn_rmat_counts(int scale, int edgefactor, uint64_t seed, double A, double B, double C, uint32_t* counts) {
+    const uint64_t n = 1ull << scale, E = (uint64_t)edgefactor << scale;
+    std::atomic<uint32_t>* c = reinterpret_cast<std::atomic<uint32_t>*>(counts);
+#pragma omp parallel for schedule(static)
+    for (int64_t v = 0; v < (int64_t)n; v++) counts[v] = 0;
+#pragma omp parallel for schedule(static)
+    for (int64_t i = 0; i < (int64_t)E; i++) {
+        Rng r(seed, (uint64_t)i);
+        uint64_t s = 0, d = 0;
+        for (int b = 0; b < scale; b++) {
+            double p = r.unif();
+            int q = p < A ? 0 : p < A + B ? 1 : p < A + B + C ? 2 : 3;
+            s = (s << 1) | (uint64_t)(q >> 1);
+            d = (d << 1) | (uint64_t)(q & 1);
+        }
+        if (s == d) continue;
+        c[s].fetch_add(1, std::memory_order_relaxed);
+        c[d].fetch_add(1, std::memory_order_relaxed);
+    }
+    return 0;
+}
+
 // Host-clustered web digraph (uk-2002 / uk-2007 shape):
 //  * hosts = contiguous id ranges, sizes power-law (alpha 1.6) in [4, 1e5];
 //  * out-degree power-law (alpha 2.1) in [1, 5000], ~8% dangling pages, rescaled to mean_deg;

@@ -102,6 +102,21 @@ def test_save_open_from_arrays(tmp_path):
     with pytest.raises(G.GcgtError) as e:
         G.from_arrays(b, nb, bad, *params)
     assert e.value.status == G.EFORMAT
+    # a file whose offsets decrease (corrupt table) is rejected like from_arrays rejects it
+    import struct
+    with open(path, "r+b") as f:
+        f.seek(8 + 8 + 8 + 16 + 8 * 3)
+        f.write(struct.pack("<Q", int(offs[5]) + 10_000_000))
+    with pytest.raises(G.GcgtError) as e:
+        G.open_cgr(path)
+    assert e.value.status == G.EFORMAT
+    cg.save(path)
+    with open(path, "r+b") as f:  # n >= 2^32 in the header
+        f.seek(8)
+        f.write(struct.pack("<Q", 1 << 33))
+    with pytest.raises(G.GcgtError) as e:
+        G.open_cgr(path)
+    assert e.value.status == G.EFORMAT
     with open(path, "r+b") as f:
         f.write(b"XXXX")
     with pytest.raises(G.GcgtError) as e:
@@ -152,3 +167,33 @@ def test_load_csr_validates_then_fails_loudly_without_gpu():
     with pytest.raises(G.GcgtError) as e:
         G.load_csr(ro, co)
     assert e.value.status == G.ECUDA
+
+
+@pytest.mark.parametrize("scale,parts", [(12, 3), (20, 4)])
+def test_rmat_slices_encode_like_the_whole_graph(scale, parts):
+    """C5's pipeline (§8(d) C5: R-MAT s29 cannot be held as one CSR): each vertex-range slice is generated alone
+    (synth.rmat_slice) and encoded alone (gcgt_encode_slice); the slices' CGRs concatenated are byte-identical to
+    the oracle's encoding of the whole graph, and each slice equals the whole CGR's bits of its range."""
+    import synth
+    ro, co = synth.rmat(scale, 16, 29)
+    n = ro.size - 1
+    b = synth.rmat_slices(scale, 16, 29, parts)
+    slices = []
+    for r in range(parts):
+        sro, sco = synth.rmat_slice(scale, 16, 29, b[r], b[r + 1])
+        s = G.encode_slice(sro, sco, b[r], n, 4, 32, 3)
+        assert G.slice_info(s) == (b[r], n)
+        slices.append(s)
+    whole = G.concat(slices)
+    wb, wnb, woffs, wn, _ = whole.view()
+    ob, onb, ooffs = O.encode_par(ro, co, 4, 32, 3)
+    assert (wn, wnb) == (n, onb) and np.array_equal(woffs, ooffs) and np.array_equal(wb, ob)
+    bits = np.unpackbits(ob)
+    for r, s in enumerate(slices):  # each slice = the whole stream's bits [offs[lo], offs[hi]), offsets re-based
+        sb, snb, soffs, sn, _ = s.view()
+        lo, hi = b[r], b[r + 1]
+        assert sn == hi - lo and np.array_equal(soffs, ooffs[lo:hi + 1] - ooffs[lo])
+        assert np.array_equal(np.unpackbits(sb)[:snb], bits[int(ooffs[lo]):int(ooffs[hi])])
+    with pytest.raises(G.GcgtError) as e:  # not consecutive
+        G.concat([slices[0], slices[-1]])
+    assert e.value.status == G.EINVAL

@@ -199,10 +199,9 @@ def test_warp_decoder_random_streams(k):
 # ---------------------------------------------------------------------------------------------------------------------
 # Direction-optimizing BFS (bottom-up levels over the in-CGR, §8 a9)
 # ---------------------------------------------------------------------------------------------------------------------
-@pytest.mark.parametrize("tune", ["", "bu_alpha=100000,bu_beta=1", "bu_alpha=100000,bu_beta=100000", "wpb_max=2",
-                                  "bu_alpha=100000,bu_beta=1,bu=2,bu_words=1,bu_batch=1", "bu=2",
-                                  "bu_alpha=100000,bu_beta=1,bu=2,bu_words=3,bu_batch=2", "fuse=1", "fuse=4,wpb_max=1",
-                                  "flatb=1", "nfilter=1", "persistent=1", "chunk=1", "chunk=16"])
+@pytest.mark.parametrize("tune", ["", "bu_alpha=100000,bu_beta=1", "bu_alpha=100000,bu_beta=100000", "graph=0",
+                                  "graph=0,bu_alpha=100000,bu_beta=1", "graph=0,chunk=2", "graph=0,chunk=16",
+                                  "hub_segs=1", "compact=0", "dir_bits=1", "dir_opt=0", "bu_alpha=1"])
 @pytest.mark.parametrize("name", ["c1", "rmat_s", "web_s", "social_s"])
 def test_bfs_direction_optimizing(name, tune, monkeypatch):
     """Symmetric graphs use the out-CGR as in-CGR; directed ones the encoded transpose.  The tunes force

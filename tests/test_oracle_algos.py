@@ -261,3 +261,18 @@ def test_bc_checksum(seed):
         lv = O.bfs(ro, co, s)
         ref += int((lv[lv > 0] - 1).sum())
     assert got == pytest.approx(ref, rel=1e-12)
+
+
+def test_bfs_cgr_sample_counts_whole_levels():
+    """The timing sample expands whole BFS levels until the arc budget is met: its arc count is the out-degree sum
+    of the vertices of the first L levels (for some L), at least the budget unless the BFS ran out."""
+    ro, co = random_graph(5000, 60000, seed=4)
+    b, nb, offs = O.encode(ro, co, 4, 32, 3)
+    ref = O.bfs(ro, co, 0)
+    deg = np.diff(ro.astype(np.int64))
+    per_level = [int(deg[ref == d].sum()) for d in range(ref.max() + 1)]
+    prefix = np.cumsum(per_level)
+    for budget in (1, 500, 5000, 20000, 10**12):
+        e = O.bfs_cgr_sample(b, offs, 4, 32, 3, 0, budget, 3)
+        assert e in set(prefix.tolist())
+        assert e >= budget or e == prefix[-1]
