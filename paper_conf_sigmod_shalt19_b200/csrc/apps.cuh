@@ -29,11 +29,20 @@ __device__ __forceinline__ void for_words(uint32_t s, uint32_t len, Fn&& fn) {
 struct BfsApp {
     const uint32_t* __restrict__ V;
     uint32_t* __restrict__ N;
+    uint32_t nfilter;  // 1: also skip targets an (L1-cached, possibly stale) read of N shows as already claimed
+    // N only gains bits during a level, so a stale read can only under-report claims: filtering on it never drops
+    // a discovery; it saves same-address reductions on popular targets (social graphs)
+    __device__ __forceinline__ static uint32_t ld_n(const uint32_t* p) {
+        uint32_t x;
+        asm volatile("ld.global.ca.u32 %0, [%1];" : "=r"(x) : "l"(p));
+        return x;
+    }
     __device__ __forceinline__ void begin(uint32_t) {}
     __device__ __forceinline__ void end() {}
     __device__ __forceinline__ void vertex(uint32_t) {}
     __device__ __forceinline__ void claim(uint32_t w, uint32_t mask) {
-        const uint32_t cand = mask & ~__ldg(V + w);
+        uint32_t cand = mask & ~__ldg(V + w);
+        if (cand && nfilter) cand &= ~ld_n(N + w);
         if (cand) red_or(N + w, cand);
     }
     __device__ __forceinline__ void one(uint32_t v) { claim(v >> 5, 1u << (v & 31)); }
@@ -41,6 +50,11 @@ struct BfsApp {
         uint32_t m[4];
 #pragma unroll
         for (uint32_t k = 0; k < 4; k++) m[k] = k < n ? __ldg(V + (v[k] >> 5)) : 0xffffffffu;
+        if (nfilter) {
+#pragma unroll
+            for (uint32_t k = 0; k < 4; k++)
+                if (!((m[k] >> (v[k] & 31)) & 1u)) m[k] |= ld_n(N + (v[k] >> 5));
+        }
 #pragma unroll
         for (uint32_t k = 0; k < 4; k++) {
             const uint32_t bit = 1u << (v[k] & 31);

@@ -27,27 +27,30 @@ __device__ __forceinline__ bool frontier_range(const uint32_t* __restrict__ F, u
 template <int K>
 __device__ __forceinline__ bool bu_residuals(GBitReader& r, uint32_t v, uint32_t cnt, const uint32_t* __restrict__ F,
                                              uint32_t& got, const volatile uint32_t* stop = nullptr) {
-    uint32_t cur = 0;
-    bool found = false;
-    for (uint32_t i = 0; i < cnt && !found; i += 4) {
+    if (cnt == 0) return false;
+    uint32_t cur = unmap_first32(v, r.template next<K>());
+    bool found = (__ldg(F + (cur >> 5)) >> (cur & 31)) & 1u;
+    uint32_t i = 1;
+    // whole batches of four: four decodes, then four frontier probes in flight together, one exit test
+    for (; !found && i + 4 <= cnt; i += 4) {
         if (stop && *stop) break;
-        const uint32_t k_n = min(4u, cnt - i);
         uint32_t id[4];
 #pragma unroll
         for (uint32_t k = 0; k < 4; k++) {
-            if (k < k_n) {
-                const uint64_t c = r.template next<K>();
-                cur = (i + k == 0) ? unmap_first32(v, c) : cur + (uint32_t)c;
-            }
+            cur += (uint32_t)r.template next<K>();
             id[k] = cur;
         }
         uint32_t fw[4];
 #pragma unroll
-        for (uint32_t k = 0; k < 4; k++) fw[k] = k < k_n ? __ldg(F + (id[k] >> 5)) : 0u;
+        for (uint32_t k = 0; k < 4; k++) fw[k] = __ldg(F + (id[k] >> 5));
 #pragma unroll
         for (uint32_t k = 0; k < 4; k++) found |= ((fw[k] >> (id[k] & 31)) & 1u) != 0;
-        got += k_n;
     }
+    for (; !found && i < cnt; i++) {  // tail
+        cur += (uint32_t)r.template next<K>();
+        found = (__ldg(F + (cur >> 5)) >> (cur & 31)) & 1u;
+    }
+    got += i;
     return found;
 }
 

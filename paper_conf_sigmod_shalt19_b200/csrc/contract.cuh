@@ -28,16 +28,17 @@ struct LevelState {
 };
 
 // Direction choice for the next BFS level (Beamer et al.'s heuristic, on vertex counts): switch to bottom-up when
-// the new frontier is large against the unvisited set and growing, back to top-down when it is small against n and
-// shrinking.  With use_bits (symmetric graphs) the top-down -> bottom-up test is Beamer's edge form with CGR bits as
+// the new frontier is large against the unvisited set (nf * alpha > unvisited) and growing, back to top-down when it
+// is small against n (nf * beta < n) and shrinking.  With use_bits (symmetric graphs) the top-down -> bottom-up test is Beamer's edge form with CGR bits as
 // the work measure: mf * alpha_bits > (unvisited vertices) * (mean record bits).
 struct DecideArgs {
     uint64_t n;
-    uint32_t alpha, beta;
+    uint32_t alpha10, beta;  // alpha in tenths
     int enabled;
     int use_bits;
     double bits_per_vertex;
-    uint32_t alpha_bits;
+    uint32_t alpha_bits10;  // in tenths
+    int grow;  // 1: switch to bottom-up only while the frontier grows (Beamer's condition)
 };
 
 struct CommitArgs {
@@ -52,8 +53,9 @@ struct CommitArgs {
     uint32_t* __restrict__ lvl_off;  // BC: queue offset of every level
     int32_t* __restrict__ levels;
     LevelState* ls;
-    unsigned long long* hub_ctr;   // reset for the next level
+    unsigned long long* hub_ctr;   // [2] hub segment / interval chunk queues, reset for the next level
     unsigned long long* hub_ctr2;  // (bottom-up hub queue) reset for the next level
+    unsigned long long* cursor;    // the expansion's work cursor [2], reset for the next level
     Offs offs_bits;                // record bits of the new frontier (used when use_mf)
     int use_mf;
     DecideArgs dec;
@@ -72,11 +74,11 @@ __device__ __forceinline__ void decide_body(volatile LevelState* ls, const Decid
     ls->visited = (uint32_t)visited;
     const uint64_t nu = d.n - visited, prev = ls->prev_nf;
     uint32_t dir = ls->dir;
-    bool to_bu = nf * d.alpha > nu;
-    if (d.use_bits) to_bu = (double)ls->mf * d.alpha_bits > (double)nu * d.bits_per_vertex;
+    bool to_bu = nf * d.alpha10 > nu * 10;
+    if (d.use_bits) to_bu = (double)ls->mf * d.alpha_bits10 > (double)nu * d.bits_per_vertex * 10.0;
     ls->mf = 0;
     if (!d.enabled || nf == 0) dir = 0;
-    else if (dir == 0 && to_bu && nf > prev) dir = 1;
+    else if (dir == 0 && to_bu && (nf > prev || !d.grow)) dir = 1;
     else if (dir == 1 && nf * d.beta < d.n && nf < prev) dir = 0;
     ls->dir = dir;
     ls->prev_nf = (uint32_t)nf;
@@ -106,13 +108,6 @@ __global__ void __launch_bounds__(kBlock) commit_kernel(CommitArgs a) {
             if (a.F && a.F[w] != b) a.F[w] = b;  // F = exactly the new frontier
         }
         nf += __popc(b);
-        if (a.use_mf && b) {
-            const uint64_t v0 = w * 32;
-            for (uint32_t m = b; m; m &= m - 1) {
-                const uint64_t v = v0 + __ffs(m) - 1;
-                mf += a.offs_bits(v + 1) - a.offs_bits(v);
-            }
-        }
         const uint32_t bal = __ballot_sync(0xffffffffu, b != 0);
         if (bal) {
             uint32_t pos = 0;
@@ -125,7 +120,11 @@ __global__ void __launch_bounds__(kBlock) commit_kernel(CommitArgs a) {
             for (uint32_t m = bal; m; m &= m - 1) {  // one coalesced 32-id store per new frontier word
                 const int j = __ffs(m) - 1;
                 const uint32_t bj = __shfl_sync(0xffffffffu, b, j);
-                if ((bj >> lane) & 1u) a.levels[(base + j) * 32 + lane] = new_level;
+                if ((bj >> lane) & 1u) {
+                    const uint64_t v = (base + j) * 32 + lane;
+                    a.levels[v] = new_level;
+                    if (a.use_mf) mf += a.offs_bits(v + 1) - a.offs_bits(v);  // coalesced offset reads
+                }
             }
         }
     }
@@ -143,8 +142,15 @@ __global__ void __launch_bounds__(kBlock) commit_kernel(CommitArgs a) {
             __threadfence();
             volatile LevelState* ls = a.ls;  // other blocks' counts arrived by atomics: read through L2
             ls->done = 0;
-            if (a.hub_ctr) *a.hub_ctr = 0;
+            if (a.hub_ctr) {
+                a.hub_ctr[0] = 0;
+                a.hub_ctr[1] = 0;
+            }
             if (a.hub_ctr2) *a.hub_ctr2 = 0;
+            if (a.cursor) {
+                a.cursor[0] = 0;
+                a.cursor[1] = 0;
+            }
             uint32_t next_len;
             if (a.bc) {
                 next_len = ls->q_next;

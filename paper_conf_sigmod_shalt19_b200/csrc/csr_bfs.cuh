@@ -117,14 +117,7 @@ __global__ void __launch_bounds__(kBlock, 4) csr_expand_kernel(const uint64_t* _
             __syncwarp();
         }
     }
-    add_stats3(st, nv, na, na * 32);
-    if (lane == 0) {  // the last warp out resets the work cursor for the next launch
-        const unsigned long long nwarp = (unsigned long long)gridDim.x * kWarps;
-        if (atomicAdd(cursor + 1, 1ull) == nwarp - 1) {
-            cursor[0] = 0;
-            cursor[1] = 0;
-        }
-    }
+    add_stats3(st, nv, na, na * 32);  // the work cursor is reset by the contraction
 }
 
 // Hub arcs of the level: warp per kCsrChunk-arc chunk (grid-stride), lanes stride the chunk (coalesced).

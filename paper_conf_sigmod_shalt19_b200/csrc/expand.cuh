@@ -29,6 +29,31 @@ struct HubEntry {
     uint32_t pad;
 };
 
+// Long interval areas.  A record with more than ck_c intervals decodes them as one serial chain (each gap is relative to
+// the previous interval's end, R10), which on a social hub (10^5 intervals) is milliseconds of one lane.  The load
+// step therefore builds a checkpoint table (the residual-segment idea of §5.2, :1092-1136, applied to intervals as a
+// derived device table; the CGR bytes are unchanged): for every such vertex, the bit position and the previous
+// interval end of every ck_c-th interval, and the position after the interval area.  The expansion hands the
+// vertex's interval chunks to the level's chunk queue, which the hub pass spreads over the grid like segments.
+struct IvEntry {
+    uint32_t u, ck0, nck, off;  // vertex, first checkpoint, chunks, first flattened chunk index
+    uint32_t itv, pad;
+};
+
+struct Checkpoints {
+    const uint32_t* __restrict__ wptr;  // per owned 32-vertex word: table rows before it
+    const uint32_t* __restrict__ bits;  // per owned word: which of its vertices have a row
+    const uint32_t* __restrict__ ck0;   // per row: first checkpoint (rows + 1 entries)
+    const uint64_t* __restrict__ after; // per row: bit position after the interval area
+    const uint64_t* __restrict__ pos;   // per checkpoint: bit position of the chunk's first gap code
+    const uint32_t* __restrict__ prev;  // per checkpoint: end of the interval before the chunk
+    const uint32_t* __restrict__ ilen;  // per row: total interval length (unsegmented records: residual count)
+    uint64_t w0;                        // first owned word
+    uint32_t ck_c;                      // intervals per chunk; rows exist for vertices with more than ck_c
+    IvEntry* q;                         // per-level chunk queue
+    unsigned long long* ctr;            // (entries << 32) | chunks
+};
+
 // Kernel-constant view of the device CGR plus the per-level hub queue.
 struct Ctx {
     const uint64_t* __restrict__ W;
@@ -40,6 +65,9 @@ struct Ctx {
     unsigned long long* cursor;   // [0] work cursor over the frontier queue, [1] finished-warp count
     const uint32_t* dir;          // BFS direction gate: top-down kernels run only while *dir == 0 (nullptr: always)
     uint32_t max_gran;            // records staged through shared memory up to this many granules (0: none)
+    uint32_t pool;                // phase B from a per-warp task pool filled over several rounds (lane refill)
+    uint32_t hub_stage;           // hub pass: segments staged through shared memory
+    Checkpoints ck;               // long interval areas (ck.bits == nullptr: none)
 };
 
 // ---- frontier sources ------------------------------------------------------------------------------------------------
@@ -94,10 +122,20 @@ struct DenseFront {
 template <int K, class R, class T>
 __device__ __forceinline__ uint32_t decode_segment(R& r, uint32_t u, T& t) {
     const uint32_t cnt = (uint32_t)(r.template next<K>() - 1);
-    uint32_t cur = 0;
-    for (uint32_t done = 0; done < cnt; done += 4) {
+    uint32_t cur = 0, done = 0;
+    for (; done + 4 <= cnt; done += 4) {  // whole batches of four: no per-id predicates
         uint32_t v[4];
-        const uint32_t nb = min(4u, cnt - done);
+#pragma unroll
+        for (uint32_t k = 0; k < 4; k++) {
+            const uint64_t c = r.template next<K>();
+            cur = (done + k == 0) ? unmap_first32(u, c) : cur + (uint32_t)c;
+            v[k] = cur;
+        }
+        t.many(v, 4);
+    }
+    if (done < cnt) {  // tail of 1..3
+        uint32_t v[4];
+        const uint32_t nb = cnt - done;
 #pragma unroll
         for (uint32_t k = 0; k < 4; k++) {
             if (k < nb) {
@@ -111,8 +149,10 @@ __device__ __forceinline__ uint32_t decode_segment(R& r, uint32_t u, T& t) {
     return cnt;
 }
 
-constexpr int kStageGran = 160;  // staging granules (16 B) per warp: 2.5 KB
+constexpr int kStageGran = 128;  // staging granules (16 B) per warp: 2 KB
 constexpr uint32_t kMaxVertexGran = 64;  // records above 8 Kbit are read from global memory
+constexpr uint32_t kPool = 160;   // phase-B task pool (segments of several rounds) per warp
+constexpr uint32_t kPoolFlush = kPool - 32 * 2;  // a round adds at most 32 x hub_segs (<= 2 when pooling) tasks
 
 struct ExpSmem {
     uint4 stage[kStageGran];
@@ -121,7 +161,33 @@ struct ExpSmem {
     uint32_t w[32], b[32], pre[33];
     uint32_t su[32], spre[33];
     uint64_t sbase[32];
+    uint64_t tpos[kPool];
+    uint32_t tu[kPool];
+    uint32_t ntask, take;
 };
+
+// Phase B from the pool: every lane takes the next segment task as soon as it finishes one (lane refill from a
+// shared-memory cursor), so a round's long segment no longer idles the other lanes; segments are read from global
+// memory (the pool outlives the round's staged records).
+template <int K, class App>
+__device__ __forceinline__ void drain_pool(const Ctx& c, const App& app, ExpSmem& sm, uint32_t& na) {
+    const uint32_t lane = lane_id();
+    const uint32_t N = sm.ntask;
+    if (lane == 0) sm.take = 32;
+    __syncwarp();
+    for (uint32_t k = lane; k < N; k = atomicAdd(&sm.take, 1u)) {
+        const uint32_t u = sm.tu[k];
+        GBitReader r;
+        r.init(reinterpret_cast<const uint32_t*>(c.W), 0, sm.tpos[k]);
+        App t = app;
+        t.begin(u);
+        na += decode_segment<K>(r, u, t);
+        t.end();
+    }
+    __syncwarp();
+    if (lane == 0) sm.ntask = 0;
+    __syncwarp();
+}
 
 __device__ __forceinline__ void lane_source(const ExpSmem& sm, const uint64_t* W, uint32_t o, const uint32_t*& src,
                                             uint64_t& j0) {
@@ -146,6 +212,10 @@ __device__ __forceinline__ void expand_body(const Ctx& c, const Front& fr, const
     }
     const uint64_t nstatic = (uint64_t)gridDim.x * kWarps * wpb;
     unsigned long long next = ((uint64_t)blockIdx.x * kWarps + wid) * wpb;
+    if (SEG && c.pool) {
+        if (lane == 0) sm.ntask = 0;
+        __syncwarp();
+    }
     for (;;) {
         const uint64_t base = __shfl_sync(0xffffffffu, next, 0);
         if (base >= qlen) break;
@@ -191,8 +261,19 @@ __device__ __forceinline__ void expand_body(const Ctx& c, const Front& fr, const
                 r.init(src, j0, p0);
                 uint64_t deg = 0;
                 if (!SEG) deg = r.template next<K>() - 1;
-                const uint32_t itv = (uint32_t)(r.template next<K>() - 1);
+                uint32_t itv = (uint32_t)(r.template next<K>() - 1);
                 uint32_t prev_end = 0, in_itv = 0;
+                if (itv > c.ck.ck_c && c.ck.bits) {  // long interval area: its chunks go grid-wide
+                    const uint64_t wl = (u >> 5) - c.ck.w0;
+                    const uint32_t row = c.ck.wptr[wl] + __popc(c.ck.bits[wl] & ((1u << (u & 31)) - 1));
+                    const uint32_t k0 = c.ck.ck0[row], nck = c.ck.ck0[row + 1] - k0;
+                    const unsigned long long old = atomicAdd(c.ck.ctr, (1ull << 32) | (unsigned long long)nck);
+                    c.ck.q[old >> 32] = IvEntry{u, k0, nck, (uint32_t)(old & 0xffffffffu), itv, 0};
+                    r.init(r.src, r.j0, c.ck.after[row]);
+                    itv = 0;
+                    in_itv = c.ck.ilen[row];  // counted as arcs by the chunk pass, not here
+                    na -= in_itv;
+                }
                 for (uint32_t i = 0; i < itv; i++) {
                     const uint64_t g = r.template next<K>();
                     const uint32_t len = (uint32_t)(r.template next<K>() - 1) + c.min_len;
@@ -230,7 +311,19 @@ __device__ __forceinline__ void expand_body(const Ctx& c, const Front& fr, const
                 }
                 t.end();
             }
-            if (SEG) {
+            if (SEG && c.pool) {
+                // ---- phase B (pooled): queue the round's segments; drain when the pool is nearly full
+                const uint32_t sincl = warp_incl_scan(nseg);
+                const uint32_t n0 = sm.ntask;
+                for (uint32_t k = 0; k < nseg; k++) {
+                    sm.tu[n0 + sincl - nseg + k] = u;
+                    sm.tpos[n0 + sincl - nseg + k] = sbase + (uint64_t)k * c.seg_bits;
+                }
+                __syncwarp();
+                if (lane == 31) sm.ntask = n0 + sincl;
+                __syncwarp();
+                if (sm.ntask >= kPoolFlush) drain_pool<K>(c, app, sm, na);
+            } else if (SEG) {
                 // ---- phase B: the round's residual segments, one per lane
                 const uint32_t sincl = warp_incl_scan(nseg);
                 sm.su[lane] = u;
@@ -258,6 +351,7 @@ __device__ __forceinline__ void expand_body(const Ctx& c, const Front& fr, const
         }
         __syncwarp();
     }
+    if (SEG && c.pool && sm.ntask) drain_pool<K>(c, app, sm, na);
 }
 
 template <int K, bool SEG, class App, class Front>
@@ -266,28 +360,24 @@ __global__ void __launch_bounds__(kBlock, 5) expand_kernel(Ctx c, Front fr, App 
     uint32_t nv = 0, na = 0, nb = 0;
     if (!(c.dir && *c.dir)) expand_body<K, SEG, App, Front>(c, fr, app, wpb, smem[threadIdx.x >> 5], nv, na, nb);
     add_stats3(c.st, nv, na, nb);
-    // the last block out resets the work cursor for the next launch
-    __syncthreads();
-    if (threadIdx.x == 0) {
-        if (atomicAdd(c.cursor + 1, 1ull) == gridDim.x - 1) {
-            c.cursor[0] = 0;
-            c.cursor[1] = 0;
-        }
-    }
+    // the work cursor is reset by the next contraction (or a memset by the caller): no per-block completion atomic
 }
 
 // ---- hub pass: the level's hub segments flattened over the whole grid -----------------------------------------------
 // A warp takes 32 consecutive flattened segments (usually 32 neighbouring segments of one hub, i.e. one contiguous
 // 1 KB run of fixed-stride segments, R16), finds their entries with one 32-ary ballot search, stages them with
 // coalesced 128-bit loads and decodes one segment per lane from shared memory.
-__device__ __forceinline__ uint32_t warp_find_hub(const HubEntry* __restrict__ q, uint32_t ne, uint32_t jb,
-                                                  uint32_t j) {
+__device__ __forceinline__ uint32_t entry_off(const HubEntry& e) { return e.seg_off; }
+__device__ __forceinline__ uint32_t entry_off(const IvEntry& e) { return e.off; }
+
+template <class E>
+__device__ __forceinline__ uint32_t warp_find_entry(const E* __restrict__ q, uint32_t ne, uint32_t jb, uint32_t j) {
     const uint32_t lane = lane_id();
     uint32_t lo = 0, hi = ne;  // invariant: off[lo] <= jb, and off[hi] > jb if hi < ne
     while (hi - lo > 1) {
         const uint32_t span = hi - lo;
         const uint32_t pos = span <= 32 ? lo + lane : lo + (uint32_t)(((uint64_t)span * lane) >> 5);
-        const bool le = (span > 32 || lane < span) && q[pos].seg_off <= jb;
+        const bool le = (span > 32 || lane < span) && entry_off(q[pos]) <= jb;
         const uint32_t L = 31 - __clz(__ballot_sync(0xffffffffu, le));
         if (span <= 32) {
             lo += L;
@@ -298,8 +388,47 @@ __device__ __forceinline__ uint32_t warp_find_hub(const HubEntry* __restrict__ q
         lo = nlo;
     }
     uint32_t e = lo;
-    while (e + 1 < ne && q[e + 1].seg_off <= j) e++;
+    while (e + 1 < ne && entry_off(q[e + 1]) <= j) e++;
     return e;
+}
+
+__device__ __forceinline__ uint32_t warp_find_hub(const HubEntry* __restrict__ q, uint32_t ne, uint32_t jb,
+                                                  uint32_t j) {
+    return warp_find_entry(q, ne, jb, j);
+}
+
+// The level's interval chunks (long interval areas, see Checkpoints): one chunk of ck_c intervals per lane, decoded from
+// its checkpoint and claimed as word ranges.
+template <int K, class App>
+__device__ __forceinline__ void chunk_pass(const Ctx& c, const App& app, uint32_t& na) {
+    const unsigned long long cc = *(volatile unsigned long long*)c.ck.ctr;
+    if (!cc) return;
+    const uint32_t lane = lane_id();
+    const uint32_t ne = (uint32_t)(cc >> 32), S = (uint32_t)(cc & 0xffffffffu);
+    const uint64_t gw0 = ((uint64_t)blockIdx.x * blockDim.x + threadIdx.x) & ~31ull;
+    const uint64_t stride = (uint64_t)gridDim.x * blockDim.x;
+    for (uint64_t jb = gw0; jb < S; jb += stride) {
+        const uint32_t j = (uint32_t)jb + lane;
+        const uint32_t k = warp_find_entry(c.ck.q, ne, (uint32_t)jb, min(j, S - 1));
+        if (j >= S) continue;
+        const IvEntry e = c.ck.q[k];
+        const uint32_t idx = j - e.off, ck = e.ck0 + idx;
+        const uint32_t cnt = min(c.ck.ck_c, e.itv - idx * c.ck.ck_c);
+        GBitReader r;
+        r.init(reinterpret_cast<const uint32_t*>(c.W), 0, c.ck.pos[ck]);
+        uint32_t prev_end = c.ck.prev[ck];
+        App t = app;
+        t.begin(e.u);
+        for (uint32_t i = 0; i < cnt; i++) {
+            const uint64_t g = r.template next<K>();
+            const uint32_t len = (uint32_t)(r.template next<K>() - 1) + c.min_len;
+            const uint32_t start = (idx == 0 && i == 0) ? unmap_first32(e.u, g) : prev_end + (uint32_t)g;
+            t.range(start, len);
+            prev_end = start + len - 1;
+            na += len;
+        }
+        t.end();
+    }
 }
 
 constexpr int kHubGran = 192;
@@ -313,12 +442,17 @@ struct HubSmem {
 template <int K, class App>
 __global__ void __launch_bounds__(kBlock) hub_kernel(Ctx c, App app) {
     __shared__ HubSmem smem[kWarps];
+    if (c.dir && *c.dir) return;  // a bottom-up level (host-driven loop)
+    uint32_t na = 0;
+    if (c.ck.bits) chunk_pass<K>(c, app, na);
     const unsigned long long hc = *(volatile unsigned long long*)c.hub_ctr;
-    if (hc == 0) return;  // no hub segments this level
+    if (hc == 0) {  // no hub segments this level
+        add_stats3(c.st, 0, na, 0);
+        return;
+    }
     HubSmem& sm = smem[threadIdx.x >> 5];
     const uint32_t lane = lane_id();
     const uint32_t nh = (uint32_t)(hc >> 32), S = (uint32_t)(hc & 0xffffffffu);
-    uint32_t na = 0;
     const uint64_t gw0 = ((uint64_t)blockIdx.x * blockDim.x + threadIdx.x) & ~31ull;
     const uint64_t stride = (uint64_t)gridDim.x * blockDim.x;
     for (uint64_t jb = gw0; jb < S; jb += stride) {
@@ -337,7 +471,7 @@ __global__ void __launch_bounds__(kBlock) hub_kernel(Ctx c, App app) {
         const uint32_t* src;
         uint64_t j0;
         stage_ranges<kHubGran>(reinterpret_cast<uint32_t*>(sm.stage), sm.owner, sm.sl, c.W, active, q, qe,
-                               c.max_gran ? 32u : 0u, src, j0);
+                               c.hub_stage ? 32u : 0u, src, j0);
         if (active) {
             BitReader r;
             r.init(src, j0, q);

@@ -61,8 +61,17 @@ struct DevCgr {
     uint32_t* rel = nullptr;    //                  u32 offset relative to the anchor
     uint64_t* full = nullptr;   // plain u64 offsets (when a 256-vertex block spans >= 2^32 bits)
     uint64_t lo = 0;
+    uint64_t base_bits = 0;     // stream bit of device word 0 (device bit positions = stream bits - base_bits)
     uint64_t offs_bytes = 0, word_bytes = 0;  // H2D volume (e2e accounting)
     Offs offs() const { return Offs{anc, rel, full, lo}; }
+};
+
+// Interval checkpoint table of the out-CGR (expand.cuh, Checkpoints), device arrays.
+struct DevCk {
+    uint32_t *wptr = nullptr, *bits = nullptr, *ck0 = nullptr, *prev = nullptr, *ilen = nullptr;
+    uint64_t *after = nullptr, *pos = nullptr;
+    IvEntry* q = nullptr;
+    uint64_t rows = 0, chunks = 0;
 };
 
 struct gcgt_graph {
@@ -75,6 +84,8 @@ struct gcgt_graph {
     uint64_t lo = 0, hi = 0;
     int rank = 0, nranks = 1;
     DevCgr out, in;
+    DevCk ck;
+    uint32_t ck_c = 32;  // intervals per checkpoint chunk (GCGT_TUNE ck_c; 0 = no table)
     bool in_alias = false;  // symmetric: in == out
     bool has_in = false;
     bool dir_opt = false;
@@ -93,12 +104,13 @@ struct gcgt_graph {
     uint32_t* lvl_off = nullptr;
     LevelState* ls = nullptr;
     HubEntry* hubq = nullptr;
-    unsigned long long* hub_ctr = nullptr;
+    unsigned long long* hub_ctr = nullptr;   // [0] hub segments, [1] interval chunks (entries << 32 | items)
     HubEntry* buq = nullptr;                 // deferred bottom-up hubs (in-records with many segments)
     unsigned long long* buq_ctr = nullptr;
     uint32_t* buq_done = nullptr;
     unsigned long long* cursor = nullptr;  // [0] work cursor, [1] finished blocks
     unsigned long long* st = nullptr;      // [vertices, arcs, bits]
+    unsigned long long* aux = nullptr;     // [4] counters of the partitioned steps (hooks, frontier size, scratch)
     uint32_t* src_dev = nullptr;           // BFS / BC source (graph replay reads it)
     int32_t* levels = nullptr;
     uint32_t* parent = nullptr;
@@ -114,15 +126,20 @@ struct gcgt_graph {
     int num_sms = 148;
     // knobs (GCGT_TUNE="key=value,..." at load; results never change)
     uint32_t hub_segs = 8;                  // more segments than this: the vertex's segments go grid-wide
-    uint32_t bu_hub_segs = 4;               // bottom-up: in-records with more segments are scanned grid-wide
-    uint32_t bu_alpha = 4, bu_beta = 128;   // direction switch on vertex counts (r1 session-4 sweep)
-    uint32_t alpha_bits = 30;
+    uint32_t bu_hub_segs = 0xFFFFFFFFu;     // bottom-up: in-records with more segments are scanned grid-wide (off:
+                                            // measured slower on C2 / C3, even on C4)
+    uint32_t bu_alpha = 40, bu_beta = 128;  // direction switch on vertex counts; alpha in tenths (r2 sweeps, C2-C4)
+    uint32_t alpha_bits = 25;               // tenths
+    bool bu_grow = true;                    // Beamer's "frontier growing" condition for the switch to bottom-up
+    bool nfilter = false;                   // BFS filter: also test an L1 read of N before the claim
+    bool hub_stage = true;                  // hub pass: segments staged through shared memory
     bool dir_bits = false;
     bool dir_opt_knob = true;
     bool use_graph = true;                  // BFS as one CUDA graph (else: chunked host-driven level loop)
     uint32_t chunk = 4;                     // host-driven loop: levels enqueued per host check
     bool compact_offs = true;
     bool td_stage = true;  // top-down: records staged through shared memory with coalesced 128-bit loads
+    bool td_pool = false;  // top-down: phase B from a per-warp segment pool with lane refill (hub_segs capped at 2)
     // BFS graph (built on first use for a given levels buffer)
     cudaGraphExec_t bfs_exec = nullptr;
     int32_t* bfs_exec_levels = nullptr;
@@ -143,6 +160,12 @@ namespace {
 
 inline int flat_grid(const gcgt_graph* g, uint64_t n) {
     return (int)std::max<uint64_t>(1, std::min<uint64_t>((n + kBlock - 1) / kBlock, (uint64_t)g->num_sms * 16));
+}
+
+// The contraction closes each level with one completion atomic per block: 4 blocks per SM keep that serial tail short
+// while the dense scan still has 32 warps per SM.
+inline int commit_grid(const gcgt_graph* g) {
+    return (int)std::max<uint64_t>(1, std::min<uint64_t>((g->nw + kBlock - 1) / kBlock, (uint64_t)g->num_sms * 4));
 }
 
 // ---- dispatch over the template parameters (zeta_k, segmented) ------------------------------------------------------
@@ -171,12 +194,16 @@ inline int occupancy(T kernel) {
 
 inline Ctx make_ctx(const gcgt_graph* g) {
     return Ctx{g->out.W, g->out.offs(), g->P.min_interval_len, 8 * g->P.residual_segment_len, g->hub_segs,
-               g->hubq, g->hub_ctr, g->st, g->cursor, nullptr, g->td_stage ? kMaxVertexGran : 0u};
+               g->hubq, g->hub_ctr, g->st, g->cursor, nullptr, g->td_stage ? kMaxVertexGran : 0u,
+               g->td_pool ? 1u : 0u, g->hub_stage ? 1u : 0u,
+               Checkpoints{g->ck.wptr, g->ck.bits, g->ck.ck0, g->ck.after, g->ck.pos, g->ck.prev, g->ck.ilen,
+                           g->lo >> 5, g->ck_c, g->ck.q, g->hub_ctr + 1}};
 }
 
 // Top-down expansion (+ hub pass) of one frontier: a persistent grid at the kernel's occupancy.
 template <class App, class Front>
-inline void launch_expand(gcgt_graph* g, cudaStream_t s, const Ctx& c, const Front& fr, const App& app) {
+inline void launch_expand(gcgt_graph* g, cudaStream_t s, const Ctx& c, const Front& fr, const App& app,
+                          bool reset = true) {
     with_k(g->P, [&](auto KK, auto SS) {
         constexpr int K = decltype(KK)::value;
         constexpr bool SEG = decltype(SS)::value;
@@ -184,12 +211,16 @@ inline void launch_expand(gcgt_graph* g, cudaStream_t s, const Ctx& c, const Fro
         if (!occ) occ = occupancy(expand_kernel<K, SEG, App, Front>);
         expand_kernel<K, SEG, App, Front><<<occ * g->num_sms, kBlock, 0, s>>>(c, fr, app, 0u);
         g->launches++;
-        if (SEG) {
+        if (SEG || g->ck.bits) {  // hub segments and / or interval chunks
             if (!occh) occh = occupancy(hub_kernel<K, App>);
             hub_kernel<K, App><<<occh * g->num_sms, kBlock, 0, s>>>(c, app);
             g->launches++;
         }
     });
+    if (reset) {  // the work cursor and hub queue for the next launch (the BFS / BC contraction does this itself)
+        cudaMemsetAsync(g->cursor, 0, 16, s);
+        cudaMemsetAsync(g->hub_ctr, 0, 16, s);
+    }
 }
 
 inline void launch_bu(gcgt_graph* g, cudaStream_t s, const uint32_t* V, const uint32_t* F, uint32_t* N,
@@ -336,6 +367,7 @@ gcgt_status upload_cgr(gcgt_graph* g, const gcgt_cgr* c, uint64_t lo, uint64_t h
     const uint64_t avail = c->words.size() > w0 ? std::min<uint64_t>(c->words.size() - w0, nwords) : 0;
     gcgt_status st;
     d->lo = lo;
+    d->base_bits = w0 * 64;
     d->word_bytes = nwords * 8;
     if (host_resident) {
         CU(cudaHostAlloc((void**)&d->hostW, nwords * sizeof(uint64_t), cudaHostAllocMapped | cudaHostAllocPortable));
@@ -392,6 +424,108 @@ uint64_t count_hub_bound(const gcgt_cgr* c, uint64_t lo, uint64_t hi, uint64_t m
     return cnt;
 }
 
+// Host reader of the canonical MSB-first bytes (FORMAT.md R1), for the load-time checkpoint table only.
+struct HostBits {
+    const uint8_t* b;
+    int bit(uint64_t i) const { return (b[i >> 3] >> (7 - (i & 7))) & 1; }
+    uint64_t read(uint32_t K, uint64_t& p) const {  // one VLC codeword (App. B; FORMAT.md R3/R4)
+        uint64_t z = 0;
+        while (!bit(p)) { z++; p++; }
+        uint64_t payload;
+        if (K == 1) payload = z + 1;
+        else { p++; payload = (z + 1) * K; }
+        uint64_t v = 0;
+        for (uint64_t t = 0; t < payload; t++) v = (v << 1) | (uint64_t)bit(p + t);
+        p += payload;
+        return v;
+    }
+};
+
+// Interval checkpoint table (expand.cuh, Checkpoints) for the owned vertices with more than ck_c intervals: decoded
+// once on the host (the header of every vertex, the interval area of the few long ones), uploaded as device tables.
+gcgt_status build_checkpoints(gcgt_graph* g, const gcgt_cgr* c) {
+    const uint32_t C = g->ck_c;
+    if (C == 0 || g->hi == g->lo) return GCGT_OK;
+    const uint64_t lo = g->lo, hi = g->hi, nloc = hi - lo, base = g->out.base_bits;
+    const uint64_t* bo = c->bit_offsets.data() - c->base;
+    const HostBits hb{reinterpret_cast<const uint8_t*>(c->words.data())};
+    const bool seg = g->P.residual_segment_len != 0;
+    const uint32_t K = g->P.zeta_k;
+    std::vector<uint32_t> itv(nloc, 0);
+#pragma omp parallel for schedule(dynamic, 65536)
+    for (int64_t i = 0; i < (int64_t)nloc; i++) {
+        uint64_t p = bo[lo + i];
+        if (p == bo[lo + i + 1]) continue;
+        if (!seg) hb.read(K, p);
+        const uint64_t x = hb.read(K, p) - 1;
+        if (x > C) itv[i] = (uint32_t)x;
+    }
+    const uint64_t w0 = lo >> 5, nwl = ((hi + 31) >> 5) - w0;
+    std::vector<uint32_t> wptr(nwl + 1, 0), bits(nwl, 0), rows_u;
+    for (uint64_t i = 0; i < nloc; i++)
+        if (itv[i]) {
+            const uint64_t v = lo + i;
+            bits[(v >> 5) - w0] |= 1u << (v & 31);
+            rows_u.push_back((uint32_t)v);
+        }
+    if (rows_u.empty()) return GCGT_OK;
+    for (uint64_t w = 0; w < nwl; w++) wptr[w + 1] = wptr[w] + __builtin_popcount(bits[w]);
+    const uint64_t R = rows_u.size();
+    std::vector<uint32_t> ck0(R + 1, 0), ilen(R, 0);
+    std::vector<uint64_t> after(R, 0);
+    for (uint64_t r = 0; r < R; r++) ck0[r + 1] = ck0[r] + (itv[rows_u[r] - lo] + C - 1) / C;
+    const uint64_t T = ck0[R];
+    std::vector<uint64_t> pos(T);
+    std::vector<uint32_t> prev(T);
+#pragma omp parallel for schedule(dynamic, 1)
+    for (int64_t r = 0; r < (int64_t)R; r++) {
+        const uint64_t u = rows_u[r];
+        const uint32_t n_itv = itv[u - lo];
+        uint64_t p = bo[u];
+        if (!seg) hb.read(K, p);
+        hb.read(K, p);
+        int64_t prev_end = 0;
+        uint64_t sum = 0;
+        for (uint32_t t = 0; t < n_itv; t++) {
+            if (t % C == 0) {
+                pos[ck0[r] + t / C] = p - base;
+                prev[ck0[r] + t / C] = (uint32_t)prev_end;
+            }
+            const uint64_t gcode = hb.read(K, p);
+            const uint64_t len = hb.read(K, p) - 1 + g->P.min_interval_len;
+            int64_t start;
+            if (t == 0) {
+                const uint64_t z = gcode - 1;
+                start = (int64_t)u + ((z & 1) ? -(int64_t)(z >> 1) : (int64_t)(z >> 1));  // R9
+            } else {
+                start = prev_end + (int64_t)gcode;  // R10
+            }
+            prev_end = start + (int64_t)len - 1;
+            sum += len;
+        }
+        after[r] = p - base;
+        ilen[r] = (uint32_t)sum;
+    }
+    DevCk& d = g->ck;
+    gcgt_status st;
+    if ((st = galloc(g, &d.wptr, nwl + 1)) || (st = galloc(g, &d.bits, nwl)) || (st = galloc(g, &d.ck0, R + 1)) ||
+        (st = galloc(g, &d.after, R)) || (st = galloc(g, &d.ilen, R)) || (st = galloc(g, &d.pos, T)) ||
+        (st = galloc(g, &d.prev, T)) || (st = galloc(g, &d.q, R + 1)))
+        return st;
+    cudaStream_t s = g->stream;
+    CU(cudaMemcpyAsync(d.wptr, wptr.data(), (nwl + 1) * 4, cudaMemcpyHostToDevice, s));
+    CU(cudaMemcpyAsync(d.bits, bits.data(), nwl * 4, cudaMemcpyHostToDevice, s));
+    CU(cudaMemcpyAsync(d.ck0, ck0.data(), (R + 1) * 4, cudaMemcpyHostToDevice, s));
+    CU(cudaMemcpyAsync(d.after, after.data(), R * 8, cudaMemcpyHostToDevice, s));
+    CU(cudaMemcpyAsync(d.ilen, ilen.data(), R * 4, cudaMemcpyHostToDevice, s));
+    CU(cudaMemcpyAsync(d.pos, pos.data(), T * 8, cudaMemcpyHostToDevice, s));
+    CU(cudaMemcpyAsync(d.prev, prev.data(), T * 4, cudaMemcpyHostToDevice, s));
+    CU(cudaStreamSynchronize(s));  // host vectors
+    d.rows = R;
+    d.chunks = T;
+    return GCGT_OK;
+}
+
 void parse_tune(gcgt_graph* g) {
     const char* tune = getenv("GCGT_TUNE");  // development knob: key=value,... (results never change)
     if (!tune) return;
@@ -415,6 +549,11 @@ void parse_tune(gcgt_graph* g) {
             else if (k == "chunk") g->chunk = (uint32_t)std::max(2ul, std::min(32ul, v & ~1ul));
             else if (k == "compact") g->compact_offs = v != 0;
             else if (k == "td_stage") g->td_stage = v != 0;
+            else if (k == "td_pool") g->td_pool = v != 0;
+            else if (k == "ck_c") g->ck_c = (uint32_t)v;
+            else if (k == "bu_grow") g->bu_grow = v != 0;
+            else if (k == "nfilter") g->nfilter = v != 0;
+            else if (k == "hub_stage") g->hub_stage = v != 0;
             else if (k == "bu_hub_segs") g->bu_hub_segs = (uint32_t)v;  // 0xFFFFFFFF (or huge): no deferral
         }
         i = j + 1;
@@ -447,6 +586,7 @@ gcgt_status init_graph(gcgt_graph* g, const gcgt_load_opts& o) {
     CU(cudaEventCreate(&g->ev1));
     for (auto& e : g->sev) CU(cudaEventCreate(&e));
     parse_tune(g);
+    if (g->td_pool) g->hub_segs = std::min<uint32_t>(g->hub_segs, 2);  // a pooled round adds <= 32 x 2 tasks
     return GCGT_OK;
 }
 
@@ -455,12 +595,13 @@ gcgt_status alloc_work(gcgt_graph* g) {
     gcgt_status st;
     g->nw = ((g->n + 31) / 32 + 1 + 3) & ~3ull;
     if ((st = galloc(g, &g->V, g->nw)) || (st = galloc(g, &g->F, g->nw)) || (st = galloc(g, &g->N, g->nw)) ||
-        (st = galloc(g, &g->q, 2 * g->nw)) || (st = galloc(g, &g->ls, 1)) || (st = galloc(g, &g->hub_ctr, 1)) ||
-        (st = galloc(g, &g->cursor, 2)) || (st = galloc(g, &g->st, 3)) || (st = galloc(g, &g->src_dev, 1)))
+        (st = galloc(g, &g->q, 2 * g->nw)) || (st = galloc(g, &g->ls, 1)) || (st = galloc(g, &g->hub_ctr, 2)) ||
+        (st = galloc(g, &g->cursor, 2)) || (st = galloc(g, &g->st, 3)) || (st = galloc(g, &g->src_dev, 1)) ||
+        (st = galloc(g, &g->aux, 4)))
         return st;
     CU(cudaMemsetAsync(g->N, 0, g->nw * 4, g->stream));
     CU(cudaMemsetAsync(g->cursor, 0, 16, g->stream));
-    CU(cudaMemsetAsync(g->hub_ctr, 0, 8, g->stream));
+    CU(cudaMemsetAsync(g->hub_ctr, 0, 16, g->stream));
     CU(cudaMemsetAsync(g->ls, 0, sizeof(LevelState), g->stream));
     return GCGT_OK;
 }
@@ -472,7 +613,7 @@ gcgt_status ensure_levels(gcgt_graph* g) {
 
 DecideArgs decide_args(const gcgt_graph* g) {
     return DecideArgs{g->n, g->bu_alpha, g->bu_beta, g->dir_opt ? 1 : 0, g->dir_bits && g->dir_opt ? 1 : 0,
-                      (double)g->nbits / (double)std::max<uint64_t>(1, g->n), g->alpha_bits};
+                      (double)g->nbits / (double)std::max<uint64_t>(1, g->n), g->alpha_bits, g->bu_grow ? 1 : 0};
 }
 
 CommitArgs bfs_commit_args(gcgt_graph* g, int parity, int32_t* lv) {
@@ -489,6 +630,7 @@ CommitArgs bfs_commit_args(gcgt_graph* g, int parity, int32_t* lv) {
     a.ls = g->ls;
     a.hub_ctr = g->hub_ctr;
     a.hub_ctr2 = g->buq_ctr;
+    a.cursor = g->cursor;
     a.dec = decide_args(g);
     a.use_mf = a.dec.use_bits;
     if (a.use_mf && !g->is_csr) a.offs_bits = g->out.offs();
@@ -507,7 +649,7 @@ namespace {
 gcgt_status enqueue_td(gcgt_graph* g, cudaStream_t s, int p) {
     const uint32_t* dir = g->dir_opt ? &g->ls->dir : nullptr;
     const QueueFront fr{g->q + (uint64_t)p * g->nw, &g->ls->qlen[p], g->F, nullptr};
-    const BfsApp app{g->V, g->N};
+    const BfsApp app{g->V, g->N, g->nfilter ? 1u : 0u};
     if (g->is_csr) {
         static int occ = 0;
         if (!occ) occ = occupancy(csr_expand_kernel<QueueFront>);
@@ -519,7 +661,7 @@ gcgt_status enqueue_td(gcgt_graph* g, cudaStream_t s, int p) {
     }
     Ctx c = make_ctx(g);
     c.dir = dir;
-    launch_expand(g, s, c, fr, app);
+    launch_expand(g, s, c, fr, app, false);
     return GCGT_OK;
 }
 
@@ -544,7 +686,7 @@ gcgt_status enqueue_commit(gcgt_graph* g, cudaStream_t s, int p, int32_t* lv, in
     a.cond = cond;
     a.use_dcond = use_dcond;
     a.dcond = dcond;
-    commit_kernel<<<flat_grid(g, g->nw * 32), kBlock, 0, s>>>(a);
+    commit_kernel<<<commit_grid(g), kBlock, 0, s>>>(a);
     g->launches++;
     return GCGT_OK;
 }
@@ -649,7 +791,8 @@ extern "C" void gcgt_unload(gcgt_graph* g) {
                     g->in_alias ? nullptr : (g->in.hostW ? nullptr : g->in.W), g->in_alias ? nullptr : g->in.anc,
                     g->in_alias ? nullptr : g->in.rel, g->in_alias ? nullptr : g->in.full,
                     g->V, g->F, g->N, g->q, g->qbits, g->lvl_off, g->ls, g->hubq, g->hub_ctr, g->cursor, g->st,
-                    g->buq, g->buq_ctr, g->buq_done,
+                    g->buq, g->buq_ctr, g->buq_done, g->aux, g->ck.wptr, g->ck.bits, g->ck.ck0, g->ck.after,
+                    g->ck.ilen, g->ck.pos, g->ck.prev, g->ck.q,
                     g->src_dev, g->levels, g->parent, g->dirty, g->sigma, g->delta, g->bc,
                     g->crow, g->ccol, g->csr_hubq,
                     g->csr_in_owned ? g->crow_in : nullptr, g->csr_in_owned ? g->ccol_in : nullptr};
@@ -730,6 +873,7 @@ extern "C" gcgt_status gcgt_load(const gcgt_cgr* c, const gcgt_load_opts* opts, 
     const uint64_t seg_bits = 8ull * g->P.residual_segment_len;
     const uint64_t nhub = seg_bits ? count_hub_bound(c, g->lo, g->hi, (uint64_t)g->hub_segs * seg_bits) : 0;
     if ((st = galloc(g.get(), &g->hubq, nhub + 1))) return st;
+    if ((st = build_checkpoints(g.get(), c))) return st;
     if (g->has_in && seg_bits && g->bu_hub_segs < 0xFFFFu) {
         const gcgt_cgr* ic = o.in_cgr ? o.in_cgr : c;
         const uint64_t nbh = count_hub_bound(ic, g->lo, g->hi, (uint64_t)g->bu_hub_segs * seg_bits);
@@ -893,7 +1037,7 @@ extern "C" gcgt_status gcgt_bfs(gcgt_graph* g, uint32_t source, int32_t* levels,
         const LevelState* h = g->h_ls();
         stats->iterations = h->nonempty + 1;  // non-empty levels (the seed level included)
         if (graph) {  // kernels the graph ran: per level the expansion kernel(s) of its direction + the contraction
-            const uint32_t td_kernels = g->is_csr ? 2 : (g->P.residual_segment_len ? 2 : 1);
+            const uint32_t td_kernels = g->is_csr ? 2 : ((g->P.residual_segment_len || g->ck.bits) ? 2 : 1);
             stats->launches += (uint64_t)h->ntd * td_kernels + h->nbu + h->ntd + h->nbu;
         }
     }
@@ -915,7 +1059,7 @@ extern "C" gcgt_status gcgt_cc(gcgt_graph* g, uint32_t* labels, int placement, g
         lab = g->parent;
     }
     cc_init<<<flat_grid(g, g->n), kBlock, 0, s>>>(lab, g->n);
-    CU(cudaMemsetAsync(g->hub_ctr, 0, 8, s));
+    CU(cudaMemsetAsync(g->hub_ctr, 0, 16, s));
     const Ctx c = make_ctx(g);
     const DenseFront fr{g->lo, g->hi};
     const CcApp app{lab, nullptr, nullptr, 0, 0};  // single GPU: no hook counting
@@ -923,7 +1067,7 @@ extern "C" gcgt_status gcgt_cc(gcgt_graph* g, uint32_t* labels, int placement, g
     launch_expand(g, s, c, fr, app);
     if ((st = kprof_end(g, s))) return st;
     cc_jump<<<flat_grid(g, g->n), kBlock, 0, s>>>(lab, g->n);
-    CU(cudaMemsetAsync(g->hub_ctr, 0, 8, s));
+    CU(cudaMemsetAsync(g->hub_ctr, 0, 16, s));
     g->launches += 2;
     if ((st = copy_out(g, labels, lab, g->n * 4, placement))) return st;
     CU(cudaStreamSynchronize(s));
@@ -961,7 +1105,7 @@ extern "C" gcgt_status gcgt_bc(gcgt_graph* g, const uint32_t* sources, uint32_t 
     cudaStream_t s = g->stream;
     const Ctx c = make_ctx(g);
     CU(cudaMemsetAsync(g->bc, 0, g->n * 8, s));
-    CU(cudaMemsetAsync(g->hub_ctr, 0, 8, s));
+    CU(cudaMemsetAsync(g->hub_ctr, 0, 16, s));
     std::vector<uint32_t> lvl_off;
     for (uint32_t si = 0; si < k; si++) {
         *g->h_src() = sources[si];
@@ -977,7 +1121,7 @@ extern "C" gcgt_status gcgt_bc(gcgt_graph* g, const uint32_t* sources, uint32_t 
                 const QueueFront fr{g->q, &g->ls->q_len, nullptr, g->qbits, &g->ls->q_off};
                 const BcFwdApp app{g->V, g->N, g->sigma, 0.0};
                 if ((st = kprof_begin(g, s))) return st;
-                launch_expand(g, s, c, fr, app);
+                launch_expand(g, s, c, fr, app, false);
                 if ((st = kprof_end(g, s))) return st;
                 CommitArgs a{};
                 a.V = g->V;
@@ -990,8 +1134,9 @@ extern "C" gcgt_status gcgt_bc(gcgt_graph* g, const uint32_t* sources, uint32_t 
                 a.levels = g->levels;
                 a.ls = g->ls;
                 a.hub_ctr = g->hub_ctr;
+                a.cursor = g->cursor;
                 a.bc = 1;
-                commit_kernel<<<flat_grid(g, g->nw * 32), kBlock, 0, s>>>(a);
+                commit_kernel<<<commit_grid(g), kBlock, 0, s>>>(a);
                 g->launches++;
             }
             CU(cudaMemcpyAsync(g->h_ls(), g->ls, sizeof(LevelState), cudaMemcpyDeviceToHost, s));
@@ -1009,7 +1154,7 @@ extern "C" gcgt_status gcgt_bc(gcgt_graph* g, const uint32_t* sources, uint32_t 
             const QueueFront fr{g->q + off, nullptr, nullptr, g->qbits + off, nullptr, lvl_off[d + 1] - off};
             const BcBwdApp app{g->levels, g->sigma, g->delta, g->bc, d + 1, sources[si], 0, 0.0, 0.0};
             launch_expand(g, s, c, fr, app);
-            CU(cudaMemsetAsync(g->hub_ctr, 0, 8, s));
+            CU(cudaMemsetAsync(g->hub_ctr, 0, 16, s));
         }
     }
     if ((st = copy_out(g, bc, g->bc, g->n * 8, placement))) return st;
@@ -1036,7 +1181,7 @@ extern "C" gcgt_status gcgt_dist_bfs_begin(gcgt_graph* g, uint32_t source) {
     CU(cudaMemsetAsync(g->V, 0, g->nw * 4, s));
     CU(cudaMemsetAsync(g->F, 0, g->nw * 4, s));
     CU(cudaMemsetAsync(g->levels, 0xff, g->n * 4, s));
-    CU(cudaMemsetAsync(g->hub_ctr, 0, 8, s));
+    CU(cudaMemsetAsync(g->hub_ctr, 0, 16, s));
     seed_kernel<<<1, 1, 0, s>>>(g->src_dev, g->V, g->F, g->q, nullptr, g->levels, g->ls, nullptr, nullptr);
     return GCGT_OK;
 }
@@ -1068,9 +1213,9 @@ extern "C" gcgt_status gcgt_dist_bfs_expand(gcgt_graph* g, uint32_t level, uint3
     CU(cudaMemsetAsync(cand, 0, nwf * 4, s));
     const Ctx c = make_ctx(g);
     const BitsFront fr{g->F, g->lo, g->hi};
-    const BfsApp app{g->V, cand};
+    const BfsApp app{g->V, cand, g->nfilter ? 1u : 0u};
     launch_expand(g, s, c, fr, app);
-    CU(cudaMemsetAsync(g->hub_ctr, 0, 8, s));
+    CU(cudaMemsetAsync(g->hub_ctr, 0, 16, s));
     return GCGT_OK;
 }
 
@@ -1081,7 +1226,7 @@ extern "C" gcgt_status gcgt_dist_bfs_commit(gcgt_graph* g, uint32_t level, const
     CU(cudaSetDevice(g->device));
     cudaStream_t s = g->stream;
     const uint64_t w_lo = g->lo / 32, nlw = (g->hi + 31) / 32 - w_lo;
-    unsigned long long* cnt = g->st;  // scratch counter (the dist steps keep no stats)
+    unsigned long long* cnt = g->aux + 2;  // scratch counter (new owned vertices; not returned)
     *reinterpret_cast<int32_t*>(g->h_misc()) = (int32_t)level;
     CU(cudaMemcpyAsync(g->src_dev, g->h_misc(), 4, cudaMemcpyHostToDevice, s));
     if (nlw)
@@ -1097,7 +1242,7 @@ extern "C" gcgt_status gcgt_dist_bfs_absorb(gcgt_graph* g, const uint32_t* front
     CU(cudaSetDevice(g->device));
     cudaStream_t s = g->stream;
     const uint64_t nwf = (g->n + 31) / 32;
-    unsigned long long* cnt = g->st + 1;
+    unsigned long long* cnt = g->aux + 1;
     CU(cudaMemsetAsync(cnt, 0, 8, s));
     dist_absorb<<<flat_grid(g, nwf), kBlock, 0, s>>>(frontier, g->F, g->V, nwf, cnt);
     CU(cudaMemcpyAsync(g->h_st() + 1, cnt, 8, cudaMemcpyDeviceToHost, s));
@@ -1122,14 +1267,14 @@ extern "C" gcgt_status gcgt_dist_cc_hook(gcgt_graph* g, uint32_t* parent, uint32
     if (!g || !parent || !hooks || (cap && !pairs)) return fail(GCGT_EINVAL, "null argument");
     CU(cudaSetDevice(g->device));
     cudaStream_t s = g->stream;
-    uint32_t* hc = reinterpret_cast<uint32_t*>(g->st);
+    uint32_t* hc = reinterpret_cast<uint32_t*>(g->aux);  // not the stats block: the engine adds its counts there
     CU(cudaMemsetAsync(hc, 0, 4, s));
-    CU(cudaMemsetAsync(g->hub_ctr, 0, 8, s));
+    CU(cudaMemsetAsync(g->hub_ctr, 0, 16, s));
     const Ctx c = make_ctx(g);
     const DenseFront fr{g->lo, g->hi};
     const CcDistApp app{parent, hc, pairs, (uint32_t)std::min<uint64_t>(cap, 0xFFFFFFFFull), 0};
     launch_expand(g, s, c, fr, app);
-    CU(cudaMemsetAsync(g->hub_ctr, 0, 8, s));
+    CU(cudaMemsetAsync(g->hub_ctr, 0, 16, s));
     CU(cudaMemcpyAsync(g->h_misc(), hc, 4, cudaMemcpyDeviceToHost, s));
     CU(cudaStreamSynchronize(s));
     CU(cudaGetLastError());

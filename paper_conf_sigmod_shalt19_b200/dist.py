@@ -82,7 +82,7 @@ def word_range(lo, hi):
 class DistBFS:
     """Partitioned BFS / CC driver.  ``ops`` provides the per-rank steps (GraphOps, or a test double)."""
 
-    def __init__(self, ops, group=None, exchange_on_host=False, alpha=4, beta=128, sparse_cc_frac=0.02):
+    def __init__(self, ops, group=None, exchange_on_host=False, alpha=4.0, beta=128, sparse_cc_frac=0.02):
         self.ops = ops
         self.group = group
         self.P = dist.get_world_size(group)
@@ -90,7 +90,7 @@ class DistBFS:
         self.host = exchange_on_host
         self.n = ops.n
         self.nwf = (self.n + 31) // 32
-        self.alpha, self.beta = alpha, beta
+        self.alpha10, self.beta = int(round(alpha * 10)), beta
         self.sparse_cap = max(64, int(self.n * sparse_cc_frac))  # hook pairs per rank below which CC goes sparse
         lo, hi = ops.range()
         # every rank's owned range (gathered once)
@@ -141,7 +141,7 @@ class DistBFS:
         if not can_bu or nf == 0:
             return 0
         nu = self.n - visited
-        if dirn == 0 and nf * self.alpha > nu and nf > prev:
+        if dirn == 0 and nf * self.alpha10 > nu * 10 and nf > prev:
             return 1
         if dirn == 1 and nf * self.beta < self.n and nf < prev:
             return 0

@@ -125,11 +125,12 @@ def test_hub_and_long_intervals():
                           np.full(tail.size, 3), [hub[5]] * 3]).astype(np.int64)
     dst = np.concatenate([hub, itv, long_run, tail, [1, 2, 3]]).astype(np.int64)
     ro, co = csr_from_edges(n, src, dst)
-    for ml, sl, k in [(4, 32, 3), (4, 8, 1), (0, 0, 3), (2, 128, 2)]:
+    for ml, sl, k in [(4, 32, 3), (4, 8, 1), (0, 0, 3), (2, 128, 2), (4, 0, 1)]:
         g = load(ro, co, ml, sl, k)
         for s in (0, 1, 2, 3):
             assert np.array_equal(g.bfs(s), O.bfs(ro, co, s)), (ml, sl, k, s)
         assert np.array_equal(g.cc(), O.cc(ro, co))
+        check_bc(g.bc([0, 1]), O.bc(ro, co, [0, 1]))
 
 
 def test_device_outputs_torch():
@@ -201,7 +202,9 @@ def test_warp_decoder_random_streams(k):
 # ---------------------------------------------------------------------------------------------------------------------
 @pytest.mark.parametrize("tune", ["", "bu_alpha=100000,bu_beta=1", "bu_alpha=100000,bu_beta=100000", "graph=0",
                                   "graph=0,bu_alpha=100000,bu_beta=1", "graph=0,chunk=2", "graph=0,chunk=16",
-                                  "hub_segs=1", "compact=0", "dir_bits=1", "dir_opt=0", "bu_alpha=1"])
+                                  "hub_segs=1", "compact=0", "dir_bits=1", "dir_opt=0", "bu_alpha=1", "td_stage=0",
+                                  "td_pool=1", "td_pool=1,td_stage=0", "bu_hub_segs=1", "bu_hub_segs=100000", "ck_c=2",
+                                  "ck_c=0", "bu_grow=0,bu_alpha=25", "hub_stage=0"])
 @pytest.mark.parametrize("name", ["c1", "rmat_s", "web_s", "social_s"])
 def test_bfs_direction_optimizing(name, tune, monkeypatch):
     """Symmetric graphs use the out-CGR as in-CGR; directed ones the encoded transpose.  The tunes force
@@ -217,6 +220,19 @@ def test_bfs_direction_optimizing(name, tune, monkeypatch):
         g = G.load(cgr, in_cgr=G.encode_transpose(ro, co, *p))
     for r in [0] + synth.pick_roots(ro, 3):
         assert np.array_equal(g.bfs(r), O.bfs(ro, co, r)), (name, tune, r)
+
+
+@pytest.mark.parametrize("tune", ["td_pool=1", "td_stage=0", "hub_segs=1", "ck_c=2", "ck_c=0"])
+@pytest.mark.parametrize("name", ["web_s", "social_s", "rmat_s"])
+def test_cc_bc_engine_knobs(name, tune, monkeypatch):
+    """CC hooking and BC run through the same expansion engine: every engine knob keeps them exact."""
+    monkeypatch.setenv("GCGT_TUNE", tune)
+    cfg = synth.CONFIGS[name]
+    ro, co = cfg.make()
+    g = load(ro, co, cfg.min_interval_len, cfg.residual_segment_len, cfg.zeta_k)
+    assert np.array_equal(g.cc(), O.cc(ro, co))
+    src = synth.bc_sources(ro, 2)
+    check_bc(g.bc(src), O.bc(ro, co, src))
 
 
 @pytest.mark.parametrize("ml,sl,k", [(4, 32, 3), (0, 0, 1), (2, 8, 5)])
