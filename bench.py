@@ -150,7 +150,7 @@ def ncu_traffic(cfg_name, levels_per_bfs):
         d = json.load(f)
     tot, launches = 0.0, 0
     for k, v in d.items():
-        if any(x in k for x in ("expand_kernel", "hub_kernel", "bu_kernel")):
+        if any(x in k for x in ("expand_kernel", "hub_kernel", "bu_kernel", "bu_flat_kernel")):
             tot += v["dram_bytes"]
             launches = max(launches, v["launches"])
     if not launches:
@@ -495,32 +495,26 @@ def measure_e2e(G, cgr, incgr, roots, edges_of_root, cfg, n, nbits, dev, local, 
     """Same metric through the public API with HOST buffers: per step gcgt_load (H2D of the CGR bytes and bit
     offsets from pinned host memory) + gcgt_bfs into a pinned host levels array (D2H) + gcgt_unload."""
     import torch
-    cudart = torch.cuda.cudart()
-    b, nb, offs, _, _ = cgr.view()
-    # re-wrap into a CGR whose arrays we can pin: the library copies into its own (pageable) vectors, so pin those
     import ctypes as C
     L = G.lib()
-    bp, op = C.c_void_p(), C.c_void_p()
-    L.gcgt_cgr_view(cgr.handle, C.byref(bp), None, C.byref(op), None, None)
-    nbytes_words = ((nbits + 63) // 64 + 2) * 8
-    reg = [(bp.value, nbytes_words), (op.value, (n + 1) * 8)]
     # H2D per load: the CGR words plus the compact bit offsets (u32 per vertex + a u64 anchor per 256 vertices)
+    nbytes_words = ((nbits + 63) // 64 + 2) * 8
     offs_h2d = (n + 1) * 4 + ((n // 256) + 1) * 8
     h2d = nbytes_words + offs_h2d
     if incgr is not None:
-        ib, io = C.c_void_p(), C.c_void_p()
         inb = C.c_uint64()
-        L.gcgt_cgr_view(incgr.handle, C.byref(ib), C.byref(inb), C.byref(io), None, None)
-        inwords = ((inb.value + 63) // 64 + 2) * 8
-        reg += [(ib.value, inwords), (io.value, (n + 1) * 8)]
-        h2d += inwords + offs_h2d
-    codes = []
-    for ptr, size in reg:
-        codes.append(int(cudart.cudaHostRegister(ptr, size, 0)))
+        L.gcgt_cgr_view(incgr.handle, None, C.byref(inb), None, None, None)
+        h2d += ((inb.value + 63) // 64 + 2) * 8 + offs_h2d
+    # the public API for repeated loads: derived load tables built once and the host arrays page-locked
+    t_pin = time.perf_counter()
+    cgr.pin()
+    if incgr is not None:
+        incgr.pin()
+    t_pin = time.perf_counter() - t_pin
     levels = torch.empty(n, dtype=torch.int32).pin_memory()
     tot_e, tot_t = 0.0, 0.0
     split = {"load_ms": [], "bfs_ms": [], "unload_ms": []}
-    try:
+    if True:
         # one untimed warm-up cycle: the first load grows the device memory pool (kept afterwards, as in a service)
         g = G.load(cgr, device=local, stream="torch", in_cgr=incgr, symmetric=cfg.symmetric)
         g.bfs(roots[0], out=levels)
@@ -541,10 +535,6 @@ def measure_e2e(G, cgr, incgr, roots, edges_of_root, cfg, n, nbits, dev, local, 
             split["load_ms"].append(round((t1 - t0) * 1e3, 1))
             split["bfs_ms"].append(round((t2 - t1) * 1e3, 1))
             split["unload_ms"].append(round((t3 - t2) * 1e3, 1))
-    finally:
-        for (ptr, _), c in zip(reg, codes):
-            if c == 0:
-                cudart.cudaHostUnregister(ptr)
     # query-service variant: the graph stays resident (loaded once, like model weights); per step the source goes
     # H2D and the whole levels array comes back D2H into pinned host memory
     g = G.load(cgr, device=local, stream="torch", in_cgr=incgr, symmetric=cfg.symmetric)
@@ -559,9 +549,9 @@ def measure_e2e(G, cgr, incgr, roots, edges_of_root, cfg, n, nbits, dev, local, 
         qe += edges_of_root[r]
     g.unload()
     return {"value": tot_e / tot_t / 1e9, "unit": "GTEPS", "h2d_bytes_per_step": int(h2d),
-            "d2h_bytes_per_step": int(4 * n), "host_register_status": codes, "per_step": split,
-            "note": "per step (after 1 untimed warm-up cycle): gcgt_load (CGR + in-CGR + bit offsets H2D from pinned "
-                    "host memory, pool allocation) + "
+            "d2h_bytes_per_step": int(4 * n), "pin_s": round(t_pin, 2), "per_step": split,
+            "note": "per step (after gcgt_cgr_pin and 1 untimed warm-up cycle): gcgt_load (CGR + in-CGR + bit "
+                    "offsets + checkpoint table H2D from page-locked host memory, pool allocation) + "
                     "gcgt_bfs with a pinned host levels array + gcgt_unload; host wall clock",
             "resident_graph": {"value": qe / qt / 1e9, "unit": "GTEPS", "h2d_bytes_per_step": 4,
                                "d2h_bytes_per_step": int(4 * n),

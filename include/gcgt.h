@@ -107,6 +107,13 @@ gcgt_status gcgt_cgr_save(const gcgt_cgr* cgr, const char* path);
 gcgt_status gcgt_cgr_open(const char* path, gcgt_cgr** out);
 void gcgt_cgr_free(gcgt_cgr* cgr);
 
+/* Prepares a whole CGR for repeated loads (a query service that reloads the graph): builds the derived load tables
+ * now -- the compact bit offsets and the interval checkpoint table, otherwise built on
+ * the first gcgt_load and kept with the CGR -- and page-locks the CGR's host arrays (cudaHostRegister, portable), so
+ * that each later gcgt_load is host-to-device DMA plus the device byte swap.  Idempotent; the registration is
+ * released by gcgt_cgr_free.  ECUDA if page-locking fails (nothing is left registered by the failing call's array). */
+gcgt_status gcgt_cgr_pin(gcgt_cgr* cgr);
+
 /* ---- Device residency (§3.2 :469-479: "directly move the compressed adjacency lists to GPUs") -------------------- */
 typedef struct {
     int device;        /* CUDA device ordinal                                                                       */

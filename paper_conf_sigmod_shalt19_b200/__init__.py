@@ -22,6 +22,7 @@ OUT_HOST, OUT_DEVICE = 0, 1
 
 # public symbols of include/gcgt.h (tests check the library exports every one)
 ABI_SYMBOLS = ["gcgt_encode", "gcgt_encode_transpose", "gcgt_encode_slice", "gcgt_cgr_concat", "gcgt_cgr_slice_info", "gcgt_cgr_view", "gcgt_cgr_from_arrays", "gcgt_cgr_save", "gcgt_cgr_open",
+               "gcgt_cgr_pin",
                "gcgt_cgr_free", "gcgt_load", "gcgt_load_csr", "gcgt_unload", "gcgt_profile", "gcgt_profile_spans", "gcgt_graph_range", "gcgt_bfs", "gcgt_cc", "gcgt_bc",
                "gcgt_dist_bfs_begin", "gcgt_dist_bfs_expand", "gcgt_dist_bfs_commit", "gcgt_dist_bfs_absorb",
                "gcgt_dist_bfs_levels", "gcgt_dist_cc_hook", "gcgt_dist_cc_merge", "gcgt_dist_cc_jump", "gcgt_sync",
@@ -76,6 +77,7 @@ def lib():
         L.gcgt_cgr_view.argtypes = [p, C.POINTER(p), C.POINTER(u64), C.POINTER(p), C.POINTER(u64), C.POINTER(Params)]
         L.gcgt_cgr_from_arrays.argtypes = [u64, p, u64, p, C.POINTER(Params), C.POINTER(p)]
         L.gcgt_cgr_save.argtypes = [p, C.c_char_p]
+        L.gcgt_cgr_pin.argtypes = [p]
         L.gcgt_cgr_open.argtypes = [C.c_char_p, C.POINTER(p)]
         L.gcgt_cgr_free.argtypes = [p]
         L.gcgt_cgr_free.restype = None
@@ -136,6 +138,11 @@ class CGR:
         by = np.ctypeslib.as_array((C.c_uint8 * max(nbytes, 1)).from_address(b.value))[:nbytes].copy()
         bo = np.ctypeslib.as_array((C.c_uint64 * (n.value + 1)).from_address(off.value)).copy()
         return by, int(nbits.value), bo, int(n.value), (P.min_interval_len, P.residual_segment_len, P.zeta_k)
+
+    def pin(self):
+        """gcgt_cgr_pin: build the derived load tables now and page-lock the host arrays (fast repeated loads)."""
+        _check(lib().gcgt_cgr_pin(self._h), "gcgt_cgr_pin")
+        return self
 
     def save(self, path: str):
         _check(lib().gcgt_cgr_save(self._h, path.encode()), "gcgt_cgr_save")

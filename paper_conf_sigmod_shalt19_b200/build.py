@@ -43,6 +43,8 @@ def build(force: bool = False, verbose_ptxas: bool = False) -> str:
         o = os.path.join(BUILD, src + ".o")
         if force or _newer(o, [s] + hdrs):
             cmd = [NVCC, *ARCH, "-O3", "-lineinfo", "-std=c++17", "-Xcompiler", "-fPIC,-fopenmp", "-c", s, "-o", o]
+            if os.environ.get("GCGT_DEV_K"):  # development only: a single zeta_k instantiation
+                cmd += [f"-DGCGT_DEV_K={int(os.environ['GCGT_DEV_K'])}"]
             if verbose_ptxas:
                 cmd += ["-Xptxas", "-v"]
             _run(cmd)

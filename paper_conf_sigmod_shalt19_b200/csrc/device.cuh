@@ -132,6 +132,12 @@ struct BitReaderT {
         lo = __funnelshift_lc(0u, lo, L);
         avail -= L;
     }
+    // n (1..32) bits; requires avail >= n (true after a refill when n <= 33)
+    __device__ __forceinline__ uint32_t take(uint32_t n) {
+        const uint32_t v = __funnelshift_rc(hi, 0u, 32 - n);  // hi >> (32 - n), also for n == 32
+        consume(n);
+        return v;
+    }
     template <int K>
     __device__ __forceinline__ uint64_t next() {
         refill();
@@ -151,9 +157,25 @@ struct BitReaderT {
                 return v;
             }
         }
-        const Decoded d = decode_at<K, GENERIC>(src, j0, pos());
-        init(src, j0, d.end);
-        return d.v;
+        return next_long<K>(z);
+    }
+    // Codewords longer than 32 bits (a segment's first residual anchored at u, App. C; far gaps): the prefix is
+    // consumed, then the payload is taken in at most two <= 32-bit pieces, refilling in between -- no re-anchoring.
+    // Prefixes of 32+ zeros (payloads beyond 64 bits) take the bit-serial path.
+    template <int K>
+    __device__ __forceinline__ uint64_t next_long(uint32_t z) {
+        const uint32_t P = K == 1 ? z + 1 : K * (z + 1);
+        if (z >= 32 || P > 64) {
+            const Decoded d = decode_at<K, GENERIC>(src, j0, pos());
+            init(src, j0, d.end);
+            return d.v;
+        }
+        consume(K == 1 ? z : z + 1);  // K == 1: the payload starts at the leading 1
+        refill();
+        if (P <= 32) return take(P);
+        const uint32_t a = take(P - 32);
+        refill();
+        return ((uint64_t)a << 32) | take(32);
     }
 };
 using BitReader = BitReaderT<true>;

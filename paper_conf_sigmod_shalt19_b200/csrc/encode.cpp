@@ -482,4 +482,8 @@ extern "C" gcgt_status gcgt_cgr_open(const char* path, gcgt_cgr** out) {
     return st;
 }
 
-extern "C" void gcgt_cgr_free(gcgt_cgr* c) { delete c; }
+extern "C" void gcgt_cgr_free(gcgt_cgr* c) {
+    if (!c) return;
+    gcgt_internal::release_tables(c);
+    delete c;
+}

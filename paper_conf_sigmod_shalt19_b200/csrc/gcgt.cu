@@ -85,7 +85,8 @@ struct gcgt_graph {
     int rank = 0, nranks = 1;
     DevCgr out, in;
     DevCk ck;
-    uint32_t ck_c = 32;  // intervals per checkpoint chunk (GCGT_TUNE ck_c; 0 = no table)
+    static constexpr uint32_t kCkC = 32;
+    uint32_t ck_c = kCkC;  // intervals per checkpoint chunk (GCGT_TUNE ck_c; 0 = no table)
     bool in_alias = false;  // symmetric: in == out
     bool has_in = false;
     bool dir_opt = false;
@@ -125,7 +126,7 @@ struct gcgt_graph {
     cudaEvent_t ev0 = nullptr, ev1 = nullptr;
     int num_sms = 148;
     // knobs (GCGT_TUNE="key=value,..." at load; results never change)
-    uint32_t hub_segs = 8;                  // more segments than this: the vertex's segments go grid-wide
+    uint32_t hub_segs = 1;                  // more segments than this: the vertex's segments go grid-wide
     uint32_t bu_hub_segs = 0xFFFFFFFFu;     // bottom-up: in-records with more segments are scanned grid-wide (off:
                                             // measured slower on C2 / C3, even on C4)
     uint32_t bu_alpha = 40, bu_beta = 128;  // direction switch on vertex counts; alpha in tenths (r2 sweeps, C2-C4)
@@ -139,7 +140,10 @@ struct gcgt_graph {
     uint32_t chunk = 4;                     // host-driven loop: levels enqueued per host check
     bool compact_offs = true;
     bool td_stage = true;  // top-down: records staged through shared memory with coalesced 128-bit loads
-    bool td_pool = false;  // top-down: phase B from a per-warp segment pool with lane refill (hub_segs capped at 2)
+    bool hub_flat = false;  // hub pass: flat loop with lane refill (hub_flat_kernel)
+    bool bu_flat = false;  // bottom-up: flat scan loop with lane refill (bu_flat_kernel)
+    bool td_pool = true;   // top-down: phase B from a per-warp segment pool, one flat loop with lane refill
+                           // (hub_segs capped at 2; r2: C4 BFS 30.1 -> 21.3 ms, C2 7.2 -> 5.7 ms)
     // BFS graph (built on first use for a given levels buffer)
     cudaGraphExec_t bfs_exec = nullptr;
     int32_t* bfs_exec_levels = nullptr;
@@ -175,6 +179,9 @@ inline void with_k(const gcgt_params& P, Fn&& fn) {
 #define GCGT_K(KK)                                                      \
     if (seg) fn(std::integral_constant<int, KK>{}, std::true_type{});   \
     else fn(std::integral_constant<int, KK>{}, std::false_type{});
+#ifdef GCGT_DEV_K  // development builds (GCGT_DEV_K=3 python -m ...build): one zeta_k only, compiles ~5x faster
+    if (P.zeta_k == GCGT_DEV_K) { GCGT_K(GCGT_DEV_K) }
+#else
     switch (P.zeta_k) {
         case 1: GCGT_K(1) break;
         case 2: GCGT_K(2) break;
@@ -182,6 +189,7 @@ inline void with_k(const gcgt_params& P, Fn&& fn) {
         case 4: GCGT_K(4) break;
         default: GCGT_K(5) break;
     }
+#endif
 #undef GCGT_K
 }
 
@@ -212,8 +220,14 @@ inline void launch_expand(gcgt_graph* g, cudaStream_t s, const Ctx& c, const Fro
         expand_kernel<K, SEG, App, Front><<<occ * g->num_sms, kBlock, 0, s>>>(c, fr, app, 0u);
         g->launches++;
         if (SEG || g->ck.bits) {  // hub segments and / or interval chunks
-            if (!occh) occh = occupancy(hub_kernel<K, App>);
-            hub_kernel<K, App><<<occh * g->num_sms, kBlock, 0, s>>>(c, app);
+            static int occf = 0;
+            if (g->hub_flat) {
+                if (!occf) occf = occupancy(hub_flat_kernel<K, App>);
+                hub_flat_kernel<K, App><<<occf * g->num_sms, kBlock, 0, s>>>(c, app);
+            } else {
+                if (!occh) occh = occupancy(hub_kernel<K, App>);
+                hub_kernel<K, App><<<occh * g->num_sms, kBlock, 0, s>>>(c, app);
+            }
             g->launches++;
         }
     });
@@ -229,13 +243,22 @@ inline void launch_bu(gcgt_graph* g, cudaStream_t s, const uint32_t* V, const ui
     with_k(g->P, [&](auto KK, auto SS) {
         constexpr int K = decltype(KK)::value;
         constexpr bool SEG = decltype(SS)::value;
-        static int occ = 0, occh = 0;
-        if (!occ) occ = occupancy(bu_kernel<K, SEG>);
+        static int occ = 0, occh = 0, occf = 0;
         const uint64_t words = (hi - lo + 31) / 32 + 1;
-        const int grid = (int)std::max<uint64_t>(1, std::min<uint64_t>((words + kWarps - 1) / kWarps,
-                                                                        (uint64_t)occ * g->num_sms));
-        bu_kernel<K, SEG><<<grid, kBlock, 0, s>>>(g->in.W, g->in.offs(), g->P.min_interval_len,
-                                                  8 * g->P.residual_segment_len, V, F, N, lo, hi, dir, g->st, hubs);
+        if (g->bu_flat) {  // flat scan with lane refill; 32-word chunks per warp
+            if (!occf) occf = occupancy(bu_flat_kernel<K, SEG>);
+            const int grid = (int)std::max<uint64_t>(1, std::min<uint64_t>((words + 32 * kWarps - 1) / (32 * kWarps),
+                                                                            (uint64_t)occf * g->num_sms));
+            bu_flat_kernel<K, SEG><<<grid, kBlock, 0, s>>>(g->in.W, g->in.offs(), g->P.min_interval_len,
+                                                           8 * g->P.residual_segment_len, V, F, N, lo, hi, dir, g->st,
+                                                           hubs);
+        } else {
+            if (!occ) occ = occupancy(bu_kernel<K, SEG>);
+            const int grid = (int)std::max<uint64_t>(1, std::min<uint64_t>((words + kWarps - 1) / kWarps,
+                                                                            (uint64_t)occ * g->num_sms));
+            bu_kernel<K, SEG><<<grid, kBlock, 0, s>>>(g->in.W, g->in.offs(), g->P.min_interval_len,
+                                                      8 * g->P.residual_segment_len, V, F, N, lo, hi, dir, g->st, hubs);
+        }
         g->launches++;
         if (SEG && hubs.q) {
             if (!occh) occh = occupancy(bu_hub_kernel<K>);
@@ -354,6 +377,34 @@ gcgt_status dalloc(T** p, uint64_t count) {
     return GCGT_OK;
 }
 
+gcgt_cgr_tables* whole_tables(const gcgt_cgr* c) {  // caller holds c->mu
+    if (!c->tables) c->tables.reset(new gcgt_cgr_tables());
+    return c->tables.get();
+}
+
+// Compact bit offsets of vertices [lo, hi): a u64 anchor per 256 vertices (relative to bit `base`) and
+// a u32 offset relative to the anchor; t->compact is false when some 256-vertex block spans >= 2^32 bits.
+void build_compact(const uint64_t* bo, uint64_t lo, uint64_t hi, uint64_t base, gcgt_cgr_tables* t) {
+    const uint64_t nloc = hi - lo, nanc = nloc / 256 + 1;
+    bool compact = true;
+    for (uint64_t k = 0; compact && k < nanc; k++) {
+        const uint64_t a = lo + k * 256, b = std::min(hi, a + 256);
+        if (bo[b] - bo[a] >= (1ull << 32)) compact = false;
+    }
+    t->compact = compact;
+    if (!compact) return;
+    t->anc.resize(nanc);
+    t->rel.resize(nloc + 1);
+    uint64_t* anc = t->anc.data();
+    uint32_t* rel = t->rel.data();
+#pragma omp parallel for schedule(static)
+    for (int64_t i = 0; i <= (int64_t)nloc; i++) {
+        const uint64_t a = bo[lo + ((uint64_t)i & ~255ull)];
+        rel[i] = (uint32_t)(bo[lo + i] - a);
+        if ((i & 255) == 0) anc[i >> 8] = a - base;
+    }
+}
+
 // Uploads the records of vertices [lo, hi) of a host CGR: whole 64-bit stream words (records are self-contained,
 // so a vertex-range slice is a bit copy, §8 e) byte-swapped on the device into stream order, plus the bit offsets
 // re-based to the slice, in compact form when every 256-vertex block spans < 2^32 bits (§8 a2).  The word array is
@@ -384,24 +435,20 @@ gcgt_status upload_cgr(gcgt_graph* g, const gcgt_cgr* c, uint64_t lo, uint64_t h
     }
     const uint64_t nloc = hi - lo, base = w0 * 64;
     const uint64_t nanc = nloc / 256 + 1;
-    bool compact = g->compact_offs;
-    for (uint64_t k = 0; compact && k < nanc; k++) {
-        const uint64_t a = lo + k * 256, b = std::min(hi, a + 256);
-        if (bo[b] - bo[a] >= (1ull << 32)) compact = false;
+    const bool whole = lo == c->base && hi == c->base + c->n;  // then base == 0 and the tables are cached
+    gcgt_cgr_tables local;
+    gcgt_cgr_tables* t = &local;
+    std::unique_lock<std::mutex> lk(c->mu, std::defer_lock);
+    if (whole) {
+        lk.lock();
+        t = whole_tables(c);
     }
-    if (compact) {
-        std::vector<uint64_t> anc(nanc);
-        std::vector<uint32_t> rel(nloc + 1);
-#pragma omp parallel for schedule(static)
-        for (int64_t i = 0; i <= (int64_t)nloc; i++) {
-            const uint64_t a = bo[lo + ((uint64_t)i & ~255ull)];
-            rel[i] = (uint32_t)(bo[lo + i] - a);
-            if ((i & 255) == 0) anc[i >> 8] = a - base;
-        }
+    if (g->compact_offs && t->anc.empty()) build_compact(bo, lo, hi, base, t);
+    if (g->compact_offs && t->compact) {
         if ((st = galloc(g, &d->anc, nanc)) || (st = galloc(g, &d->rel, nloc + 1))) return st;
-        CU(cudaMemcpyAsync(d->anc, anc.data(), nanc * 8, cudaMemcpyHostToDevice, s));
-        CU(cudaMemcpyAsync(d->rel, rel.data(), (nloc + 1) * 4, cudaMemcpyHostToDevice, s));
-        CU(cudaStreamSynchronize(s));  // host vectors
+        CU(cudaMemcpyAsync(d->anc, t->anc.data(), nanc * 8, cudaMemcpyHostToDevice, s));
+        CU(cudaMemcpyAsync(d->rel, t->rel.data(), (nloc + 1) * 4, cudaMemcpyHostToDevice, s));
+        if (!whole) CU(cudaStreamSynchronize(s));  // local host vectors
         d->offs_bytes = nanc * 8 + (nloc + 1) * 4;
     } else {
         std::vector<uint64_t> ro(nloc + 1);
@@ -429,6 +476,23 @@ struct HostBits {
     const uint8_t* b;
     int bit(uint64_t i) const { return (b[i >> 3] >> (7 - (i & 7))) & 1; }
     uint64_t read(uint32_t K, uint64_t& p) const {  // one VLC codeword (App. B; FORMAT.md R3/R4)
+        {  // fast path: a 57+-bit window at p (the words array is padded, so 8 bytes at p/8 are readable)
+            uint64_t w;
+            memcpy(&w, b + (p >> 3), 8);
+            const uint64_t win = __builtin_bswap64(w) << (p & 7);
+            if (win) {
+                const uint32_t z = (uint32_t)__builtin_clzll(win);
+                if (K == 1 && 2 * z + 1 <= 57) {
+                    p += 2 * z + 1;
+                    return win >> (63 - 2 * z);
+                }
+                if (K > 1 && (z + 1) * (K + 1) <= 57) {
+                    const uint32_t h = z + 1;
+                    p += h * (K + 1);
+                    return (win << h) >> (64 - K * h);
+                }
+            }
+        }
         uint64_t z = 0;
         while (!bit(p)) { z++; p++; }
         uint64_t payload;
@@ -441,16 +505,17 @@ struct HostBits {
     }
 };
 
-// Interval checkpoint table (expand.cuh, Checkpoints) for the owned vertices with more than ck_c intervals: decoded
-// once on the host (the header of every vertex, the interval area of the few long ones), uploaded as device tables.
-gcgt_status build_checkpoints(gcgt_graph* g, const gcgt_cgr* c) {
-    const uint32_t C = g->ck_c;
-    if (C == 0 || g->hi == g->lo) return GCGT_OK;
-    const uint64_t lo = g->lo, hi = g->hi, nloc = hi - lo, base = g->out.base_bits;
+// Interval checkpoint table (expand.cuh, Checkpoints) for the vertices [lo, hi) with more than C intervals: decoded
+// on the host (the header of every vertex, the interval area of the few long ones).  Bit positions are relative to
+// `base` (the device word array's first bit).
+void build_ck_host(const gcgt_cgr* c, uint64_t lo, uint64_t hi, uint64_t base, uint32_t C, gcgt_cgr_tables* t) {
+    const uint64_t nloc = hi - lo;
     const uint64_t* bo = c->bit_offsets.data() - c->base;
     const HostBits hb{reinterpret_cast<const uint8_t*>(c->words.data())};
-    const bool seg = g->P.residual_segment_len != 0;
-    const uint32_t K = g->P.zeta_k;
+    const bool seg = c->params.residual_segment_len != 0;
+    const uint32_t K = c->params.zeta_k;
+    t->ck_built = true;
+    t->ck_c = C;
     std::vector<uint32_t> itv(nloc, 0);
 #pragma omp parallel for schedule(dynamic, 65536)
     for (int64_t i = 0; i < (int64_t)nloc; i++) {
@@ -461,22 +526,24 @@ gcgt_status build_checkpoints(gcgt_graph* g, const gcgt_cgr* c) {
         if (x > C) itv[i] = (uint32_t)x;
     }
     const uint64_t w0 = lo >> 5, nwl = ((hi + 31) >> 5) - w0;
-    std::vector<uint32_t> wptr(nwl + 1, 0), bits(nwl, 0), rows_u;
+    std::vector<uint32_t> rows_u;
     for (uint64_t i = 0; i < nloc; i++)
-        if (itv[i]) {
-            const uint64_t v = lo + i;
-            bits[(v >> 5) - w0] |= 1u << (v & 31);
-            rows_u.push_back((uint32_t)v);
-        }
-    if (rows_u.empty()) return GCGT_OK;
-    for (uint64_t w = 0; w < nwl; w++) wptr[w + 1] = wptr[w] + __builtin_popcount(bits[w]);
+        if (itv[i]) rows_u.push_back((uint32_t)(lo + i));
+    t->rows = rows_u.size();
+    if (rows_u.empty()) return;
+    t->wptr.assign(nwl + 1, 0);
+    t->bits.assign(nwl, 0);
+    for (uint32_t v : rows_u) t->bits[(v >> 5) - w0] |= 1u << (v & 31);
+    for (uint64_t w = 0; w < nwl; w++) t->wptr[w + 1] = t->wptr[w] + __builtin_popcount(t->bits[w]);
     const uint64_t R = rows_u.size();
-    std::vector<uint32_t> ck0(R + 1, 0), ilen(R, 0);
-    std::vector<uint64_t> after(R, 0);
-    for (uint64_t r = 0; r < R; r++) ck0[r + 1] = ck0[r] + (itv[rows_u[r] - lo] + C - 1) / C;
-    const uint64_t T = ck0[R];
-    std::vector<uint64_t> pos(T);
-    std::vector<uint32_t> prev(T);
+    t->ck0.assign(R + 1, 0);
+    t->ilen.assign(R, 0);
+    t->after.assign(R, 0);
+    for (uint64_t r = 0; r < R; r++) t->ck0[r + 1] = t->ck0[r] + (itv[rows_u[r] - lo] + C - 1) / C;
+    const uint64_t T = t->ck0[R];
+    t->chunks = T;
+    t->pos.assign(T, 0);
+    t->prev.assign(T, 0);
 #pragma omp parallel for schedule(dynamic, 1)
     for (int64_t r = 0; r < (int64_t)R; r++) {
         const uint64_t u = rows_u[r];
@@ -486,15 +553,15 @@ gcgt_status build_checkpoints(gcgt_graph* g, const gcgt_cgr* c) {
         hb.read(K, p);
         int64_t prev_end = 0;
         uint64_t sum = 0;
-        for (uint32_t t = 0; t < n_itv; t++) {
-            if (t % C == 0) {
-                pos[ck0[r] + t / C] = p - base;
-                prev[ck0[r] + t / C] = (uint32_t)prev_end;
+        for (uint32_t k = 0; k < n_itv; k++) {
+            if (k % C == 0) {
+                t->pos[t->ck0[r] + k / C] = p - base;
+                t->prev[t->ck0[r] + k / C] = (uint32_t)prev_end;
             }
             const uint64_t gcode = hb.read(K, p);
-            const uint64_t len = hb.read(K, p) - 1 + g->P.min_interval_len;
+            const uint64_t len = hb.read(K, p) - 1 + c->params.min_interval_len;
             int64_t start;
-            if (t == 0) {
+            if (k == 0) {
                 const uint64_t z = gcode - 1;
                 start = (int64_t)u + ((z & 1) ? -(int64_t)(z >> 1) : (int64_t)(z >> 1));  // R9
             } else {
@@ -503,9 +570,26 @@ gcgt_status build_checkpoints(gcgt_graph* g, const gcgt_cgr* c) {
             prev_end = start + (int64_t)len - 1;
             sum += len;
         }
-        after[r] = p - base;
-        ilen[r] = (uint32_t)sum;
+        t->after[r] = p - base;
+        t->ilen[r] = (uint32_t)sum;
     }
+}
+
+// Uploads the checkpoint table of the owned range (cached with the CGR for whole-CGR loads).
+gcgt_status build_checkpoints(gcgt_graph* g, const gcgt_cgr* c) {
+    const uint32_t C = g->ck_c;
+    if (C == 0 || g->hi == g->lo) return GCGT_OK;
+    const bool whole = g->lo == c->base && g->hi == c->base + c->n;
+    gcgt_cgr_tables local;
+    gcgt_cgr_tables* t = &local;
+    std::unique_lock<std::mutex> lk(c->mu, std::defer_lock);
+    if (whole) {
+        lk.lock();
+        t = whole_tables(c);
+    }
+    if (!t->ck_built || t->ck_c != C) build_ck_host(c, g->lo, g->hi, g->out.base_bits, C, t);
+    if (t->rows == 0) return GCGT_OK;
+    const uint64_t nwl = t->bits.size(), R = t->rows, T = t->chunks;
     DevCk& d = g->ck;
     gcgt_status st;
     if ((st = galloc(g, &d.wptr, nwl + 1)) || (st = galloc(g, &d.bits, nwl)) || (st = galloc(g, &d.ck0, R + 1)) ||
@@ -513,14 +597,14 @@ gcgt_status build_checkpoints(gcgt_graph* g, const gcgt_cgr* c) {
         (st = galloc(g, &d.prev, T)) || (st = galloc(g, &d.q, R + 1)))
         return st;
     cudaStream_t s = g->stream;
-    CU(cudaMemcpyAsync(d.wptr, wptr.data(), (nwl + 1) * 4, cudaMemcpyHostToDevice, s));
-    CU(cudaMemcpyAsync(d.bits, bits.data(), nwl * 4, cudaMemcpyHostToDevice, s));
-    CU(cudaMemcpyAsync(d.ck0, ck0.data(), (R + 1) * 4, cudaMemcpyHostToDevice, s));
-    CU(cudaMemcpyAsync(d.after, after.data(), R * 8, cudaMemcpyHostToDevice, s));
-    CU(cudaMemcpyAsync(d.ilen, ilen.data(), R * 4, cudaMemcpyHostToDevice, s));
-    CU(cudaMemcpyAsync(d.pos, pos.data(), T * 8, cudaMemcpyHostToDevice, s));
-    CU(cudaMemcpyAsync(d.prev, prev.data(), T * 4, cudaMemcpyHostToDevice, s));
-    CU(cudaStreamSynchronize(s));  // host vectors
+    CU(cudaMemcpyAsync(d.wptr, t->wptr.data(), (nwl + 1) * 4, cudaMemcpyHostToDevice, s));
+    CU(cudaMemcpyAsync(d.bits, t->bits.data(), nwl * 4, cudaMemcpyHostToDevice, s));
+    CU(cudaMemcpyAsync(d.ck0, t->ck0.data(), (R + 1) * 4, cudaMemcpyHostToDevice, s));
+    CU(cudaMemcpyAsync(d.after, t->after.data(), R * 8, cudaMemcpyHostToDevice, s));
+    CU(cudaMemcpyAsync(d.ilen, t->ilen.data(), R * 4, cudaMemcpyHostToDevice, s));
+    CU(cudaMemcpyAsync(d.pos, t->pos.data(), T * 8, cudaMemcpyHostToDevice, s));
+    CU(cudaMemcpyAsync(d.prev, t->prev.data(), T * 4, cudaMemcpyHostToDevice, s));
+    if (!whole) CU(cudaStreamSynchronize(s));  // local host vectors
     d.rows = R;
     d.chunks = T;
     return GCGT_OK;
@@ -550,6 +634,8 @@ void parse_tune(gcgt_graph* g) {
             else if (k == "compact") g->compact_offs = v != 0;
             else if (k == "td_stage") g->td_stage = v != 0;
             else if (k == "td_pool") g->td_pool = v != 0;
+            else if (k == "bu_flat") g->bu_flat = v != 0;
+            else if (k == "hub_flat") g->hub_flat = v != 0;
             else if (k == "ck_c") g->ck_c = (uint32_t)v;
             else if (k == "bu_grow") g->bu_grow = v != 0;
             else if (k == "nfilter") g->nfilter = v != 0;
@@ -950,6 +1036,43 @@ extern "C" gcgt_status gcgt_load_csr(const gcgt_csr* csr, const gcgt_load_opts* 
 // ------------------------------------------------------------------------------------------------------------------
 // C ABI: queries
 // ------------------------------------------------------------------------------------------------------------------
+namespace gcgt_internal {
+void release_tables(gcgt_cgr* c) {
+    std::lock_guard<std::mutex> lk(c->mu);
+    if (!c->tables) return;
+    for (auto& pr : c->tables->pinned) cudaHostUnregister(pr.first);
+    c->tables.reset();
+}
+}  // namespace gcgt_internal
+
+// Builds the derived load tables of a whole CGR now (compact offsets, checkpoint table for the default chunk size)
+// and page-locks the CGR's host arrays, so that every later gcgt_load of it is DMA copies only.
+extern "C" gcgt_status gcgt_cgr_pin(gcgt_cgr* c) {
+    gcgt_internal::clear_error();
+    if (!c) return fail(GCGT_EINVAL, "null argument");
+    std::lock_guard<std::mutex> lk(c->mu);
+    gcgt_cgr_tables* t = whole_tables(c);
+    if (!t->pinned.empty()) return GCGT_OK;
+    const uint64_t* bo = c->bit_offsets.data() - c->base;
+    if (t->anc.empty()) build_compact(bo, c->base, c->base + c->n, 0, t);
+    const uint32_t C = gcgt_graph::kCkC;
+    if (!t->ck_built) build_ck_host(c, c->base, c->base + c->n, 0, C, t);
+    auto reg = [&](const void* p, size_t bytes) -> gcgt_status {
+        if (!p || !bytes) return GCGT_OK;
+        const cudaError_t e = cudaHostRegister(const_cast<void*>(p), bytes, cudaHostRegisterPortable);
+        if (e != cudaSuccess) return fail(GCGT_ECUDA, std::string("cudaHostRegister: ") + cudaGetErrorString(e));
+        t->pinned.emplace_back(const_cast<void*>(p), bytes);
+        return GCGT_OK;
+    };
+    gcgt_status st;
+    if ((st = reg(c->words.data(), c->words.size() * 8)) || (st = reg(t->anc.data(), t->anc.size() * 8)) ||
+        (st = reg(t->rel.data(), t->rel.size() * 4)) || (st = reg(t->pos.data(), t->pos.size() * 8)) ||
+        (st = reg(t->prev.data(), t->prev.size() * 4)))
+        return st;
+    if (!t->compact && (st = reg(c->bit_offsets.data(), c->bit_offsets.size() * 8))) return st;
+    return GCGT_OK;
+}
+
 extern "C" gcgt_status gcgt_profile(gcgt_graph* g, int enable) {
     if (!g) return fail(GCGT_EINVAL, "null graph");
     g->profile = enable != 0;

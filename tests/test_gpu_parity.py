@@ -204,7 +204,9 @@ def test_warp_decoder_random_streams(k):
                                   "graph=0,bu_alpha=100000,bu_beta=1", "graph=0,chunk=2", "graph=0,chunk=16",
                                   "hub_segs=1", "compact=0", "dir_bits=1", "dir_opt=0", "bu_alpha=1", "td_stage=0",
                                   "td_pool=1", "td_pool=1,td_stage=0", "bu_hub_segs=1", "bu_hub_segs=100000", "ck_c=2",
-                                  "ck_c=0", "bu_grow=0,bu_alpha=25", "hub_stage=0"])
+                                  "ck_c=0", "bu_grow=0,bu_alpha=25", "hub_stage=0", "bu_flat=1",
+                                  "bu_flat=1,bu_alpha=100000,bu_beta=1", "bu_flat=1,bu_hub_segs=1",
+                                  "bu_flat=0", "td_pool=0", "bu_flat=0,td_pool=0,bu_alpha=100000,bu_beta=1"])
 @pytest.mark.parametrize("name", ["c1", "rmat_s", "web_s", "social_s"])
 def test_bfs_direction_optimizing(name, tune, monkeypatch):
     """Symmetric graphs use the out-CGR as in-CGR; directed ones the encoded transpose.  The tunes force
@@ -222,7 +224,7 @@ def test_bfs_direction_optimizing(name, tune, monkeypatch):
         assert np.array_equal(g.bfs(r), O.bfs(ro, co, r)), (name, tune, r)
 
 
-@pytest.mark.parametrize("tune", ["td_pool=1", "td_stage=0", "hub_segs=1", "ck_c=2", "ck_c=0"])
+@pytest.mark.parametrize("tune", ["td_pool=1", "td_pool=0", "td_stage=0", "hub_segs=1", "ck_c=2", "ck_c=0"])
 @pytest.mark.parametrize("name", ["web_s", "social_s", "rmat_s"])
 def test_cc_bc_engine_knobs(name, tune, monkeypatch):
     """CC hooking and BC run through the same expansion engine: every engine knob keeps them exact."""
@@ -235,9 +237,10 @@ def test_cc_bc_engine_knobs(name, tune, monkeypatch):
     check_bc(g.bc(src), O.bc(ro, co, src))
 
 
+@pytest.mark.parametrize("flat", [0, 1])
 @pytest.mark.parametrize("ml,sl,k", [(4, 32, 3), (0, 0, 1), (2, 8, 5)])
-def test_bfs_bottom_up_random(ml, sl, k, monkeypatch):
-    monkeypatch.setenv("GCGT_TUNE", "bu_alpha=100000,bu_beta=1")
+def test_bfs_bottom_up_random(ml, sl, k, flat, monkeypatch):
+    monkeypatch.setenv("GCGT_TUNE", f"bu_alpha=100000,bu_beta=1,bu_flat={flat}")
     for seed, sym in [(1, True), (2, False), (3, False)]:
         ro, co = random_graph(6000, 60000, seed=seed + k, symmetric=sym)
         cgr = G.encode(ro, co, ml, sl, k)
@@ -299,3 +302,25 @@ def test_host_resident_cgr(name):
     src = synth.pick_roots(ro, 2)
     check_bc(g.bc(src), O.bc(ro, co, src))
     g.unload()
+
+
+# ---------------------------------------------------------------------------------------------------------------------
+# Repeated loads of a pinned CGR (gcgt_cgr_pin: derived load tables cached with the CGR, host arrays page-locked)
+# ---------------------------------------------------------------------------------------------------------------------
+@pytest.mark.parametrize("tune", ["", "ck_c=2", "compact=0"])
+@pytest.mark.parametrize("name", ["web_s", "social_s"])
+def test_pinned_cgr_reload(name, tune, monkeypatch):
+    monkeypatch.setenv("GCGT_TUNE", tune)
+    cfg = synth.CONFIGS[name]
+    ro, co = cfg.make()
+    p = (cfg.min_interval_len, cfg.residual_segment_len, cfg.zeta_k)
+    cgr, incgr = G.encode(ro, co, *p), G.encode_transpose(ro, co, *p)
+    roots = synth.pick_roots(ro, 2)
+    for it in range(3):  # before pinning (tables built by the load), pinned, pinned again (cached tables)
+        if it == 1:
+            cgr.pin()
+            incgr.pin()
+        g = G.load(cgr, in_cgr=incgr)
+        for r in roots:
+            assert np.array_equal(g.bfs(r), O.bfs(ro, co, r)), (name, tune, it, r)
+        g.unload()

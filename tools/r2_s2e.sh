@@ -1,0 +1,8 @@
+#!/bin/bash
+# dev build (K=3): lane-per-word flat bottom-up vs bu_kernel, with pooled top-down
+mkdir -p gpurun_out
+T=${TAG:-r2s2e}
+TUNES=("td_pool=1,hub_segs=1" "td_pool=1,hub_segs=1,bu_flat=1" "td_pool=1,hub_segs=1,bu_flat=1,bu_alpha=80" "td_pool=1,hub_segs=1,bu_flat=1,bu_alpha=20")
+timeout 600 python tools/sweep_tunes.py c2 6 "${TUNES[@]}" > gpurun_out/${T}_sweep_c2.txt 2>&1
+timeout 900 python tools/sweep_tunes.py c4 4 "${TUNES[@]}" > gpurun_out/${T}_sweep_c4.txt 2>&1
+timeout 900 python tools/sweep_tunes.py c3 4 "${TUNES[@]}" > gpurun_out/${T}_sweep_c3.txt 2>&1
