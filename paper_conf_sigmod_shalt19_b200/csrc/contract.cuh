@@ -24,7 +24,8 @@ struct LevelState {
     uint32_t q_off, q_len, q_next;  // BC: current level's range in the all-levels queue, next level's length
     uint32_t ntd, nbu;  // levels run top-down / bottom-up (BFS; kernel-launch accounting of the graph path)
     uint32_t pad;
-    unsigned long long mf;  // record bits of the new frontier (dir_bits direction test)
+    unsigned long long mf;  // record bits of the new frontier (dir_bits / dir_edges direction tests)
+    unsigned long long mu;  // in-record bits of the vertices visited so far (dir_edges)
 };
 
 // Direction choice for the next BFS level (Beamer et al.'s heuristic, on vertex counts): switch to bottom-up when
@@ -39,6 +40,8 @@ struct DecideArgs {
     double bits_per_vertex;
     uint32_t alpha_bits10;  // in tenths
     int grow;  // 1: switch to bottom-up only while the frontier grows (Beamer's condition)
+    int use_edges;      // Beamer's edge rule with CGR bits as the work measure: mf * alpha > mu
+    double mu_total;    // in-CGR bits of all vertices (mu = mu_total - bits of the visited ones)
 };
 
 struct CommitArgs {
@@ -57,7 +60,8 @@ struct CommitArgs {
     unsigned long long* hub_ctr2;  // (bottom-up hub queue) reset for the next level
     unsigned long long* cursor;    // the expansion's work cursor [2], reset for the next level
     Offs offs_bits;                // record bits of the new frontier (used when use_mf)
-    int use_mf;
+    Offs offs_in;                  // in-record bits of the newly visited vertices (used when use_mu)
+    int use_mf, use_mu;
     DecideArgs dec;
     int bc;
     int use_cond, use_dcond;
@@ -76,6 +80,10 @@ __device__ __forceinline__ void decide_body(volatile LevelState* ls, const Decid
     uint32_t dir = ls->dir;
     bool to_bu = nf * d.alpha10 > nu * 10;
     if (d.use_bits) to_bu = (double)ls->mf * d.alpha_bits10 > (double)nu * d.bits_per_vertex * 10.0;
+    // edge rule (Beamer et al.: m_f > m_u / alpha) with record bits as edge counts: the top-down cost of the next
+    // level is the out-record bits of the new frontier, the bottom-up cost at most the in-record bits of the
+    // unvisited vertices
+    if (d.use_edges) to_bu = (double)ls->mf * d.alpha_bits10 > (d.mu_total - (double)ls->mu) * 10.0;
     ls->mf = 0;
     if (!d.enabled || nf == 0) dir = 0;
     else if (dir == 0 && to_bu && (nf > prev || !d.grow)) dir = 1;
@@ -94,7 +102,7 @@ __global__ void __launch_bounds__(kBlock) commit_kernel(CommitArgs a) {
     const uint64_t gw = ((uint64_t)blockIdx.x * blockDim.x + threadIdx.x) >> 5;
     const uint64_t nwarps = ((uint64_t)gridDim.x * blockDim.x) >> 5;
     uint32_t nf = 0;
-    uint64_t mf = 0;
+    uint64_t mf = 0, mu = 0;
     uint32_t* qlen = a.bc ? &a.ls->q_next : a.qn_len;
     for (uint64_t base = a.w_lo + gw * 32; base < a.w_hi; base += nwarps * 32) {
         const uint64_t w = base + lane;
@@ -124,6 +132,7 @@ __global__ void __launch_bounds__(kBlock) commit_kernel(CommitArgs a) {
                     const uint64_t v = (base + j) * 32 + lane;
                     a.levels[v] = new_level;
                     if (a.use_mf) mf += a.offs_bits(v + 1) - a.offs_bits(v);  // coalesced offset reads
+                    if (a.use_mu) mu += a.offs_in(v + 1) - a.offs_in(v);
                 }
             }
         }
@@ -133,6 +142,10 @@ __global__ void __launch_bounds__(kBlock) commit_kernel(CommitArgs a) {
     if (a.use_mf) {
         for (int o = 16; o; o >>= 1) mf += __shfl_xor_sync(0xffffffffu, mf, o);
         if (lane == 0 && mf) atomicAdd(&a.ls->mf, (unsigned long long)mf);
+    }
+    if (a.use_mu) {
+        for (int o = 16; o; o >>= 1) mu += __shfl_xor_sync(0xffffffffu, mu, o);
+        if (lane == 0 && mu) atomicAdd(&a.ls->mu, (unsigned long long)mu);
     }
     // the last block out closes the level: direction, counters, level number, loop condition
     __syncthreads();

@@ -135,12 +135,15 @@ struct gcgt_graph {
     bool nfilter = false;                   // BFS filter: also test an L1 read of N before the claim
     bool hub_stage = true;                  // hub pass: segments staged through shared memory
     bool dir_bits = false;
+    bool dir_edges = false;                 // Beamer's edge rule on CGR bits (DecideArgs::use_edges)
+    uint32_t alpha_edges = 140;             // tenths
+    uint64_t in_nbits = 0;                  // bits of the loaded in-records (dir_edges)
     bool dir_opt_knob = true;
     bool use_graph = true;                  // BFS as one CUDA graph (else: chunked host-driven level loop)
     uint32_t chunk = 4;                     // host-driven loop: levels enqueued per host check
     bool compact_offs = true;
     bool td_stage = true;  // top-down: records staged through shared memory with coalesced 128-bit loads
-    bool hub_flat = false;  // hub pass: flat loop with lane refill (hub_flat_kernel)
+    bool hub_flat = true;   // hub pass: flat loop with lane refill (hub_flat_kernel; r2: C4 21.3 -> 21.0 ms)
     bool bu_flat = false;  // bottom-up: flat scan loop with lane refill (bu_flat_kernel)
     bool td_pool = true;   // top-down: phase B from a per-warp segment pool, one flat loop with lane refill
                            // (hub_segs capped at 2; r2: C4 BFS 30.1 -> 21.3 ms, C2 7.2 -> 5.7 ms)
@@ -628,6 +631,8 @@ void parse_tune(gcgt_graph* g) {
             else if (k == "bu_beta") g->bu_beta = (uint32_t)v;
             else if (k == "dir_bits") g->dir_bits = v != 0;
             else if (k == "alpha_bits") g->alpha_bits = (uint32_t)v;
+            else if (k == "dir_edges") g->dir_edges = v != 0;
+            else if (k == "alpha_edges") g->alpha_edges = (uint32_t)v;
             else if (k == "dir_opt") g->dir_opt_knob = v != 0;
             else if (k == "graph") g->use_graph = v != 0;
             else if (k == "chunk") g->chunk = (uint32_t)std::max(2ul, std::min(32ul, v & ~1ul));
@@ -699,7 +704,9 @@ gcgt_status ensure_levels(gcgt_graph* g) {
 
 DecideArgs decide_args(const gcgt_graph* g) {
     return DecideArgs{g->n, g->bu_alpha, g->bu_beta, g->dir_opt ? 1 : 0, g->dir_bits && g->dir_opt ? 1 : 0,
-                      (double)g->nbits / (double)std::max<uint64_t>(1, g->n), g->alpha_bits, g->bu_grow ? 1 : 0};
+                      (double)g->nbits / (double)std::max<uint64_t>(1, g->n), g->dir_edges ? g->alpha_edges
+                                                                                            : g->alpha_bits,
+                      g->bu_grow ? 1 : 0, g->dir_edges && g->dir_opt && !g->is_csr ? 1 : 0, (double)g->in_nbits};
 }
 
 CommitArgs bfs_commit_args(gcgt_graph* g, int parity, int32_t* lv) {
@@ -718,7 +725,9 @@ CommitArgs bfs_commit_args(gcgt_graph* g, int parity, int32_t* lv) {
     a.hub_ctr2 = g->buq_ctr;
     a.cursor = g->cursor;
     a.dec = decide_args(g);
-    a.use_mf = a.dec.use_bits;
+    a.use_mf = a.dec.use_bits || a.dec.use_edges;
+    a.use_mu = a.dec.use_edges;
+    if (a.use_mu) a.offs_in = g->in.offs();
     if (a.use_mf && !g->is_csr) a.offs_bits = g->out.offs();
     if (a.use_mf && g->is_csr) a.offs_bits = Offs{nullptr, nullptr, g->crow, 0};
     return a;
@@ -949,10 +958,12 @@ extern "C" gcgt_status gcgt_load(const gcgt_cgr* c, const gcgt_load_opts* opts, 
     if (o.in_cgr) {
         if ((st = upload_cgr(g.get(), o.in_cgr, g->lo, g->hi, o.host_resident != 0, &g->in))) return st;
         g->has_in = true;
+        g->in_nbits = o.in_cgr->nbits;
     } else if (o.symmetric) {
         g->in = g->out;
         g->in_alias = true;
         g->has_in = true;
+        g->in_nbits = c->nbits;
     }
     g->dir_opt = g->has_in && o.direction_optimizing != 0 && g->dir_opt_knob;
     if ((st = alloc_work(g.get()))) return st;

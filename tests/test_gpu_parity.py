@@ -206,7 +206,8 @@ def test_warp_decoder_random_streams(k):
                                   "td_pool=1", "td_pool=1,td_stage=0", "bu_hub_segs=1", "bu_hub_segs=100000", "ck_c=2",
                                   "ck_c=0", "bu_grow=0,bu_alpha=25", "hub_stage=0", "bu_flat=1",
                                   "bu_flat=1,bu_alpha=100000,bu_beta=1", "bu_flat=1,bu_hub_segs=1",
-                                  "bu_flat=0", "td_pool=0", "bu_flat=0,td_pool=0,bu_alpha=100000,bu_beta=1"])
+                                  "bu_flat=0", "td_pool=0", "bu_flat=0,td_pool=0,bu_alpha=100000,bu_beta=1", "hub_flat=0",
+                                  "dir_edges=1", "dir_edges=1,alpha_edges=10", "dir_edges=1,alpha_edges=1000"])
 @pytest.mark.parametrize("name", ["c1", "rmat_s", "web_s", "social_s"])
 def test_bfs_direction_optimizing(name, tune, monkeypatch):
     """Symmetric graphs use the out-CGR as in-CGR; directed ones the encoded transpose.  The tunes force
@@ -224,7 +225,8 @@ def test_bfs_direction_optimizing(name, tune, monkeypatch):
         assert np.array_equal(g.bfs(r), O.bfs(ro, co, r)), (name, tune, r)
 
 
-@pytest.mark.parametrize("tune", ["td_pool=1", "td_pool=0", "td_stage=0", "hub_segs=1", "ck_c=2", "ck_c=0"])
+@pytest.mark.parametrize("tune", ["td_pool=1", "td_pool=0", "td_stage=0", "hub_segs=1", "ck_c=2", "ck_c=0", "hub_flat=0",
+                                  "td_pool=0,hub_segs=8"])
 @pytest.mark.parametrize("name", ["web_s", "social_s", "rmat_s"])
 def test_cc_bc_engine_knobs(name, tune, monkeypatch):
     """CC hooking and BC run through the same expansion engine: every engine knob keeps them exact."""
