@@ -150,7 +150,7 @@ def ncu_traffic(cfg_name, levels_per_bfs):
         d = json.load(f)
     tot, launches = 0.0, 0
     for k, v in d.items():
-        if any(x in k for x in ("expand_kernel", "hub_kernel", "bu_kernel", "bu_flat_kernel")):
+        if any(x in k for x in ("expand_kernel", "hub_kernel", "bu_kernel")):
             tot += v["dram_bytes"]
             launches = max(launches, v["launches"])
     if not launches:

@@ -42,6 +42,7 @@ struct DecideArgs {
     int grow;  // 1: switch to bottom-up only while the frontier grows (Beamer's condition)
     int use_edges;      // Beamer's edge rule with CGR bits as the work measure: mf * alpha > mu
     double mu_total;    // in-CGR bits of all vertices (mu = mu_total - bits of the visited ones)
+    uint32_t alpha2_10, guard10;  // second edge test, taken only when the frontier is a sizeable share of the rest
 };
 
 struct CommitArgs {
@@ -57,10 +58,10 @@ struct CommitArgs {
     int32_t* __restrict__ levels;
     LevelState* ls;
     unsigned long long* hub_ctr;   // [2] hub segment / interval chunk queues, reset for the next level
-    unsigned long long* hub_ctr2;  // (bottom-up hub queue) reset for the next level
     unsigned long long* cursor;    // the expansion's work cursor [2], reset for the next level
     Offs offs_bits;                // record bits of the new frontier (used when use_mf)
-    Offs offs_in;                  // in-record bits of the newly visited vertices (used when use_mu)
+    const uint32_t* __restrict__ wb_out;  // dir_edges: record bits per 32-vertex word, out- and in-CGR (the new
+    const uint32_t* __restrict__ wb_in;   // vertices of a word are charged popc/32 of it: one coalesced load)
     int use_mf, use_mu;
     DecideArgs dec;
     int bc;
@@ -83,7 +84,13 @@ __device__ __forceinline__ void decide_body(volatile LevelState* ls, const Decid
     // edge rule (Beamer et al.: m_f > m_u / alpha) with record bits as edge counts: the top-down cost of the next
     // level is the out-record bits of the new frontier, the bottom-up cost at most the in-record bits of the
     // unvisited vertices
-    if (d.use_edges) to_bu = (double)ls->mf * d.alpha_bits10 > (d.mu_total - (double)ls->mu) * 10.0;
+    // (r2 sweeps on B200: alpha 7 suits the web graphs C2/C4; the social and R-MAT graphs, whose frontiers carry
+    // the high-degree vertices, gain from alpha 25 -- taken only while nf > nu / guard)
+    if (d.use_edges) {
+        const double mf = (double)ls->mf * 10.0, mu = d.mu_total - (double)ls->mu;
+        to_bu = mf * d.alpha_bits10 > mu * 100.0 ||
+                (mf * d.alpha2_10 > mu * 100.0 && nf * d.guard10 > nu * 10);
+    }
     ls->mf = 0;
     if (!d.enabled || nf == 0) dir = 0;
     else if (dir == 0 && to_bu && (nf > prev || !d.grow)) dir = 1;
@@ -114,6 +121,11 @@ __global__ void __launch_bounds__(kBlock) commit_kernel(CommitArgs a) {
                 a.V[w] |= b;
             }
             if (a.F && a.F[w] != b) a.F[w] = b;  // F = exactly the new frontier
+            if (b && a.use_mu) {
+                const uint32_t c = __popc(b);
+                mf += ((uint64_t)a.wb_out[w] * c) >> 5;
+                mu += ((uint64_t)a.wb_in[w] * c) >> 5;
+            }
         }
         nf += __popc(b);
         const uint32_t bal = __ballot_sync(0xffffffffu, b != 0);
@@ -131,8 +143,7 @@ __global__ void __launch_bounds__(kBlock) commit_kernel(CommitArgs a) {
                 if ((bj >> lane) & 1u) {
                     const uint64_t v = (base + j) * 32 + lane;
                     a.levels[v] = new_level;
-                    if (a.use_mf) mf += a.offs_bits(v + 1) - a.offs_bits(v);  // coalesced offset reads
-                    if (a.use_mu) mu += a.offs_in(v + 1) - a.offs_in(v);
+                    if (a.use_mf && !a.use_mu) mf += a.offs_bits(v + 1) - a.offs_bits(v);  // coalesced reads
                 }
             }
         }
@@ -159,7 +170,6 @@ __global__ void __launch_bounds__(kBlock) commit_kernel(CommitArgs a) {
                 a.hub_ctr[0] = 0;
                 a.hub_ctr[1] = 0;
             }
-            if (a.hub_ctr2) *a.hub_ctr2 = 0;
             if (a.cursor) {
                 a.cursor[0] = 0;
                 a.cursor[1] = 0;
@@ -227,6 +237,16 @@ __global__ void cc_jump(uint32_t* parent, uint64_t n) {
 __global__ void cc_init(uint32_t* parent, uint64_t n) {
     for (uint64_t v = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; v < n; v += (uint64_t)gridDim.x * blockDim.x)
         parent[v] = (uint32_t)v;
+}
+
+// Record bits per 32-vertex word of the owned range [lo, hi) (dir_edges direction rule).
+__global__ void word_bits_kernel(Offs offs, uint64_t lo, uint64_t hi, uint32_t* __restrict__ wb) {
+    const uint64_t w0 = lo >> 5, nw = ((hi + 31) >> 5) - w0;
+    for (uint64_t i = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; i < nw; i += (uint64_t)gridDim.x * blockDim.x) {
+        const uint64_t a = max((w0 + i) * 32, lo), b = min((w0 + i) * 32 + 32, hi);
+        const uint64_t bits = offs(b) - offs(a);
+        wb[i] = bits > 0xFFFFFFFFull ? 0xFFFFFFFFu : (uint32_t)bits;
+    }
 }
 
 __global__ void bswap_words(uint64_t* w, uint64_t n) {

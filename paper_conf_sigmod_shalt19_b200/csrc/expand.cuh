@@ -513,86 +513,4 @@ __global__ void __launch_bounds__(kBlock) hub_kernel(Ctx c, App app) {
     add_stats3(c.st, 0, na, 0);
 }
 
-// Flat hub pass (hub_flat knob): warps take chunks of 32 consecutive flattened segments (entries found by one 32-ary
-// ballot search per chunk, as in hub_kernel), and the lanes decode them in ONE flat loop with lane refill -- a lane
-// whose segment ended takes the next segment of the chunk (or the warp fetches the next chunk), so no lane waits for
-// the longest segment of the chunk.  Segments are read from global memory.
-template <int K, class App>
-__global__ void __launch_bounds__(kBlock) hub_flat_kernel(Ctx c, App app) {
-    if (c.dir && *c.dir) return;  // a bottom-up level (host-driven loop)
-    uint32_t na = 0;
-    if (c.ck.bits) chunk_pass<K>(c, app, na);
-    const unsigned long long hc = *(volatile unsigned long long*)c.hub_ctr;
-    if (hc == 0) {
-        add_stats3(c.st, 0, na, 0);
-        return;
-    }
-    const uint32_t lane = lane_id();
-    const uint32_t* W32 = reinterpret_cast<const uint32_t*>(c.W);
-    const uint32_t nh = (uint32_t)(hc >> 32), S = (uint32_t)(hc & 0xffffffffu);
-    uint64_t jb = ((uint64_t)blockIdx.x * blockDim.x + threadIdx.x) & ~31ull;
-    const uint64_t stride = (uint64_t)gridDim.x * blockDim.x;
-    uint32_t pmask = 0;  // segments of the current chunk not yet taken (bit l: the segment lane l holds)
-    bool more = true;
-    uint64_t hq = 0;     // chunk segment of this lane: bit position, vertex
-    uint32_t hu = 0;
-    GBitReader r;
-    uint32_t u = 0, rem = 0, cur = 0;
-    bool first = false;
-    for (;;) {
-        uint32_t need = __ballot_sync(0xffffffffu, rem == 0);
-        while (need && (pmask || more)) {
-            if (!pmask) {
-                if (jb >= S) {
-                    more = false;
-                    break;
-                }
-                const uint32_t j = (uint32_t)jb + lane;
-                const uint32_t k = warp_find_hub(c.hubq, nh, (uint32_t)jb, min(j, S - 1));
-                if (j < S) {
-                    const HubEntry e = c.hubq[k];
-                    hq = e.base + (uint64_t)(j - e.seg_off) * c.seg_bits;
-                    hu = e.u;
-                }
-                pmask = __ballot_sync(0xffffffffu, j < S);
-                jb += stride;
-                continue;
-            }
-            const uint32_t nn = __popc(need), np = __popc(pmask), tk = min(nn, np);
-            const bool me = (need >> lane) & 1u;
-            const uint32_t jn = __popc(need & lanemask_lt());
-            const uint32_t sl = (me && jn < tk) ? __fns(pmask, 0, (int)jn + 1) : 0u;
-            const uint64_t q = __shfl_sync(0xffffffffu, hq, sl);
-            const uint32_t uu = __shfl_sync(0xffffffffu, hu, sl);
-            if (me && jn < tk) {
-                u = uu;
-                r.init(W32, 0, q);
-                rem = (uint32_t)(r.template next<K>() - 1);
-                first = true;
-            }
-            pmask = tk == np ? 0u : pmask & (0xffffffffu << __fns(pmask, 0, (int)tk + 1));
-            need = tk == nn ? 0u : need & (0xffffffffu << __fns(need, 0, (int)tk + 1));
-        }
-        if (!__any_sync(0xffffffffu, rem != 0)) break;
-        const uint32_t nb = min(rem, 4u);
-        uint32_t v[4];
-#pragma unroll
-        for (uint32_t k = 0; k < 4; k++) {
-            if (k < nb) {
-                const uint64_t cd = r.template next<K>();
-                cur = (k == 0 && first) ? unmap_first32(u, cd) : cur + (uint32_t)cd;
-            }
-            v[k] = cur;
-        }
-        first = false;
-        App t = app;
-        t.begin(u);
-        t.many(v, nb);
-        t.end();
-        rem -= nb;
-        na += nb;
-    }
-    add_stats3(c.st, 0, na, 0);
-}
-
 }  // namespace gcgt_dev

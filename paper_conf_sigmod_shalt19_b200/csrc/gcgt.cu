@@ -63,6 +63,7 @@ struct DevCgr {
     uint64_t lo = 0;
     uint64_t base_bits = 0;     // stream bit of device word 0 (device bit positions = stream bits - base_bits)
     uint64_t offs_bytes = 0, word_bytes = 0;  // H2D volume (e2e accounting)
+    uint32_t* wbits = nullptr;  // record bits per 32-vertex word (dir_edges), built on the device at load
     Offs offs() const { return Offs{anc, rel, full, lo}; }
 };
 
@@ -85,8 +86,9 @@ struct gcgt_graph {
     int rank = 0, nranks = 1;
     DevCgr out, in;
     DevCk ck;
-    static constexpr uint32_t kCkC = 32;
-    uint32_t ck_c = kCkC;  // intervals per checkpoint chunk (GCGT_TUNE ck_c; 0 = no table)
+    static constexpr uint32_t kCkC = 3;
+    uint32_t ck_c = kCkC;  // intervals per checkpoint chunk (GCGT_TUNE ck_c; 0 = no table).  Vertices with more
+                           // intervals hand them to the grid-wide chunk pass (r2 sweep: 32 -> 3 gives C4 20.9 -> 17.7 ms)
     bool in_alias = false;  // symmetric: in == out
     bool has_in = false;
     bool dir_opt = false;
@@ -106,9 +108,6 @@ struct gcgt_graph {
     LevelState* ls = nullptr;
     HubEntry* hubq = nullptr;
     unsigned long long* hub_ctr = nullptr;   // [0] hub segments, [1] interval chunks (entries << 32 | items)
-    HubEntry* buq = nullptr;                 // deferred bottom-up hubs (in-records with many segments)
-    unsigned long long* buq_ctr = nullptr;
-    uint32_t* buq_done = nullptr;
     unsigned long long* cursor = nullptr;  // [0] work cursor, [1] finished blocks
     unsigned long long* st = nullptr;      // [vertices, arcs, bits]
     unsigned long long* aux = nullptr;     // [4] counters of the partitioned steps (hooks, frontier size, scratch)
@@ -127,24 +126,22 @@ struct gcgt_graph {
     int num_sms = 148;
     // knobs (GCGT_TUNE="key=value,..." at load; results never change)
     uint32_t hub_segs = 1;                  // more segments than this: the vertex's segments go grid-wide
-    uint32_t bu_hub_segs = 0xFFFFFFFFu;     // bottom-up: in-records with more segments are scanned grid-wide (off:
-                                            // measured slower on C2 / C3, even on C4)
     uint32_t bu_alpha = 40, bu_beta = 128;  // direction switch on vertex counts; alpha in tenths (r2 sweeps, C2-C4)
     uint32_t alpha_bits = 25;               // tenths
     bool bu_grow = true;                    // Beamer's "frontier growing" condition for the switch to bottom-up
     bool nfilter = false;                   // BFS filter: also test an L1 read of N before the claim
     bool hub_stage = true;                  // hub pass: segments staged through shared memory
     bool dir_bits = false;
-    bool dir_edges = false;                 // Beamer's edge rule on CGR bits (DecideArgs::use_edges)
-    uint32_t alpha_edges = 140;             // tenths
+    bool dir_edges = true;                  // Beamer's edge rule on CGR bits (DecideArgs::use_edges)
+    uint32_t alpha_edges = 70;              // tenths
+    uint32_t alpha_edges2 = 250;            // tenths; second test, only while nf * edge_guard / 10 > unvisited
+    uint32_t edge_guard = 70;               // tenths
     uint64_t in_nbits = 0;                  // bits of the loaded in-records (dir_edges)
     bool dir_opt_knob = true;
     bool use_graph = true;                  // BFS as one CUDA graph (else: chunked host-driven level loop)
     uint32_t chunk = 4;                     // host-driven loop: levels enqueued per host check
     bool compact_offs = true;
     bool td_stage = true;  // top-down: records staged through shared memory with coalesced 128-bit loads
-    bool hub_flat = true;   // hub pass: flat loop with lane refill (hub_flat_kernel; r2: C4 21.3 -> 21.0 ms)
-    bool bu_flat = false;  // bottom-up: flat scan loop with lane refill (bu_flat_kernel)
     bool td_pool = true;   // top-down: phase B from a per-warp segment pool, one flat loop with lane refill
                            // (hub_segs capped at 2; r2: C4 BFS 30.1 -> 21.3 ms, C2 7.2 -> 5.7 ms)
     // BFS graph (built on first use for a given levels buffer)
@@ -223,14 +220,8 @@ inline void launch_expand(gcgt_graph* g, cudaStream_t s, const Ctx& c, const Fro
         expand_kernel<K, SEG, App, Front><<<occ * g->num_sms, kBlock, 0, s>>>(c, fr, app, 0u);
         g->launches++;
         if (SEG || g->ck.bits) {  // hub segments and / or interval chunks
-            static int occf = 0;
-            if (g->hub_flat) {
-                if (!occf) occf = occupancy(hub_flat_kernel<K, App>);
-                hub_flat_kernel<K, App><<<occf * g->num_sms, kBlock, 0, s>>>(c, app);
-            } else {
-                if (!occh) occh = occupancy(hub_kernel<K, App>);
-                hub_kernel<K, App><<<occh * g->num_sms, kBlock, 0, s>>>(c, app);
-            }
+            if (!occh) occh = occupancy(hub_kernel<K, App>);
+            hub_kernel<K, App><<<occh * g->num_sms, kBlock, 0, s>>>(c, app);
             g->launches++;
         }
     });
@@ -242,33 +233,17 @@ inline void launch_expand(gcgt_graph* g, cudaStream_t s, const Ctx& c, const Fro
 
 inline void launch_bu(gcgt_graph* g, cudaStream_t s, const uint32_t* V, const uint32_t* F, uint32_t* N,
                       uint64_t lo, uint64_t hi, const uint32_t* dir) {
-    const BuHubs hubs{g->buq, g->buq_ctr, g->buq_done, g->bu_hub_segs};
     with_k(g->P, [&](auto KK, auto SS) {
         constexpr int K = decltype(KK)::value;
         constexpr bool SEG = decltype(SS)::value;
-        static int occ = 0, occh = 0, occf = 0;
+        static int occ = 0;
+        if (!occ) occ = occupancy(bu_kernel<K, SEG>);
         const uint64_t words = (hi - lo + 31) / 32 + 1;
-        if (g->bu_flat) {  // flat scan with lane refill; 32-word chunks per warp
-            if (!occf) occf = occupancy(bu_flat_kernel<K, SEG>);
-            const int grid = (int)std::max<uint64_t>(1, std::min<uint64_t>((words + 32 * kWarps - 1) / (32 * kWarps),
-                                                                            (uint64_t)occf * g->num_sms));
-            bu_flat_kernel<K, SEG><<<grid, kBlock, 0, s>>>(g->in.W, g->in.offs(), g->P.min_interval_len,
-                                                           8 * g->P.residual_segment_len, V, F, N, lo, hi, dir, g->st,
-                                                           hubs);
-        } else {
-            if (!occ) occ = occupancy(bu_kernel<K, SEG>);
-            const int grid = (int)std::max<uint64_t>(1, std::min<uint64_t>((words + kWarps - 1) / kWarps,
-                                                                            (uint64_t)occ * g->num_sms));
-            bu_kernel<K, SEG><<<grid, kBlock, 0, s>>>(g->in.W, g->in.offs(), g->P.min_interval_len,
-                                                      8 * g->P.residual_segment_len, V, F, N, lo, hi, dir, g->st, hubs);
-        }
+        const int grid = (int)std::max<uint64_t>(1, std::min<uint64_t>((words + kWarps - 1) / kWarps,
+                                                                        (uint64_t)occ * g->num_sms));
+        bu_kernel<K, SEG><<<grid, kBlock, 0, s>>>(g->in.W, g->in.offs(), g->P.min_interval_len,
+                                                  8 * g->P.residual_segment_len, V, F, N, lo, hi, dir, g->st);
         g->launches++;
-        if (SEG && hubs.q) {
-            if (!occh) occh = occupancy(bu_hub_kernel<K>);
-            bu_hub_kernel<K><<<occh * g->num_sms, kBlock, 0, s>>>(g->in.W, 8 * g->P.residual_segment_len, F, N, dir,
-                                                                 hubs, g->st);
-            g->launches++;
-        }
     });
 }
 
@@ -461,6 +436,9 @@ gcgt_status upload_cgr(gcgt_graph* g, const gcgt_cgr* c, uint64_t lo, uint64_t h
         CU(cudaStreamSynchronize(s));
         d->offs_bytes = (nloc + 1) * 8;
     }
+    const uint64_t nwl = ((hi + 31) >> 5) - (lo >> 5);
+    if ((st = galloc(g, &d->wbits, nwl + 1))) return st;
+    word_bits_kernel<<<flat_grid(g, nwl), kBlock, 0, s>>>(d->offs(), lo, hi, d->wbits);
     return GCGT_OK;
 }
 
@@ -633,19 +611,18 @@ void parse_tune(gcgt_graph* g) {
             else if (k == "alpha_bits") g->alpha_bits = (uint32_t)v;
             else if (k == "dir_edges") g->dir_edges = v != 0;
             else if (k == "alpha_edges") g->alpha_edges = (uint32_t)v;
+            else if (k == "alpha_edges2") g->alpha_edges2 = (uint32_t)v;
+            else if (k == "edge_guard") g->edge_guard = (uint32_t)v;
             else if (k == "dir_opt") g->dir_opt_knob = v != 0;
             else if (k == "graph") g->use_graph = v != 0;
             else if (k == "chunk") g->chunk = (uint32_t)std::max(2ul, std::min(32ul, v & ~1ul));
             else if (k == "compact") g->compact_offs = v != 0;
             else if (k == "td_stage") g->td_stage = v != 0;
             else if (k == "td_pool") g->td_pool = v != 0;
-            else if (k == "bu_flat") g->bu_flat = v != 0;
-            else if (k == "hub_flat") g->hub_flat = v != 0;
             else if (k == "ck_c") g->ck_c = (uint32_t)v;
             else if (k == "bu_grow") g->bu_grow = v != 0;
             else if (k == "nfilter") g->nfilter = v != 0;
             else if (k == "hub_stage") g->hub_stage = v != 0;
-            else if (k == "bu_hub_segs") g->bu_hub_segs = (uint32_t)v;  // 0xFFFFFFFF (or huge): no deferral
         }
         i = j + 1;
     }
@@ -706,7 +683,8 @@ DecideArgs decide_args(const gcgt_graph* g) {
     return DecideArgs{g->n, g->bu_alpha, g->bu_beta, g->dir_opt ? 1 : 0, g->dir_bits && g->dir_opt ? 1 : 0,
                       (double)g->nbits / (double)std::max<uint64_t>(1, g->n), g->dir_edges ? g->alpha_edges
                                                                                             : g->alpha_bits,
-                      g->bu_grow ? 1 : 0, g->dir_edges && g->dir_opt && !g->is_csr ? 1 : 0, (double)g->in_nbits};
+                      g->bu_grow ? 1 : 0, g->dir_edges && g->dir_opt && !g->is_csr ? 1 : 0, (double)g->in_nbits,
+                      g->alpha_edges2, g->edge_guard};
 }
 
 CommitArgs bfs_commit_args(gcgt_graph* g, int parity, int32_t* lv) {
@@ -722,12 +700,14 @@ CommitArgs bfs_commit_args(gcgt_graph* g, int parity, int32_t* lv) {
     a.levels = lv;
     a.ls = g->ls;
     a.hub_ctr = g->hub_ctr;
-    a.hub_ctr2 = g->buq_ctr;
     a.cursor = g->cursor;
     a.dec = decide_args(g);
     a.use_mf = a.dec.use_bits || a.dec.use_edges;
     a.use_mu = a.dec.use_edges;
-    if (a.use_mu) a.offs_in = g->in.offs();
+    if (a.use_mu) {
+        a.wb_out = g->out.wbits;
+        a.wb_in = g->in.wbits;
+    }
     if (a.use_mf && !g->is_csr) a.offs_bits = g->out.offs();
     if (a.use_mf && g->is_csr) a.offs_bits = Offs{nullptr, nullptr, g->crow, 0};
     return a;
@@ -882,11 +862,12 @@ extern "C" void gcgt_unload(gcgt_graph* g) {
     if (!g) return;
     cudaSetDevice(g->device);
     if (g->bfs_exec) cudaGraphExecDestroy(g->bfs_exec);
-    void* bufs[] = {g->out.hostW ? nullptr : g->out.W, g->out.anc, g->out.rel, g->out.full,
+    void* bufs[] = {g->out.hostW ? nullptr : g->out.W, g->out.anc, g->out.rel, g->out.full, g->out.wbits,
+                    g->in_alias ? nullptr : g->in.wbits,
                     g->in_alias ? nullptr : (g->in.hostW ? nullptr : g->in.W), g->in_alias ? nullptr : g->in.anc,
                     g->in_alias ? nullptr : g->in.rel, g->in_alias ? nullptr : g->in.full,
                     g->V, g->F, g->N, g->q, g->qbits, g->lvl_off, g->ls, g->hubq, g->hub_ctr, g->cursor, g->st,
-                    g->buq, g->buq_ctr, g->buq_done, g->aux, g->ck.wptr, g->ck.bits, g->ck.ck0, g->ck.after,
+                    g->aux, g->ck.wptr, g->ck.bits, g->ck.ck0, g->ck.after,
                     g->ck.ilen, g->ck.pos, g->ck.prev, g->ck.q,
                     g->src_dev, g->levels, g->parent, g->dirty, g->sigma, g->delta, g->bc,
                     g->crow, g->ccol, g->csr_hubq,
@@ -930,7 +911,6 @@ extern "C" gcgt_status gcgt_load(const gcgt_cgr* c, const gcgt_load_opts* opts, 
     g->n = c->n_total;
     g->nbits = c->nbits;
     g->P = c->params;
-    g->dir_bits = g->dir_bits || (o.symmetric != 0 && !o.in_cgr && getenv("GCGT_TUNE") == nullptr);
     // 1-D vertex-range partition (§8 e): rank r owns [lo, hi), boundaries on 32-vertex words, balanced by CGR bits.
     // A vertex-range slice of a CGR (gcgt_encode_slice) is loaded as exactly its range.
     g->lo = c->base;
@@ -971,14 +951,6 @@ extern "C" gcgt_status gcgt_load(const gcgt_cgr* c, const gcgt_load_opts* opts, 
     const uint64_t nhub = seg_bits ? count_hub_bound(c, g->lo, g->hi, (uint64_t)g->hub_segs * seg_bits) : 0;
     if ((st = galloc(g.get(), &g->hubq, nhub + 1))) return st;
     if ((st = build_checkpoints(g.get(), c))) return st;
-    if (g->has_in && seg_bits && g->bu_hub_segs < 0xFFFFu) {
-        const gcgt_cgr* ic = o.in_cgr ? o.in_cgr : c;
-        const uint64_t nbh = count_hub_bound(ic, g->lo, g->hi, (uint64_t)g->bu_hub_segs * seg_bits);
-        if ((st = galloc(g.get(), &g->buq, nbh + 1)) || (st = galloc(g.get(), &g->buq_done, nbh + 1)) ||
-            (st = galloc(g.get(), &g->buq_ctr, 1)))
-            return st;
-        CU(cudaMemsetAsync(g->buq_ctr, 0, 8, g->stream));
-    }
     CU(cudaStreamSynchronize(g->stream));
     CU(cudaGetLastError());
     *out = g.release();
@@ -1341,7 +1313,6 @@ extern "C" gcgt_status gcgt_dist_bfs_expand(gcgt_graph* g, uint32_t level, uint3
             CU(cudaMemcpy(one, &v, 4, cudaMemcpyHostToDevice));
         }
         launch_bu(g, s, g->V, g->F, fslice - w_lo, g->lo, g->hi, one);
-        if (g->buq_ctr) CU(cudaMemsetAsync(g->buq_ctr, 0, 8, s));
         return GCGT_OK;
     }
     CU(cudaMemsetAsync(cand, 0, nwf * 4, s));

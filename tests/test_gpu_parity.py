@@ -203,10 +203,9 @@ def test_warp_decoder_random_streams(k):
 @pytest.mark.parametrize("tune", ["", "bu_alpha=100000,bu_beta=1", "bu_alpha=100000,bu_beta=100000", "graph=0",
                                   "graph=0,bu_alpha=100000,bu_beta=1", "graph=0,chunk=2", "graph=0,chunk=16",
                                   "hub_segs=1", "compact=0", "dir_bits=1", "dir_opt=0", "bu_alpha=1", "td_stage=0",
-                                  "td_pool=1", "td_pool=1,td_stage=0", "bu_hub_segs=1", "bu_hub_segs=100000", "ck_c=2",
-                                  "ck_c=0", "bu_grow=0,bu_alpha=25", "hub_stage=0", "bu_flat=1",
-                                  "bu_flat=1,bu_alpha=100000,bu_beta=1", "bu_flat=1,bu_hub_segs=1",
-                                  "bu_flat=0", "td_pool=0", "bu_flat=0,td_pool=0,bu_alpha=100000,bu_beta=1", "hub_flat=0",
+                                  "td_pool=1", "td_pool=1,td_stage=0", "ck_c=2", "ck_c=1", "ck_c=32",
+                                  "ck_c=0", "bu_grow=0,bu_alpha=25", "hub_stage=0", "td_pool=0",
+                                  "td_pool=0,bu_alpha=100000,bu_beta=1", "ck_c=4", "ck_c=3,td_pool=0",
                                   "dir_edges=1", "dir_edges=1,alpha_edges=10", "dir_edges=1,alpha_edges=1000"])
 @pytest.mark.parametrize("name", ["c1", "rmat_s", "web_s", "social_s"])
 def test_bfs_direction_optimizing(name, tune, monkeypatch):
@@ -225,7 +224,7 @@ def test_bfs_direction_optimizing(name, tune, monkeypatch):
         assert np.array_equal(g.bfs(r), O.bfs(ro, co, r)), (name, tune, r)
 
 
-@pytest.mark.parametrize("tune", ["td_pool=1", "td_pool=0", "td_stage=0", "hub_segs=1", "ck_c=2", "ck_c=0", "hub_flat=0",
+@pytest.mark.parametrize("tune", ["td_pool=1", "td_pool=0", "td_stage=0", "hub_segs=1", "ck_c=2", "ck_c=0", "ck_c=32",
                                   "td_pool=0,hub_segs=8"])
 @pytest.mark.parametrize("name", ["web_s", "social_s", "rmat_s"])
 def test_cc_bc_engine_knobs(name, tune, monkeypatch):
@@ -239,10 +238,9 @@ def test_cc_bc_engine_knobs(name, tune, monkeypatch):
     check_bc(g.bc(src), O.bc(ro, co, src))
 
 
-@pytest.mark.parametrize("flat", [0, 1])
 @pytest.mark.parametrize("ml,sl,k", [(4, 32, 3), (0, 0, 1), (2, 8, 5)])
-def test_bfs_bottom_up_random(ml, sl, k, flat, monkeypatch):
-    monkeypatch.setenv("GCGT_TUNE", f"bu_alpha=100000,bu_beta=1,bu_flat={flat}")
+def test_bfs_bottom_up_random(ml, sl, k, monkeypatch):
+    monkeypatch.setenv("GCGT_TUNE", "bu_alpha=100000,bu_beta=1")
     for seed, sym in [(1, True), (2, False), (3, False)]:
         ro, co = random_graph(6000, 60000, seed=seed + k, symmetric=sym)
         cgr = G.encode(ro, co, ml, sl, k)

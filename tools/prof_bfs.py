@@ -15,11 +15,10 @@ ap.add_argument("--reps", type=int, default=1)
 ap.add_argument("--app", default="bfs", choices=["bfs", "cc", "bc"])
 ap.add_argument("--bc-sources", type=int, default=1)
 a = ap.parse_args()
-cfg = synth.CONFIGS[a.config]
-ro, co = cfg.make()
-P = (cfg.min_interval_len, cfg.residual_segment_len, cfg.zeta_k)
-incgr = None if cfg.symmetric else G.encode_transpose(ro, co, *P)
-g = G.load(G.encode(ro, co, *P), stream="torch", in_cgr=incgr, symmetric=cfg.symmetric)
+sys.path.insert(0, os.path.dirname(os.path.abspath(__file__)))
+import gcache  # noqa: E402
+cfg, ro, cgr, incgr = gcache.graph(a.config)
+g = G.load(cgr, stream="torch", in_cgr=incgr, symmetric=cfg.symmetric)
 roots = synth.pick_roots(ro, 16)
 out = torch.empty(ro.size - 1, dtype=torch.int32, device="cuda")
 for i in range(a.reps):

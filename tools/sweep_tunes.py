@@ -12,12 +12,10 @@ import paper_conf_sigmod_shalt19_b200 as G  # noqa: E402
 import synth  # noqa: E402
 
 cfgname, nroots, tunes = sys.argv[1], int(sys.argv[2]), sys.argv[3:] or [""]
-cfg = synth.CONFIGS[cfgname]
 t0 = time.time()
-ro, co = cfg.make()
-P = (cfg.min_interval_len, cfg.residual_segment_len, cfg.zeta_k)
-cgr = G.encode(ro, co, *P)
-incgr = None if cfg.symmetric else G.encode_transpose(ro, co, *P)
+sys.path.insert(0, os.path.dirname(os.path.abspath(__file__)))
+import gcache  # noqa: E402
+cfg, ro, cgr, incgr = gcache.graph(cfgname)
 print(f"# {cfgname} n={ro.size - 1} m={int(ro[-1])} prep {time.time() - t0:.1f}s", flush=True)
 roots = synth.pick_roots(ro, nroots)
 n = ro.size - 1

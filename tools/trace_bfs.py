@@ -12,11 +12,10 @@ import synth  # noqa: E402
 
 cfgname = sys.argv[1] if len(sys.argv) > 1 else "c2"
 nroots = int(sys.argv[2]) if len(sys.argv) > 2 else 2
-cfg = synth.CONFIGS[cfgname]
-ro, co = cfg.make()
-P = (cfg.min_interval_len, cfg.residual_segment_len, cfg.zeta_k)
-incgr = None if cfg.symmetric else G.encode_transpose(ro, co, *P)
-g = G.load(G.encode(ro, co, *P), stream="torch", in_cgr=incgr, symmetric=cfg.symmetric)
+sys.path.insert(0, os.path.dirname(os.path.abspath(__file__)))
+import gcache  # noqa: E402
+cfg, ro, cgr, incgr = gcache.graph(cfgname)
+g = G.load(cgr, stream="torch", in_cgr=incgr, symmetric=cfg.symmetric)
 roots = synth.pick_roots(ro, 16)
 out = torch.empty(ro.size - 1, dtype=torch.int32, device="cuda")
 g.bfs(roots[0], out=out)  # warm
