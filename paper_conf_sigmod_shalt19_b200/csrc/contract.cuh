@@ -42,7 +42,7 @@ struct DecideArgs {
     int grow;  // 1: switch to bottom-up only while the frontier grows (Beamer's condition)
     int use_edges;      // Beamer's edge rule with CGR bits as the work measure: mf * alpha > mu
     double mu_total;    // in-CGR bits of all vertices (mu = mu_total - bits of the visited ones)
-    uint32_t alpha2_10, guard10;  // second edge test, taken only when the frontier is a sizeable share of the rest
+    uint32_t alpha2_10, guard10;  // second edge test, taken only when the frontier grew by more than guard10 / 10
 };
 
 struct CommitArgs {
@@ -84,12 +84,14 @@ __device__ __forceinline__ void decide_body(volatile LevelState* ls, const Decid
     // edge rule (Beamer et al.: m_f > m_u / alpha) with record bits as edge counts: the top-down cost of the next
     // level is the out-record bits of the new frontier, the bottom-up cost at most the in-record bits of the
     // unvisited vertices
-    // (r2 sweeps on B200: alpha 7 suits the web graphs C2/C4; the social and R-MAT graphs, whose frontiers carry
-    // the high-degree vertices, gain from alpha 25 -- taken only while nf > nu / guard)
-    if (d.use_edges) {
+    // (r2 sweeps on B200: the vertex-count test suits the web graphs C2/C4; the social and R-MAT graphs gain from
+    // the edge test with alpha 25, taken only on explosive frontier growth (nf > guard * previous frontier): there the
+    // frontier holds the high-degree vertices -- an expensive top-down level -- and the next level reaches most of
+    // the rest, so bottom-up scans stop early; the web graphs' frontiers grow ~1.5x per level at that point)
+    if (d.use_edges) {  // in addition to the vertex-count test
         const double mf = (double)ls->mf * 10.0, mu = d.mu_total - (double)ls->mu;
-        to_bu = mf * d.alpha_bits10 > mu * 100.0 ||
-                (mf * d.alpha2_10 > mu * 100.0 && nf * d.guard10 > nu * 10);
+        to_bu = to_bu || mf * d.alpha_bits10 > mu * 100.0 ||
+                (mf * d.alpha2_10 > mu * 100.0 && nf * 10 > prev * d.guard10);
     }
     ls->mf = 0;
     if (!d.enabled || nf == 0) dir = 0;

@@ -133,9 +133,9 @@ struct gcgt_graph {
     bool hub_stage = true;                  // hub pass: segments staged through shared memory
     bool dir_bits = false;
     bool dir_edges = true;                  // Beamer's edge rule on CGR bits (DecideArgs::use_edges)
-    uint32_t alpha_edges = 70;              // tenths
-    uint32_t alpha_edges2 = 250;            // tenths; second test, only while nf * edge_guard / 10 > unvisited
-    uint32_t edge_guard = 70;               // tenths
+    uint32_t alpha_edges = 0;               // tenths (0: only the guarded second test)
+    uint32_t alpha_edges2 = 250;            // tenths; second test, only when nf > edge_guard / 10 * previous nf
+    uint32_t edge_guard = 40;               // tenths
     uint64_t in_nbits = 0;                  // bits of the loaded in-records (dir_edges)
     bool dir_opt_knob = true;
     bool use_graph = true;                  // BFS as one CUDA graph (else: chunked host-driven level loop)

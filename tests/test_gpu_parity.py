@@ -205,7 +205,8 @@ def test_warp_decoder_random_streams(k):
                                   "hub_segs=1", "compact=0", "dir_bits=1", "dir_opt=0", "bu_alpha=1", "td_stage=0",
                                   "td_pool=1", "td_pool=1,td_stage=0", "ck_c=2", "ck_c=1", "ck_c=32",
                                   "ck_c=0", "bu_grow=0,bu_alpha=25", "hub_stage=0", "td_pool=0",
-                                  "td_pool=0,bu_alpha=100000,bu_beta=1", "ck_c=4", "ck_c=3,td_pool=0",
+                                  "td_pool=0,bu_alpha=100000,bu_beta=1", "ck_c=4", "ck_c=3,td_pool=0", "dir_edges=0",
+                                  "edge_guard=10,alpha_edges2=1000", "alpha_edges=140",
                                   "dir_edges=1", "dir_edges=1,alpha_edges=10", "dir_edges=1,alpha_edges=1000"])
 @pytest.mark.parametrize("name", ["c1", "rmat_s", "web_s", "social_s"])
 def test_bfs_direction_optimizing(name, tune, monkeypatch):
