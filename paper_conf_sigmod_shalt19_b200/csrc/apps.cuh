@@ -98,7 +98,8 @@ struct BcFwdApp {
 // A vertex's arcs are split over tasks (interval area + segments), so each task adds its partial sum to delta(u)
 // and bc(u) (u != source); delta is zeroed per source.  Zero partials are skipped, so exact zeros stay exact.
 struct BcBwdApp {
-    const int32_t* __restrict__ levels;
+    const uint32_t* __restrict__ LB;  // bitmap of level d+1 (n/8 bytes, L2-resident): the successor test of every arc
+                                      // without touching the 4n-byte levels array
     const double* __restrict__ sigma;
     double* __restrict__ delta;
     double* __restrict__ bc;
@@ -112,12 +113,22 @@ struct BcBwdApp {
         acc = 0.0;
     }
     __device__ __forceinline__ void vertex(uint32_t) {}
+    __device__ __forceinline__ void add(uint32_t w) { acc += sv / sigma[w] * (1.0 + delta[w]); }
     __device__ __forceinline__ void one(uint32_t w) {
-        if (__ldg(levels + w) == next) acc += sv / sigma[w] * (1.0 + delta[w]);
+        if ((__ldg(LB + (w >> 5)) >> (w & 31)) & 1u) add(w);
     }
-    GCGT_MANY_BY_ONE
+    __device__ __forceinline__ void many(const uint32_t (&v)[4], uint32_t n) {
+        uint32_t m[4];
+#pragma unroll
+        for (uint32_t k = 0; k < 4; k++) m[k] = k < n ? __ldg(LB + (v[k] >> 5)) : 0u;
+#pragma unroll
+        for (uint32_t k = 0; k < 4; k++)
+            if ((m[k] >> (v[k] & 31)) & 1u) add(v[k]);
+    }
     __device__ __forceinline__ void range(uint32_t s, uint32_t len) {
-        for (uint32_t t = 0; t < len; t++) one(s + t);
+        for_words(s, len, [&](uint32_t w, uint32_t mask) {
+            for (uint32_t b = __ldg(LB + w) & mask; b; b &= b - 1) add(w * 32 + (__ffs(b) - 1));
+        });
     }
     __device__ __forceinline__ void end() {
         // lanes finishing tasks of the same vertex (a hub's segments sit side by side in the hub queue) first sum

@@ -241,6 +241,13 @@ __global__ void cc_init(uint32_t* parent, uint64_t n) {
         parent[v] = (uint32_t)v;
 }
 
+// BC backward: writes (set) or clears the bitmap words of one level from its queue range (words + frontier bits).
+__global__ void bc_level_bits(const uint32_t* __restrict__ q, const uint32_t* __restrict__ qbits, uint32_t len,
+                              uint32_t* __restrict__ LB, int set) {
+    for (uint32_t i = blockIdx.x * blockDim.x + threadIdx.x; i < len; i += gridDim.x * blockDim.x)
+        LB[q[i]] = set ? qbits[i] : 0u;
+}
+
 // Record bits per 32-vertex word of the owned range [lo, hi) (dir_edges direction rule).
 __global__ void word_bits_kernel(Offs offs, uint64_t lo, uint64_t hi, uint32_t* __restrict__ wb) {
     const uint64_t w0 = lo >> 5, nw = ((hi + 31) >> 5) - w0;

@@ -1256,11 +1256,14 @@ extern "C" gcgt_status gcgt_bc(gcgt_graph* g, const uint32_t* sources, uint32_t 
         CU(cudaStreamSynchronize(s));
         for (int d = (int)D - 2; d >= 0; d--) {  // the last level has no successors
             const uint32_t off = lvl_off[d];
-            *g->h_misc() = lvl_off[d + 1] - off;
+            const uint32_t off1 = lvl_off[d + 1], len1 = lvl_off[d + 2] - off1;  // level d+1's queue range
+            bc_level_bits<<<flat_grid(g, len1), kBlock, 0, s>>>(g->q + off1, g->qbits + off1, len1, g->N, 1);
             const QueueFront fr{g->q + off, nullptr, nullptr, g->qbits + off, nullptr, lvl_off[d + 1] - off};
-            const BcBwdApp app{g->levels, g->sigma, g->delta, g->bc, d + 1, sources[si], 0, 0.0, 0.0};
+            const BcBwdApp app{g->N, g->sigma, g->delta, g->bc, d + 1, sources[si], 0, 0.0, 0.0};
             launch_expand(g, s, c, fr, app);
             CU(cudaMemsetAsync(g->hub_ctr, 0, 16, s));
+            bc_level_bits<<<flat_grid(g, len1), kBlock, 0, s>>>(g->q + off1, g->qbits + off1, len1, g->N, 0);
+            g->launches += 2;
         }
     }
     if ((st = copy_out(g, bc, g->bc, g->n * 8, placement))) return st;
