@@ -248,6 +248,19 @@ __global__ void bc_level_bits(const uint32_t* __restrict__ q, const uint32_t* __
         LB[q[i]] = set ? qbits[i] : 0u;
 }
 
+// BC backward: X(v) = (1 + delta(v)) / sigma(v) for the vertices of one level (its queue range), once their delta
+// is final.
+__global__ void bc_level_x(const uint32_t* __restrict__ q, const uint32_t* __restrict__ qbits, uint32_t len,
+                           const double* __restrict__ sigma, const double* __restrict__ delta, double* __restrict__ X) {
+    for (uint32_t i = blockIdx.x * blockDim.x + threadIdx.x; i < len * 32; i += gridDim.x * blockDim.x) {
+        const uint32_t e = i >> 5, b = i & 31;
+        if ((qbits[e] >> b) & 1u) {
+            const uint64_t v = (uint64_t)q[e] * 32 + b;
+            X[v] = (1.0 + delta[v]) / sigma[v];
+        }
+    }
+}
+
 // Record bits per 32-vertex word of the owned range [lo, hi) (dir_edges direction rule).
 __global__ void word_bits_kernel(Offs offs, uint64_t lo, uint64_t hi, uint32_t* __restrict__ wb) {
     const uint64_t w0 = lo >> 5, nw = ((hi + 31) >> 5) - w0;

@@ -115,7 +115,7 @@ struct gcgt_graph {
     int32_t* levels = nullptr;
     uint32_t* parent = nullptr;
     uint32_t* dirty = nullptr;             // dist CC: changed-parent bitmap
-    double *sigma = nullptr, *delta = nullptr, *bc = nullptr;
+    double *sigma = nullptr, *delta = nullptr, *bc = nullptr, *bcx = nullptr;
     // pinned host mirror (one small block): level state, counters, source
     uint8_t* hp = nullptr;
     LevelState* h_ls() const { return reinterpret_cast<LevelState*>(hp); }
@@ -126,9 +126,10 @@ struct gcgt_graph {
     int num_sms = 148;
     // knobs (GCGT_TUNE="key=value,..." at load; results never change)
     uint32_t hub_segs = 1;                  // more segments than this: the vertex's segments go grid-wide
-    uint32_t bu_alpha = 40, bu_beta = 128;  // direction switch on vertex counts; alpha in tenths (r2 sweeps, C2-C4)
+    uint32_t bu_alpha = 30, bu_beta = 128;  // direction switch on vertex counts; alpha in tenths (r2 sweeps, C2-C4)
     uint32_t alpha_bits = 25;               // tenths
-    bool bu_grow = true;                    // Beamer's "frontier growing" condition for the switch to bottom-up
+    bool bu_grow = false;                   // Beamer's "frontier growing" condition for the switch to bottom-up
+                                            // (r2 sweep, alpha 3 without it: C2 4.28, C3 6.55, C4 17.60 ms)
     bool nfilter = false;                   // BFS filter: also test an L1 read of N before the claim
     bool hub_stage = true;                  // hub pass: segments staged through shared memory
     bool dir_bits = false;
@@ -869,7 +870,7 @@ extern "C" void gcgt_unload(gcgt_graph* g) {
                     g->V, g->F, g->N, g->q, g->qbits, g->lvl_off, g->ls, g->hubq, g->hub_ctr, g->cursor, g->st,
                     g->aux, g->ck.wptr, g->ck.bits, g->ck.ck0, g->ck.after,
                     g->ck.ilen, g->ck.pos, g->ck.prev, g->ck.q,
-                    g->src_dev, g->levels, g->parent, g->dirty, g->sigma, g->delta, g->bc,
+                    g->src_dev, g->levels, g->parent, g->dirty, g->sigma, g->delta, g->bc, g->bcx,
                     g->crow, g->ccol, g->csr_hubq,
                     g->csr_in_owned ? g->crow_in : nullptr, g->csr_in_owned ? g->ccol_in : nullptr};
     if (g->stream) {
@@ -1194,6 +1195,7 @@ extern "C" gcgt_status gcgt_bc(gcgt_graph* g, const uint32_t* sources, uint32_t 
     gcgt_status st;
     if (!g->sigma) {
         if ((st = galloc(g, &g->sigma, g->n)) || (st = galloc(g, &g->delta, g->n)) || (st = galloc(g, &g->bc, g->n)) ||
+            (st = galloc(g, &g->bcx, g->n)) ||
             (st = galloc(g, &g->qbits, g->n + g->nw)) || (st = galloc(g, &g->lvl_off, g->n + 3 + 2 * gcgt_graph::kKev)))
             return st;
         uint32_t* bigq = nullptr;
@@ -1258,12 +1260,14 @@ extern "C" gcgt_status gcgt_bc(gcgt_graph* g, const uint32_t* sources, uint32_t 
             const uint32_t off = lvl_off[d];
             const uint32_t off1 = lvl_off[d + 1], len1 = lvl_off[d + 2] - off1;  // level d+1's queue range
             bc_level_bits<<<flat_grid(g, len1), kBlock, 0, s>>>(g->q + off1, g->qbits + off1, len1, g->N, 1);
+            bc_level_x<<<flat_grid(g, (uint64_t)len1 * 32), kBlock, 0, s>>>(g->q + off1, g->qbits + off1, len1,
+                                                                            g->sigma, g->delta, g->bcx);
             const QueueFront fr{g->q + off, nullptr, nullptr, g->qbits + off, nullptr, lvl_off[d + 1] - off};
-            const BcBwdApp app{g->N, g->sigma, g->delta, g->bc, d + 1, sources[si], 0, 0.0, 0.0};
+            const BcBwdApp app{g->N, g->bcx, g->sigma, g->delta, g->bc, sources[si], 0, 0.0};
             launch_expand(g, s, c, fr, app);
             CU(cudaMemsetAsync(g->hub_ctr, 0, 16, s));
             bc_level_bits<<<flat_grid(g, len1), kBlock, 0, s>>>(g->q + off1, g->qbits + off1, len1, g->N, 0);
-            g->launches += 2;
+            g->launches += 3;
         }
     }
     if ((st = copy_out(g, bc, g->bc, g->n * 8, placement))) return st;
