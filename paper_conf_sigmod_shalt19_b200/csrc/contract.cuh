@@ -95,7 +95,9 @@ __device__ __forceinline__ void decide_body(volatile LevelState* ls, const Decid
     }
     ls->mf = 0;
     if (!d.enabled || nf == 0) dir = 0;
-    else if (dir == 0 && to_bu && (nf > prev || !d.grow)) dir = 1;
+    // (never into bottom-up with a frontier below the bottom-up -> top-down threshold: a whole-graph scan for the
+    // last few vertices)
+    else if (dir == 0 && to_bu && (nf > prev || !d.grow) && nf * d.beta >= d.n) dir = 1;
     else if (dir == 1 && nf * d.beta < d.n && nf < prev) dir = 0;
     ls->dir = dir;
     ls->prev_nf = (uint32_t)nf;
