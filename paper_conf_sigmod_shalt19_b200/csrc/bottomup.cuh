@@ -93,8 +93,8 @@ __device__ __forceinline__ bool bu_scan(GBitReader& r, uint64_t p0, uint64_t p1,
     return found;
 }
 
-template <int K, bool SEG, int MINB = 6>
-__global__ void __launch_bounds__(kBlock, MINB) bu_kernel(const uint64_t* __restrict__ W, Offs offs, uint32_t min_len,
+template <int K, bool SEG>
+__global__ void __launch_bounds__(kBlock, 6) bu_kernel(const uint64_t* __restrict__ W, Offs offs, uint32_t min_len,
                                                        uint32_t seg_bits, const uint32_t* __restrict__ V,
                                                        const uint32_t* __restrict__ F, uint32_t* __restrict__ N,
                                                        uint64_t lo, uint64_t hi, const uint32_t* __restrict__ dir,

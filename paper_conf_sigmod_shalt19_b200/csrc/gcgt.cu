@@ -133,7 +133,6 @@ struct gcgt_graph {
     bool nfilter = false;                   // BFS filter: also test an L1 read of N before the claim
     bool hub_stage = true;                  // hub pass: segments staged through shared memory
     bool dir_bits = false;
-    bool bu_minb8 = false;                  // bottom-up kernel at 8 blocks per SM (32 registers)
     bool dir_edges = true;                  // Beamer's edge rule on CGR bits (DecideArgs::use_edges)
     uint32_t alpha_edges = 0;               // tenths (0: only the guarded second test)
     uint32_t alpha_edges2 = 250;            // tenths; second test, only when nf > edge_guard / 10 * previous nf
@@ -238,21 +237,13 @@ inline void launch_bu(gcgt_graph* g, cudaStream_t s, const uint32_t* V, const ui
     with_k(g->P, [&](auto KK, auto SS) {
         constexpr int K = decltype(KK)::value;
         constexpr bool SEG = decltype(SS)::value;
-        static int occ = 0, occ8 = 0;
+        static int occ = 0;
+        if (!occ) occ = occupancy(bu_kernel<K, SEG>);
         const uint64_t words = (hi - lo + 31) / 32 + 1;
-        if (g->bu_minb8) {  // 8 blocks (64 warps) per SM at 32 registers
-            if (!occ8) occ8 = occupancy(bu_kernel<K, SEG, 8>);
-            const int grid = (int)std::max<uint64_t>(1, std::min<uint64_t>((words + kWarps - 1) / kWarps,
-                                                                            (uint64_t)occ8 * g->num_sms));
-            bu_kernel<K, SEG, 8><<<grid, kBlock, 0, s>>>(g->in.W, g->in.offs(), g->P.min_interval_len,
-                                                         8 * g->P.residual_segment_len, V, F, N, lo, hi, dir, g->st);
-        } else {
-            if (!occ) occ = occupancy(bu_kernel<K, SEG>);
-            const int grid = (int)std::max<uint64_t>(1, std::min<uint64_t>((words + kWarps - 1) / kWarps,
-                                                                            (uint64_t)occ * g->num_sms));
-            bu_kernel<K, SEG><<<grid, kBlock, 0, s>>>(g->in.W, g->in.offs(), g->P.min_interval_len,
-                                                      8 * g->P.residual_segment_len, V, F, N, lo, hi, dir, g->st);
-        }
+        const int grid = (int)std::max<uint64_t>(1, std::min<uint64_t>((words + kWarps - 1) / kWarps,
+                                                                        (uint64_t)occ * g->num_sms));
+        bu_kernel<K, SEG><<<grid, kBlock, 0, s>>>(g->in.W, g->in.offs(), g->P.min_interval_len,
+                                                  8 * g->P.residual_segment_len, V, F, N, lo, hi, dir, g->st);
         g->launches++;
     });
 }
@@ -621,7 +612,6 @@ void parse_tune(gcgt_graph* g) {
             else if (k == "alpha_bits") g->alpha_bits = (uint32_t)v;
             else if (k == "dir_edges") g->dir_edges = v != 0;
             else if (k == "alpha_edges") g->alpha_edges = (uint32_t)v;
-            else if (k == "bu_minb8") g->bu_minb8 = v != 0;
             else if (k == "alpha_edges2") g->alpha_edges2 = (uint32_t)v;
             else if (k == "edge_guard") g->edge_guard = (uint32_t)v;
             else if (k == "dir_opt") g->dir_opt_knob = v != 0;
