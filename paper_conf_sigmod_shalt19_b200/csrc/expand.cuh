@@ -11,10 +11,13 @@
 //  2. Phase A (lane per vertex): the record header and the interval area (Alg. 2 l.1-32, :650-688), decoded from
 //     shared memory; each interval is claimed as a word range (the Two-Phase "expand a long run in parallel" idea at
 //     word granularity: 32 ids per operation).  Then segNum (Fig. 6, :1057-1069).
-//  3. Phase B (lane per residual segment): the round's segments — self-contained by R17 ("breaks the sequential
-//     dependencies", :945-946) — are flattened over the lanes and decoded from shared memory, four neighbour ids per
-//     batch of filter probes.  A vertex with more than hub_segs segments hands them to the level's hub queue instead;
-//     the hub pass spreads them over the whole grid (Task Stealing + Residual Segmentation, §4.3/§5.2, at grid scale).
+//  3. Phase B: the round's residual segments — self-contained by R17 ("breaks the sequential dependencies",
+//     :945-946) — become tasks of a per-warp pool (default, `pool`): once it holds >= kPoolFlush tasks it is drained by
+//     ONE flat loop with lane refill (drain_pool), four neighbour ids per step and lane, so no lane waits for the
+//     longest segment of a round.  (pool = 0: the round's segments one per lane from shared memory.)  A vertex with
+//     more than hub_segs segments (default 1) hands them to the level's hub queue instead, and a vertex with more than
+//     ck_c intervals (default 3) its interval chunks to the chunk queue; the hub pass spreads both over the whole grid
+//     (Task Stealing + Residual Segmentation, §4.3/§5.2, at grid scale).
 #pragma once
 #include "apps.cuh"
 

@@ -2,8 +2,9 @@
 // partitioned (multi-GPU) steps, and the C ABI around them (include/gcgt.h).
 //
 // Pipeline per level (expansion - filtering - contraction, §6, Fig. 7(a)):
-//   top-down   expand_kernel (records staged through shared memory, lane per vertex / per residual segment) and
-//              hub_kernel (segments of high-degree vertices over the whole grid)            — expand.cuh
+//   top-down   expand_kernel (records staged through shared memory, lane per vertex for the header and intervals,
+//              residual segments through a per-warp pool drained by a flat lane-refill loop) and hub_kernel
+//              (long interval areas and multi-segment vertices over the whole grid)        — expand.cuh
 //   bottom-up  bu_kernel (in-records scanned until the first frontier parent)                — bottomup.cuh
 //   contract   commit_kernel (N -> V / F / levels / next queue; direction; level counter)   — contract.cuh
 // The level state lives on the device, so BFS runs as one CUDA graph: a while-node whose body holds two levels,
