@@ -225,9 +225,15 @@ __global__ void seed_kernel(const uint32_t* __restrict__ src_p, uint32_t* V, uin
 
 // levels of the vertices the search never reached: -1 (every visited vertex's level was written exactly once, by the
 // seed or by the contraction that discovered it, so the levels array needs no initialising pass).
+// One thread per 32-vertex word: after a full traversal nearly every word is all-visited, so the pass reads n/8
+// bytes and writes almost nothing.
 __global__ void finalize_levels(const uint32_t* __restrict__ V, int32_t* __restrict__ levels, uint64_t n) {
-    for (uint64_t v = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; v < n; v += (uint64_t)gridDim.x * blockDim.x)
-        if (!((__ldg(V + (v >> 5)) >> (v & 31)) & 1u)) levels[v] = -1;
+    const uint64_t nw = (n + 31) / 32;
+    for (uint64_t w = (uint64_t)blockIdx.x * blockDim.x + threadIdx.x; w < nw; w += (uint64_t)gridDim.x * blockDim.x) {
+        uint32_t unv = ~__ldg(V + w);
+        if (n - w * 32 < 32) unv &= (1u << (n - w * 32)) - 1;
+        for (; unv; unv &= unv - 1) levels[w * 32 + (__ffs(unv) - 1)] = -1;
+    }
 }
 
 __global__ void cc_jump(uint32_t* parent, uint64_t n) {

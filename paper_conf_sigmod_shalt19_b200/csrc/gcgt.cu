@@ -1137,7 +1137,7 @@ extern "C" gcgt_status gcgt_bfs(gcgt_graph* g, uint32_t source, int32_t* levels,
             if (g->h_ls()->qlen[level & 1] == 0) break;
         }
     }
-    finalize_levels<<<flat_grid(g, g->n), kBlock, 0, s>>>(g->V, lv, g->n);
+    finalize_levels<<<flat_grid(g, (g->n + 31) / 32), kBlock, 0, s>>>(g->V, lv, g->n);
     g->launches++;
     if ((st = copy_out(g, levels, lv, g->n * 4, placement))) return st;
     if ((st = end_call(g, stats, 0))) return st;
